@@ -1,0 +1,403 @@
+"""Pins for the oracle (oracle/culi_oracle.cpp) against things other than itself:
+the paper's worked examples, closed forms, brute force on tiny inputs with Python's own integers,
+floats and lists, and invariants.  None of these retype the oracle's code: every expected value here
+is computed by Python semantics (big integers reduced mod 2**64, IEEE floats, lists) or printed in the
+paper / SURVEY §8(c).12b.
+"""
+from __future__ import annotations
+
+import itertools
+import math
+import os
+import random
+
+import pytest
+
+from paper_conf_cluster_subdbn18_b200 import workloads as W
+
+GOLDEN = os.path.join(os.path.dirname(__file__), "golden")
+
+
+def load_tsv(name):
+    rows = []
+    with open(os.path.join(GOLDEN, name)) as f:
+        for line in f:
+            if not line.strip() or line.startswith("#"):
+                continue
+            parts = line.rstrip("\n").split("\t")
+            rows.append(parts)
+    return rows
+
+
+@pytest.fixture()
+def sess(oracle_mod):
+    s = oracle_mod.Session()
+    s.define("\n".join([W.FIB_DEF, W.FACT_DEF, W.SUM_DEF, W.WHEN_DEF]))
+    return s
+
+
+def wrap64(v: int) -> int:
+    return (v + 2**63) % 2**64 - 2**63
+
+
+def fib_py(n: int) -> int:
+    a, b = 0, 1
+    for _ in range(n):
+        a, b = b, a + b
+    return a
+
+
+# ---- paper worked examples (tests/golden/paper_examples.tsv, each row cites PAPER.md) ---------------
+@pytest.mark.parametrize("row", load_tsv("paper_examples.tsv"), ids=lambda r: r[0][:40])
+def test_paper_examples(sess, row):
+    form, expected, steps = row[0], row[1], int(row[2])
+    r = sess.eval1(form)
+    assert r.printed == expected
+    assert r.steps == steps
+
+
+# ---- SURVEY §8(c).12b step/semantics pins ---------------------------------------------------------
+@pytest.mark.parametrize("row", load_tsv("step_pins.tsv"), ids=lambda r: r[0][:40])
+def test_step_pins(sess, row):
+    form, expected, steps = row[0], row[1], int(row[2])
+    r = sess.eval1(form)
+    assert (r.printed, r.steps) == (expected, steps)
+
+
+# ---- closed forms (c.12) -------------------------------------------------------------------------
+def test_fib_closed_form(sess):
+    ns = list(range(0, 23))
+    res = sess.eval("\n".join("(fib %d)" % n for n in ns))
+    for n, r in zip(ns, res):
+        assert r.err == 0
+        assert int(r.printed) == fib_py(n)
+        # S_fib(n) = 27 F(n+1) - 17, from the recurrence body(n) = 20 + body(n-1) + body(n-2)
+        assert r.steps == 27 * fib_py(n + 1) - 17
+
+
+def test_fact_closed_form(sess):
+    ns = list(range(0, 26))
+    res = sess.eval("\n".join("(fact %d)" % n for n in ns))
+    for n, r in zip(ns, res):
+        assert int(r.printed) == wrap64(math.factorial(n))     # int64 two's-complement wrap
+        assert r.steps == (15 * n - 5 if n >= 2 else 10)
+
+
+def test_sum_closed_form_and_depth_limit(sess):
+    ns = [0, 1, 2, 10, 100, 300, 340]
+    res = sess.eval("\n".join("(sum %d)" % n for n in ns))
+    for n, r in zip(ns, res):
+        assert int(r.printed) == n * (n + 1) // 2
+        assert r.steps == 15 * n + 10
+    # depth grows by 3 per recursion level: (sum n) needs depth 3n+4 -> 341 is the first failure at 1024
+    assert sess.eval1("(sum 340)").printed == str(340 * 341 // 2)
+    r = sess.eval1("(sum 341)")
+    assert r.printed == "#<error DEPTH>"
+    assert sess.eval1("(sum 400)").printed == "#<error DEPTH>"
+
+
+def test_depth_limit_is_exact(oracle_mod):
+    # (sum n) reaches depth 3n+4; with max_depth = 3n+4 it succeeds, with 3n+3 it fails.
+    for n in (5, 17, 40):
+        ok = oracle_mod.Session(max_depth=3 * n + 4)
+        ok.define(W.SUM_DEF)
+        assert ok.eval1("(sum %d)" % n).printed == str(n * (n + 1) // 2)
+        bad = oracle_mod.Session(max_depth=3 * n + 3)
+        bad.define(W.SUM_DEF)
+        assert bad.eval1("(sum %d)" % n).printed == "#<error DEPTH>"
+
+
+def test_fuel_limit(oracle_mod):
+    s = oracle_mod.Session(fuel=198)
+    s.define(W.FIB_DEF)
+    r = s.eval1("(fib 5)")                 # needs 199 steps
+    assert (r.printed, r.steps) == ("#<error FUEL>", 199)
+    s2 = oracle_mod.Session(fuel=199)
+    s2.define(W.FIB_DEF)
+    assert s2.eval1("(fib 5)").printed == "5"
+
+
+# ---- brute force: every arithmetic tree of op-depth <= 2 over {+,-,*} and ints {-2..2} -----------------
+def _trees(depth):
+    leaves = [str(v) for v in range(-2, 3)]
+    if depth == 0:
+        for l in leaves:
+            yield l, int(l), 0
+        return
+    subs = list(_trees(depth - 1))
+    for op in "+-*":
+        for (ta, va, oa), (tb, vb, ob) in itertools.product(subs, subs):
+            v = {"+": va + vb, "-": va - vb, "*": va * vb}[op]
+            yield "(%s %s %s)" % (op, ta, tb), v, oa + ob + 1
+
+
+def test_bruteforce_arith_trees(sess):
+    trees = [t for t in _trees(1)] + [t for t in _trees(2)]
+    # keep depth-2 trees exhaustive for the two left shapes, sample the rest deterministically
+    rnd = random.Random(7)
+    if len(trees) > 6000:
+        trees = trees[:2000] + rnd.sample(trees[2000:], 4000)
+    res = sess.eval("\n".join(t for t, _, _ in trees))
+    for (text, val, ops), r in zip(trees, res):
+        assert int(r.printed) == wrap64(val), text
+        assert r.steps == 3 * ops + 1, text          # 2 per list (list + head) + 1 per leaf; leaves = ops+1
+
+
+def test_int64_wrap_random(sess):
+    rnd = random.Random(11)
+    forms, exp = [], []
+    for _ in range(500):
+        a, b, c = (rnd.randrange(-2**63, 2**63) for _ in range(3))
+        op1, op2 = rnd.choice("+-*"), rnd.choice("+-*")
+        f = lambda o, x, y: {"+": x + y, "-": x - y, "*": x * y}[o]
+        forms.append("(%s (%s %d %d) %d)" % (op2, op1, a, b, c))
+        exp.append(wrap64(f(op2, wrap64(f(op1, a, b)), c)))
+    res = sess.eval("\n".join(forms))
+    assert [int(r.printed) for r in res] == exp
+
+
+def _trunc_div(a, b):
+    q = abs(a) // abs(b)
+    return q if (a >= 0) == (b > 0) else -q
+
+
+def test_division_rem_mod_bruteforce(sess):
+    vals = list(range(-7, 8)) + [2**63 - 1, -2**63, 2**62 + 3, -(2**62) - 5]
+    forms, exp = [], []
+    for a in vals:
+        for b in vals:
+            for op in ("/", "rem", "mod"):
+                forms.append("(%s %d %d)" % (op, a, b))
+                if b == 0:
+                    exp.append("#<error DIV0>")
+                elif op == "/":
+                    exp.append(str(wrap64(_trunc_div(a, b))))
+                elif op == "rem":
+                    exp.append(str(a - b * _trunc_div(a, b)))
+                else:
+                    exp.append(str(a % b))            # Python % is floor mod (sign of the divisor)
+    res = sess.eval("\n".join(forms))
+    assert [r.printed for r in res] == exp
+
+
+def test_float_arith_bit_exact(sess):
+    rnd = random.Random(3)
+    forms, exp = [], []
+    for _ in range(400):
+        a, b, c = (rnd.uniform(-1e3, 1e3) for _ in range(3))
+        forms.append("(/ (+ (* %r %r) %r) 2.0)" % (a, b, c))
+        exp.append((a * b + c) / 2.0)
+        forms.append("(- %r %r %r)" % (a, b, c))
+        exp.append(a - b - c)
+        forms.append("(sqrt %r)" % abs(a))
+        exp.append(math.sqrt(abs(a)))
+    res = sess.eval("\n".join(forms))
+    for r, e in zip(res, exp):
+        assert float(r.printed) == e                # bit-exact (shortest repr round-trips)
+
+
+def test_mixed_int_float_fold(sess):
+    # left fold from the first argument; an INT accumulator switches to f64 at the first FLOAT step
+    r = sess.eval("(+ 9007199254740993 1 0.5)\n(+ 9007199254740993 0.5 1)\n(* 3 0.5 3)\n(- 5)\n(- 2.5)")
+    assert float(r[0].printed) == float(9007199254740994) + 0.5
+    assert float(r[1].printed) == (float(9007199254740993) + 0.5) + 1.0
+    assert r[2].printed == "4.5"
+    assert r[3].printed == "-5"
+    assert r[4].printed == "-2.5"
+
+
+def test_c3_closure_float(oracle_mod):
+    wl = W.c3(64)
+    s = oracle_mod.Session()
+    s.define(wl.defs)
+    xs = [float(t) for t in wl.defs.split("'(")[1].rstrip(")\n").split()]
+    r = s.eval1(wl.forms)
+    got = [float(t) for t in r.printed.strip("()").split()]
+    exp = [((0.75 * x) * (0.75 * x) + (x + 1.5)) / 2.0 for x in xs]
+    assert got == exp
+    assert r.steps == 5 + 20 * 64
+
+
+# ---- brute force: list builtins against Python lists -----------------------------------------------
+def _lisp(xs):
+    if xs is None:
+        return "nil"
+    return "(" + " ".join(str(x) for x in xs) + ")" if xs else "nil"
+
+
+def test_list_builtins_bruteforce(sess):
+    rnd = random.Random(5)
+    forms, exp = [], []
+    for _ in range(300):
+        a = [rnd.randint(-9, 9) for _ in range(rnd.randint(0, 5))]
+        b = [rnd.randint(-9, 9) for _ in range(rnd.randint(0, 5))]
+        la, lb = "(list%s)" % "".join(" %d" % v for v in a), "(list%s)" % "".join(" %d" % v for v in b)
+        k = rnd.randint(0, 6)
+        forms += ["(append %s %s)" % (la, lb), "(reverse %s)" % la, "(length %s)" % la,
+                  "(nth %d %s)" % (k, la), "(car %s)" % la, "(cdr %s)" % la,
+                  "(cons %d %s)" % (k, lb), "(equal %s %s)" % (la, lb),
+                  "(append %s)" % la, "(append %s %s %s)" % (la, lb, la)]
+        exp += [_lisp(a + b), _lisp(a[::-1]), str(len(a)),
+                str(a[k]) if k < len(a) else "nil", str(a[0]) if a else "nil", _lisp(a[1:]),
+                _lisp([k] + b), "T" if a == b else "nil", _lisp(a), _lisp(a + b + a)]
+    res = sess.eval("\n".join(forms))
+    assert [r.printed for r in res] == exp
+
+
+def test_list_errors_and_edges(sess):
+    cases = {
+        "(car 5)": "#<error TYPE>", "(length (cons 1 2))": "#<error TYPE>",
+        "(nth -1 (list 1))": "#<error ARG>", "(nth 'a (list 1))": "#<error TYPE>",
+        "(append (cons 1 2) nil)": "#<error TYPE>", "(append nil (cons 1 2))": "(1 . 2)",
+        "(append)": "nil", "(reverse nil)": "nil", "(length nil)": "0", "(car nil)": "nil",
+        "(cdr nil)": "nil", "(cons 1 (cons 2 3))": "(1 2 . 3)", "(list)": "nil",
+        "(equal \"ab\" \"ab\")": "T", "(eq \"ab\" \"ab\")": "nil", "(eq 'a 'a)": "T",
+        "(eq 1.0 1.0)": "T", "(eq 0.0 -0.0)": "nil", "(= 0.0 -0.0)": "T", "(eq car car)": "T",
+        "(symbolp nil)": "T", "(symbolp T)": "T", "(symbolp 'q)": "T", "(symbolp 1)": "nil",
+        "(atom (list))": "T", "(consp (list 1))": "T", "(numberp 1.5)": "T", "(null 0)": "nil",
+        "(not nil)": "T", "(+)": "0", "(*)": "1", "(-)": "#<error ARITY>", "(/)": "#<error ARITY>",
+        "(/ 2)": "0", "(/ 2.0)": "0.5", "(< 1 2 3)": "#<error ARITY>", "(< 1 'a)": "#<error TYPE>",
+        "(/ 1 0 'a)": "#<error TYPE>", "(/ 1 0 2.0)": "#<error DIV0>", "(/ 0 0.0)": "nan",
+        "(/ -9223372036854775808 -1)": "-9223372036854775808",
+        "(rem -9223372036854775808 -1)": "0", "(trunc 2.9)": "2", "(trunc -2.9)": "-2",
+        "(trunc 1e300)": "#<error ARG>", "(trunc (/ 0 0.0))": "#<error ARG>", "(trunc 7)": "7",
+        "(float 3)": "3.0", "(sqrt 4)": "2.0", "(sqrt -1)": "nan", "(sqrt 'a)": "#<error TYPE>",
+        "(+ 1e308 1e308)": "inf", "(- 1e308 -1e308 )": "inf", "(+ 0.1 0.2)": "0.30000000000000004",
+        "(quote)": "#<error SYNTAX>", "(quote 1 2)": "#<error SYNTAX>", "(if 1 2 3 4)": "#<error SYNTAX>",
+        "(lambda)": "#<error SYNTAX>", "(lambda (1) 1)": "#<error SYNTAX>",
+        "(lambda (car) 1)": "#<error SYNTAX>", "((lambda () 7))": "7", "((lambda (x)) 1)": "nil",
+        "((lambda (x x) x) 1 2)": "1", "((lambda (x) x))": "#<error ARITY>",
+        "(let ((a 1) (a 2)) a)": "1", "(let ((a 1)) (let ((a 2) (b a)) b))": "1",
+        "(let (a) a)": "#<error SYNTAX>", "(let ((a)) a)": "#<error SYNTAX>", "(let ())": "nil",
+        "(progn)": "nil", "(defun f (x) x)": "#<error DEFINE_IN_BATCH>",
+        "(defmacro m (x) x)": "#<error DEFINE_IN_BATCH>", "\"a b\"": "\"a b\"",
+        "(||| 0 + nil)": "nil", "(||| -1 + nil)": "#<error ARG>", "(||| 3 + (1 2))": "#<error ARG>",
+        "(||| 2 + (1 2 3) (4 5))": "(5 7)", "(||| 2 if (1 2))": "#<error TYPE>",
+        "(||| 'a + (1))": "#<error TYPE>", "(||| 1 +)": "#<error ARITY>",
+        "(||| 2 (lambda (x y) x) (1 2))": "#<error ARITY>", "(||| 1 + (cons 1 2))": "#<error ARG>",
+        "(||| 2 car (1 2))": "#<error TYPE>", "(||| 2 when (1 2))": "#<error TYPE>",
+        "(1 . 2)": "(1 . 2)", "(when 1 2 3)": "#<error ARITY>", "(fib 5 6)": "#<error ARITY>",
+        "((list 1 2) 3)": "((1 2) 3)", "(nil 1)": "(nil 1)", "(T (+ 1 1))": "(T 2)",
+        "(car (cons 1 2) 3)": "#<error ARITY>", "(equal (list 1 (list 2 \"x\")) (list 1 (list 2 \"x\")))": "T",
+        "#<foo>": "#<foo>", "(eq fib fib)": "T", "fib": "#<lambda>", "when": "#<macro>",
+        "car": "#<builtin car>", "if": "#<special if>", "(list car if)": "(#<builtin car> #<special if>)",
+    }
+    forms = list(cases)
+    res = sess.eval("\n".join(forms))
+    got = {f: r.printed for f, r in zip(forms, res)}
+    assert got == cases
+
+
+def test_dotted_data_is_a_symbol_not_syntax(sess):
+    # c.1 has no dotted-pair syntax: "." reads as a symbol; improper lists only come from cons
+    r = sess.eval1("(list 1 . 2)")
+    assert r.printed == "(1 . 2)"
+    r = sess.eval1("(car (list (cons 1 2)))")
+    assert r.printed == "(1 . 2)"
+
+
+def test_eval_of_improper_list_is_syntax_error(oracle_mod):
+    s = oracle_mod.Session()
+    s.define("(defmacro bad () (cons 1 2))")
+    r = s.eval1("(bad)")
+    assert r.printed == "#<error SYNTAX>"
+    assert r.steps == 2 + 4 + 1                        # list + head, body (cons 1 2), then the expansion
+
+
+# ---- invariants --------------------------------------------------------------------------------------
+def test_macro_equals_hand_expansion(sess, oracle_mod):
+    rnd = random.Random(9)
+    for _ in range(100):
+        c = rnd.choice(["(< %d %d)" % (rnd.randint(-3, 3), rnd.randint(-3, 3)), "nil", "T", "1"])
+        x = "(+ %d %d)" % (rnd.randint(-9, 9), rnd.randint(-9, 9))
+        m = sess.eval1("(when %s %s)" % (c, x))
+        h = sess.eval1("(if %s %s nil)" % (c, x))
+        assert m.printed == h.printed
+        # expansion body (list 'if c x nil) costs 7 steps; the macro call adds list + head
+        assert m.steps == 2 + 7 + h.steps
+
+
+def test_par_equals_sequential_map(sess):
+    rnd = random.Random(4)
+    for _ in range(30):
+        n = rnd.randint(0, 8)
+        a = [rnd.randint(0, 12) for _ in range(n + rnd.randint(0, 2))]
+        b = [rnd.randint(-5, 5) for _ in range(n + rnd.randint(0, 2))]
+        la, lb = "(%s)" % " ".join(map(str, a)) if a else "nil", "(%s)" % " ".join(map(str, b)) if b else "nil"
+        par = sess.eval1("(||| %d fib '%s)" % (n, la))
+        seq = sess.eval1("(list%s)" % "".join(" (fib %d)" % v for v in a[:n]))
+        assert par.printed == seq.printed
+        par2 = sess.eval1("(||| %d - '%s '%s)" % (n, la, lb))
+        assert par2.printed == _lisp([wrap64(x - y) for x, y in zip(a[:n], b[:n])])
+
+
+def test_print_read_idempotent(sess, oracle_mod):
+    rnd = random.Random(2)
+
+    def datum(d):
+        k = rnd.randint(0, 6 if d < 3 else 4)
+        if k == 0:
+            return str(rnd.randint(-10**18, 10**18))
+        if k == 1:
+            return repr(rnd.uniform(-1e6, 1e6))
+        if k == 2:
+            return rnd.choice(["a", "foo-bar", "|||", "+", "E", "1+", "x.y", "nil", "T"])
+        if k == 3:
+            return '"s %d"' % rnd.randint(0, 9)
+        if k == 4:
+            return repr(rnd.choice([1e300, -0.0, 5e-324, 1.5, 2.0, 1e16, 123456.789]))
+        return "(%s)" % " ".join(datum(d + 1) for _ in range(rnd.randint(0, 4)))
+
+    text = "\n".join(datum(0) for _ in range(300))
+    once = sess.read_print(text)
+    twice = sess.read_print("\n".join(once))
+    assert once == twice
+
+
+def test_reader_classification(sess):
+    toks = {"+": "+", "-": "-", "E": "E", "1+": "1+", "+5": "5", "-0": "0", "1.": "1.0", ".5": "0.5",
+            "1e3": "1000.0", "1E-2": "0.01", "-.5e1": "-5.0", "1.5.2": "1.5.2", "e5": "e5",
+            "nil": "nil", "T": "T", "t": "t", "NIL": "NIL", "()": "nil", "|||": "|||"}
+    out = sess.read_print("\n".join(toks))
+    assert dict(zip(toks, out)) == toks
+
+
+def test_reader_errors(oracle_mod):
+    s = oracle_mod.Session()
+    for bad in ["(+ 1 2", ")", "(a))", '"abc', "99999999999999999999", "'"]:
+        with pytest.raises(oracle_mod.OracleError):
+            s.read_print(bad)
+
+
+def test_global_persistence(oracle_mod):
+    # the environment persists across inputs; late binding (L447-448)
+    s = oracle_mod.Session()
+    s.define("(define k 1) (define g (lambda (x) (+ x k)))")
+    assert s.eval1("(g 10)").printed == "11"
+    s.define("(define k 5)")
+    assert s.eval1("(g 10)").printed == "15"
+
+
+def test_define_failure_leaves_no_binding(oracle_mod):
+    s = oracle_mod.Session()
+    with pytest.raises(oracle_mod.OracleError, match="form 1: DIV0"):
+        s.define("(define a 1) (define b (/ 1 0)) (define c 3)")
+    assert s.eval("a\nb\nc") and [r.printed for r in s.eval("a\nb\nc")] == ["1", "b", "c"]
+
+
+def test_generators_deterministic():
+    for name, gen, kw in [("C1", W.c1, {"n": 50}), ("C2", W.c2, {"n": 50}), ("C4", W.c4, {"n": 50}),
+                          ("C5", W.c5, {"n": 50}), ("C3", W.c3, {"n": 50})]:
+        a, b = gen(**kw), gen(**kw)
+        assert a.sha256() == b.sha256(), name
+
+
+def test_generated_batches_run_clean(oracle_mod):
+    # every generated form evaluates without an error under the oracle (sanity of the recipes)
+    for wl in (W.c1(200), W.c2(40, lo=5, hi=12), W.c4(300), W.c5(300)):
+        s = oracle_mod.Session()
+        if wl.defs:
+            s.define(wl.defs)
+        res = s.eval(wl.forms)
+        assert len(res) == wl.nforms
+        assert all(r.err == 0 for r in res), [r for r in res if r.err][:3]
