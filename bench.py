@@ -1,0 +1,412 @@
+#!/usr/bin/env python3
+"""bench.py — forms/sec and eval-steps/sec of the CuLi hot path on B200 (BASELINE.json `metric`).
+
+One "step" = one pass of the whole hot path over one batch of synthetic input already resident in HBM:
+dispatch (classify + sort), the eval kernel, result export, and (N > 1) the NCCL all-gather of the
+result records.  Default workload: configs[1] = C2, 65,536 (fib n) forms with n in 15..22 per GPU
+(weak scaling: every rank evaluates its own 65,536-form shard of an N x 65,536 batch; the global
+environment is defined on rank 0 and broadcast over NCCL once per session).
+
+  python bench.py [--gpus N] [--steps K] [--warmup W] [--workload C2] [--impl culi|reference]
+
+`--impl reference` times the oracle (the plain recursive CPU interpreter, oracle/) on the host cores on a
+bounded sample of the same workload (this tier has no runnable reference implementation).
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+from paper_conf_cluster_subdbn18_b200 import workloads as W  # noqa: E402
+
+L2_FLUSH_BYTES = 512 << 20          # > 126 MB L2: flushed between timed iterations
+PEAKS_PATH = os.path.join(ROOT, "MEASURED_PEAKS.json")
+WORKLOADS = {
+    "C1": lambda n_rank, rank: W.c1(1024 * n_rank),
+    "C2": lambda n_rank, rank: W.c2(65536 * n_rank),
+    "C3": lambda n_rank, rank: W.c3(1 << 20),
+    "C4": lambda n_rank, rank: W.c4(262144 * n_rank),
+    "C5": lambda n_rank, rank: W.c5(16777216),
+}
+SCALING = {"C1": "weak", "C2": "weak", "C3": "replicas", "C4": "weak", "C5": "strong"}
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--workload", default=os.environ.get("CULI_WORKLOAD", "C2"))
+    ap.add_argument("--impl", default="culi", choices=["culi", "reference"])
+    ap.add_argument("--e2e-steps", type=int, default=3)
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--flags", type=int, default=0)
+    return ap.parse_args()
+
+
+# ------------------------------------------------------------------------------------------------ clocks
+class ClockSampler:
+    """nvidia-smi clocks + throttle reasons sampled during the timed region (B200_PROFILING.md)."""
+
+    Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,"
+         "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+         "clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, device: int):
+        self.device = device
+        self.samples = []
+        self._stop = threading.Event()
+        self._t = None
+
+    def _run(self):
+        while not self._stop.is_set():
+            try:
+                out = subprocess.run(["nvidia-smi", "-i", str(self.device), "--query-gpu=" + self.Q,
+                                      "--format=csv,noheader,nounits"], capture_output=True, text=True,
+                                     timeout=5).stdout.strip()
+                if out:
+                    self.samples.append([x.strip() for x in out.split(",")])
+            except Exception:  # noqa: BLE001
+                pass
+            self._stop.wait(0.2)
+
+    def __enter__(self):
+        self._t = threading.Thread(target=self._run, daemon=True)
+        self._t.start()
+        return self
+
+    def __exit__(self, *a):
+        self._stop.set()
+        self._t.join(timeout=10)
+
+    def summary(self):
+        if not self.samples:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["unsampled"]}
+        sm = [float(s[0]) for s in self.samples if s[0].replace(".", "").isdigit()]
+        mx = [float(s[1]) for s in self.samples if s[1].replace(".", "").isdigit()]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[k] for s in self.samples for k in range(4)
+                          if len(s) > 2 + k and s[2 + k].lower() == "active"})
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": reasons, "samples": len(self.samples)}
+
+
+def host_cores():
+    try:
+        return len(os.sched_getaffinity(0))
+    except Exception:  # noqa: BLE001
+        return os.cpu_count() or 1
+
+
+# ---------------------------------------------------------------------------------------- oracle legs
+def cpu_sample(wl: W.Workload, max_forms: int):
+    """A bounded, strided sample of the workload's forms (the same text the GPU evaluates)."""
+    lines = wl.form_lines()
+    if wl.units != wl.nforms:            # ||| workloads: a shorter map of the same closure
+        return wl, "full workload (single ||| form)"
+    stride = max(1, len(lines) // max_forms)
+    sample = lines[::stride][:max_forms]
+    return (W.Workload(wl.name, wl.defs, "\n".join(sample) + "\n", len(sample), len(sample), wl.seed),
+            "every %d-th form of %s (%d of %d forms)" % (stride, wl.name, len(sample), len(lines)))
+
+
+def run_oracle(wl: W.Workload, max_forms: int, threads: int):
+    import oracle
+    sample, desc = cpu_sample(wl, max_forms)
+    s = oracle.Session()
+    if sample.defs:
+        s.define(sample.defs)
+    r = s.eval_batch(sample.forms, nthreads=threads, want_output=False)
+    return sample, desc, r
+
+
+ORACLE_SAMPLE = {"C1": 1024, "C2": 4096, "C3": 1 << 20, "C4": 262144, "C5": 262144}
+
+
+def reference_arm(args):
+    """--impl reference: the oracle on the host cores, rank 0 only (others exit 0)."""
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return
+    wl = WORKLOADS[args.workload](1, 0)
+    threads = host_cores()
+    times, steps_tot, units = [], 0, 0
+    for it in range(args.warmup + args.steps):
+        sample, desc, r = run_oracle(wl, ORACLE_SAMPLE[args.workload], threads)
+        if it >= args.warmup:
+            times.append(r.seconds)
+            steps_tot += r.total_steps
+            units += sample.units
+    t = sum(times)
+    value = units / t
+    line = {
+        "metric": "forms/sec", "value": value, "unit": "forms/s", "impl": "reference",
+        "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
+        "ms_per_step": 1e3 * t / len(times), "higher_is_better": True, "scaling": SCALING[args.workload],
+        "vs_baseline": None, "dtype": "int64+f64", "data": "synthetic",
+        "eval_steps_per_sec": steps_tot / t,
+        "config": {"workload": "%s (configs[%d])" % (args.workload, int(args.workload[1]) - 1 if args.workload != "C0" else 0),
+                   "sample": desc},
+        "cpu_baseline": {"value": value, "unit": "forms/s", "cores": threads, "kind": "oracle",
+                         "sample": desc},
+        "e2e": {"value": value, "unit": "forms/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }
+    print(json.dumps(line), flush=True)
+
+
+# ------------------------------------------------------------------------------------------- culi leg
+def load_peaks():
+    try:
+        with open(PEAKS_PATH) as f:
+            return json.load(f), "measured"
+    except Exception:  # noqa: BLE001
+        return {"hbm_gbs": 6650.0, "sm_max_mhz": 1965.0}, "fallback"
+
+
+def load_inst_profile(workload: str):
+    """Warp instructions per eval-kernel launch from the committed ncu capture (profiles/)."""
+    p = os.path.join(ROOT, "profiles", "eval_inst_%s.json" % workload.lower())
+    try:
+        with open(p) as f:
+            return json.load(f)
+    except Exception:  # noqa: BLE001
+        return None
+
+
+def culi_arm(args):
+    import torch
+    import torch.distributed as dist
+    from paper_conf_cluster_subdbn18_b200 import culi
+    from paper_conf_cluster_subdbn18_b200 import build as B
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    if world != args.gpus:
+        args.gpus = world
+    torch.cuda.set_device(local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    B.build()
+    culi.load()
+    stream = torch.cuda.current_stream()
+    dev = torch.device("cuda", local)
+
+    # ---- workload + shard (rank r takes forms i mod k == r)
+    wl = WORKLOADS[args.workload](world if SCALING[args.workload] == "weak" else 1, rank)
+    if SCALING[args.workload] in ("weak", "strong") and world > 1:
+        shard_text, shard_idx = W.shard_lines(wl.forms, rank, world)
+    else:
+        shard_text, shard_idx = wl.forms, list(range(wl.nforms))
+    units_rank = wl.units if wl.units != wl.nforms else len(shard_idx)
+
+    heap = 1 << 26 if args.workload in ("C1", "C2") else 1 << 30
+    ctx = culi.Context(device=local, stream=stream.cuda_stream, heap_nodes=heap, flags=args.flags)
+
+    # ---- define on rank 0, broadcast the environment over NCCL (a3 + a10)
+    t_env = None
+    if world == 1:
+        if wl.defs:
+            ctx.define(wl.defs)
+    else:
+        size = torch.zeros(1, dtype=torch.int64, device=dev)
+        if rank == 0:
+            if wl.defs:
+                ctx.define(wl.defs)
+            size[0] = ctx.env_export_size()
+        dist.broadcast(size, 0)
+        buf = torch.empty(int(size.item()), dtype=torch.uint8, device=dev)
+        if rank == 0:
+            ctx.env_export(buf.data_ptr(), buf.numel())
+        torch.cuda.synchronize()
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        e0.record()
+        dist.broadcast(buf, 0)
+        e1.record()
+        torch.cuda.synchronize()
+        t_env = e0.elapsed_time(e1)
+        if rank != 0:
+            ctx.env_import(buf.data_ptr(), buf.numel())
+
+    # ---- read (host, outside the timed region) + upload (a1, a2)
+    t0 = time.perf_counter()
+    img = ctx.read(shard_text)
+    t_read = time.perf_counter() - t0
+    h = ctx.upload(img)
+    nrec = ctx.records_device(None)
+    rec = torch.empty(max(nrec, 8), dtype=torch.uint8, device=dev)
+    gathered = torch.empty(world * rec.numel(), dtype=torch.uint8, device=dev) if world > 1 else None
+    flush = torch.empty(L2_FLUSH_BYTES, dtype=torch.uint8, device=dev)
+
+    def step():
+        ctx.eval_uploaded(h)
+        if world > 1:
+            ctx.records_device(rec.data_ptr(), rec.numel())
+            dist.all_gather_into_tensor(gathered, rec)
+
+    for _ in range(args.warmup):
+        step()
+    torch.cuda.synchronize()
+    res = ctx.fetch_results(h)                  # parity-relevant numbers of this exact batch
+    total_steps, n_err = res.totals()
+    del res
+
+    # ---- timed region: K steps, CUDA events on the launching stream, L2 flushed between steps
+    ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
+          for _ in range(args.steps)]
+    eval_ms, disp_ms, exp_ms = [], [], []
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    with ClockSampler(local) as clk:
+        for k in range(args.steps):
+            flush.fill_(k & 0xff)
+            ev[k][0].record(stream)
+            step()
+            ev[k][1].record(stream)
+            ms3, kernels, high = ctx.last_timing()
+            disp_ms.append(ms3[0])
+            eval_ms.append(ms3[1])
+            exp_ms.append(ms3[2])
+        torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    step_ms = [a.elapsed_time(b) for a, b in ev]
+    t_rank = sum(step_ms) / 1e3
+    t_max = t_rank
+    if world > 1:
+        tt = torch.tensor([t_rank], dtype=torch.float64, device=dev)
+        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        t_max = float(tt.item())
+        agg = torch.tensor([units_rank, total_steps], dtype=torch.float64, device=dev)
+        dist.all_reduce(agg)
+        units_all, steps_all = float(agg[0].item()), float(agg[1].item())
+    else:
+        units_all, steps_all = float(units_rank), float(total_steps)
+    value = units_all * args.steps / t_max
+    steps_per_sec = steps_all * args.steps / t_max
+
+    # ---- e2e: the public C-ABI with host buffers (H2D of the image, D2H of records + payload)
+    h2d = img.nnodes * 9 + img.nforms * 4
+    e2e_ms, d2h = [], 0
+    ctx.release(h)
+    for k in range(args.e2e_steps):
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        if world > 1:
+            dist.barrier()
+        a.record(stream)
+        r = ctx.eval_batch(img)
+        if world > 1:
+            blob = r.serialize()
+            t = torch.frombuffer(bytearray(blob), dtype=torch.uint8).to(dev)
+            sizes = [torch.zeros(1, dtype=torch.int64, device=dev) for _ in range(world)]
+            dist.all_gather(sizes, torch.tensor([t.numel()], dtype=torch.int64, device=dev))
+            mx = int(max(s.item() for s in sizes))
+            pad = torch.zeros(mx, dtype=torch.uint8, device=dev)
+            pad[: t.numel()] = t
+            outs = [torch.empty(mx, dtype=torch.uint8, device=dev) for _ in range(world)]
+            dist.all_gather(outs, pad)
+            if rank == 0:
+                blobs = [o[: int(s.item())].cpu().numpy().tobytes() for o, s in zip(outs, sizes)]
+                idx = [list(range(q, wl.nforms, world)) for q in range(world)]
+                culi.merge_results(blobs, idx)
+        else:
+            d2h = len(r.serialize())
+        b.record(stream)
+        torch.cuda.synchronize()
+        e2e_ms.append(a.elapsed_time(b))
+        del r
+    t_e2e = sum(e2e_ms) / 1e3
+    if world > 1:
+        tt = torch.tensor([t_e2e], dtype=torch.float64, device=dev)
+        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        t_e2e = float(tt.item())
+    e2e_value = units_all * len(e2e_ms) / t_e2e
+
+    if rank != 0:
+        if world > 1:
+            dist.barrier()
+            dist.destroy_process_group()
+        return
+
+    # ---- roofline of the dominant kernel (the eval kernel)
+    peaks, peak_src = load_peaks()
+    eval_s = statistics.mean(eval_ms) / 1e3
+    clocks = clk.summary()
+    prof = load_inst_profile(args.workload)
+    if args.workload == "C3":
+        # algorithmic bytes per element: read cons + float node, write cons + float node (9 B each)
+        traffic_alg = 36.0 * wl.units
+        ach = traffic_alg / eval_s / 1e9
+        roof = {"bound": "hbm", "achieved": ach, "peak": peaks["hbm_gbs"], "unit": "GB/s",
+                "frac": ach / peaks["hbm_gbs"], "traffic": prof.get("dram_bytes") if prof else None,
+                "peak_source": peak_src}
+    else:
+        sm_mhz = peaks.get("sm_max_mhz", 1965.0)
+        peak_inst = 148 * 4 * sm_mhz * 1e6 / 1e9          # warp instructions / ns -> G warp-inst/s
+        inst = prof.get("warp_inst_per_launch") if prof else None
+        ach = inst / eval_s / 1e9 if inst else None
+        roof = {"bound": "alu", "achieved": ach, "peak": peak_inst, "unit": "Gwarp-inst/s",
+                "frac": (ach / peak_inst) if ach else None,
+                "traffic": prof.get("dram_bytes") if prof else None,
+                "peak_source": "148 SMs x 4 SMSP x 1 warp-inst/clk x %.0f MHz (B200_PROFILING.md)" % sm_mhz,
+                "achieved_source": ("ncu smsp__inst_executed.sum of profiles/eval_inst_%s.json / live "
+                                    "eval-kernel time" % args.workload.lower()) if inst else None}
+
+    cpu = None
+    if world == 1 and not args.no_cpu_baseline:
+        threads = host_cores()
+        sample, desc, r = run_oracle(wl, ORACLE_SAMPLE[args.workload], threads)
+        cpu = {"value": sample.units / r.seconds, "unit": "forms/s", "cores": threads, "kind": "oracle",
+               "sample": desc, "eval_steps_per_sec": r.total_steps / r.seconds}
+
+    ms_step = 1e3 * t_max / args.steps
+    line = {
+        "metric": "forms/sec", "value": value, "unit": "forms/s", "n_gpus": world, "steps": args.steps,
+        "warmup": args.warmup, "ms_per_step": ms_step, "higher_is_better": True,
+        "scaling": SCALING[args.workload] if world > 1 else "weak", "vs_baseline": None,
+        "dtype": "int64+f64", "data": "synthetic",
+        "eval_steps_per_sec": steps_per_sec,
+        "config": {"workload": "%s (BASELINE configs[%d]): %s" % (
+                       args.workload, {"C1": 0, "C2": 1, "C3": 2, "C4": 3, "C5": 4}.get(args.workload, 0),
+                       {"C1": "1,024 integer arithmetic forms", "C2": "65,536 (fib n), n in 15..22",
+                        "C3": "(||| 1048576 f xs), closure+let+float", "C4": "262,144 macro forms",
+                        "C5": "16.8M mixed forms"}[args.workload]),
+                   "forms_per_gpu": len(shard_idx), "units_per_gpu": units_rank,
+                   "parallelism": "dp%d" % world, "l2": "flushed between timed steps (512 MB write)",
+                   "binning": not (args.flags & 1)},
+        "gpu_launches": kernels * args.steps,
+        "phases_ms": {"dispatch": statistics.mean(disp_ms), "eval": statistics.mean(eval_ms),
+                      "export": statistics.mean(exp_ms)},
+        "errors_in_batch": n_err, "read_s": t_read, "env_broadcast_ms": t_env,
+        "roofline": roof,
+        "cpu_baseline": cpu,
+        "e2e": {"value": e2e_value, "unit": "forms/s", "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
+                "ms_per_step": 1e3 * t_e2e / len(e2e_ms)},
+        "clocks": clocks,
+    }
+    print(json.dumps(line), flush=True)
+    if world > 1:
+        dist.barrier()
+        dist.destroy_process_group()
+
+
+def main():
+    args = parse()
+    if args.impl == "reference":
+        reference_arm(args)
+    else:
+        culi_arm(args)
+
+
+if __name__ == "__main__":
+    main()

@@ -1,0 +1,166 @@
+/* =====================================================================================================
+ * culi.h — C-ABI of libculi.so, the B200-native (sm_100a) hot path of CuLi
+ * ("And Now for Something Completely Different: Running Lisp on GPUs", Süß, Döring, Brinkmann, Nagel;
+ * /root/reference/PAPER.md, cited "PAPER Lnnn §x").
+ *
+ * The calls follow the paper's read-eval-print split: the host reads text into a compact node array
+ * (§III-B.b, moved to the host per L85-89), `culi_define` persists global bindings on the
+ * device (the global environment persists for the session, L98-101, L389), `culi_eval_batch` evaluates N
+ * independent forms on the device (eval: L438-462 §III-B.c; independent parallel evaluation: L546-589
+ * §III-D), and results are copied back for printing on the host (L463-475 §III-B.d).
+ * Semantics of every form are SURVEY.md §8(c) / DESIGN.md §3.
+ *
+ * Conventions (all entry points):
+ *   - Return value: 0 = CULI_OK, negative = API failure (culi_status).  Lisp-level errors (type errors,
+ *     arity, depth, fuel ...) are NOT API failures: they are per-form result codes (culi_err).
+ *   - Plain pointers and sizes only.  Host pointers unless the name says dev_*.
+ *   - Ownership: the caller owns every buffer it passes in (text, out buffers, device buffers given in
+ *     culi_opts).  The library owns culi_ctx / culi_image / culi_results until the matching *_free /
+ *     culi_shutdown.  No call retains a caller pointer after it returns, except opts->stream.
+ *   - Threading: one ctx per host thread; every device operation of a ctx is ordered on opts->stream.
+ *   - There is no CPU fallback: without a usable CUDA device culi_init fails with CULI_E_CUDA.
+ * ===================================================================================================== */
+#ifndef CULI_H
+#define CULI_H
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef enum {
+  CULI_OK = 0,
+  CULI_E_ARG = -1,        /* bad argument, NULL pointer, buffer too small (needed size reported)      */
+  CULI_E_PARSE = -2,      /* read error: unbalanced parens (L484-486), unterminated string, int64
+                             literal out of range; *err_offset = byte offset                             */
+  CULI_E_HEAP_FULL = -3,  /* device heap / stacks exhausted: the batch results are invalid            */
+  CULI_E_CUDA = -4,       /* a CUDA runtime call failed (no device, launch failure ...)               */
+  CULI_E_NCCL = -5,       /* reserved for collective failures reported by the caller's binding          */
+  CULI_E_DEFINE = -6,     /* culi_define: a definition form evaluated to an error (*failed_index)       */
+  CULI_E_STATE = -7       /* call out of order (e.g. import into a ctx that already has definitions)   */
+} culi_status;
+
+/* Per-form Lisp error codes.  CULI_ERR_OOM is a resource error, never parity-checked. */
+typedef enum {
+  CULI_ERR_NONE = 0, CULI_ERR_TYPE = 1, CULI_ERR_ARITY = 2, CULI_ERR_DIV0 = 3, CULI_ERR_SYNTAX = 4,
+  CULI_ERR_ARG = 5, CULI_ERR_DEPTH = 6, CULI_ERR_FUEL = 7, CULI_ERR_DEFINE_IN_BATCH = 8, CULI_ERR_OOM = 9
+} culi_err;
+
+/* Value tags as reported by culi_result_info. */
+typedef enum {
+  CULI_NIL = 0, CULI_T = 1, CULI_INT = 2, CULI_FLOAT = 3, CULI_STRING = 4, CULI_SYMBOL = 5,
+  CULI_CONS = 6, CULI_BUILTIN = 7, CULI_SPECIAL = 8, CULI_CLOSURE = 9, CULI_MACRO = 10,
+  CULI_ERROR = 13
+} culi_tag;
+
+typedef struct culi_ctx culi_ctx;
+typedef struct culi_image culi_image;
+typedef struct culi_results culi_results;
+
+typedef struct {
+  int device;              /* CUDA device ordinal                                                       */
+  void* stream;            /* cudaStream_t (e.g. torch.cuda.current_stream().cuda_stream); NULL = the
+                              legacy default stream.  Borrowed: must outlive the ctx.                    */
+  uint64_t heap_nodes;     /* node capacity of the SoA heap (tag u8 + word u64 per node); 0 = default
+                              (64 Mi nodes = 576 MB).  The paper's node array was fixed at compile time
+                              (L361-365); here it is sized at init.                                     */
+  uint32_t max_depth;      /* canonical eval-nesting limit (c.10); 0 = default 1024; at most 4095         */
+  uint64_t fuel;           /* canonical step limit per top-level form (c.10); 0 = default 2^40            */
+  uint32_t vstack_entries; /* value-stack entries per resident thread; 0 = default 4096                   */
+  uint32_t slots;          /* resident eval threads (stack slots); 0 = default (SM count x 512)          */
+  uint32_t flags;          /* CULI_F_* below                                                              */
+} culi_opts;
+
+#define CULI_F_NO_BINNING 1u   /* evaluate forms in input order (no classify+sort dispatch, §8(a)5)     */
+#define CULI_F_NO_FANOUT  2u   /* evaluate top-level ||| forms in one thread (no fan-out, §8(a)6)        */
+#define CULI_F_NO_STAGING 4u   /* do not stage the global frame / hot code in shared memory (§8(a)4)     */
+#define CULI_F_NO_VOTING  8u   /* disable warp opcode voting in the eval loop                            */
+
+/* Fill *opts with defaults (device 0, default stream, default sizes). */
+void culi_default_opts(culi_opts* opts);
+
+/* Create a session: allocates the device heap, stacks and global table on opts->device and installs the
+ * builtins and special forms in the global environment (the master thread set up the
+ * global environment; here it is one host->device copy).  Returns CULI_E_CUDA without a device. */
+int culi_init(const culi_opts* opts, culi_ctx** out);
+void culi_shutdown(culi_ctx* ctx);
+
+/* ---- read (host) ---------------------------------------------------------------------------------
+ * Parse `len` bytes of text into a compact node image; every top-level
+ * datum is one form.  Symbols are interned into ctx's table (dense u32 ids).  On CULI_E_PARSE,
+ * *err_offset (if non-NULL) receives the byte offset of the offending character / opening paren. */
+int culi_read(culi_ctx* ctx, const char* text, size_t len, culi_image** out, size_t* err_offset);
+uint32_t culi_image_nforms(const culi_image* img);
+uint64_t culi_image_nnodes(const culi_image* img);
+void culi_image_free(culi_image* img);
+
+/* ---- define (device, sequential) -----------------------------------------------------------------
+ * Upload `defs` into the persistent heap segment and evaluate its forms in order on the device with
+ * define/defun/defmacro enabled; bindings persist until culi_shutdown (L98-101, L316-319, L346-347).
+ * Stops at the first form whose evaluation errors: returns CULI_E_DEFINE, *failed_index = its index,
+ * *failed_err = its culi_err; that binding is not created (earlier ones stay). */
+int culi_define(culi_ctx* ctx, const culi_image* defs, uint32_t* failed_index, uint8_t* failed_err);
+
+/* ---- eval (device, data-parallel) ------------------------------------------------------------------
+ * Evaluate the image's forms as N independent evaluations (one thread each; top-level ||| forms fan out
+ * over threads).  The global environment is read-only: define/defun/defmacro yield the
+ * per-form error CULI_ERR_DEFINE_IN_BATCH.  Synchronous on ctx's stream: on return the results (records
+ * + serialized list/string values) are in host memory and the batch's heap segment has been released.
+ * On CULI_E_HEAP_FULL no results are returned. */
+int culi_eval_batch(culi_ctx* ctx, const culi_image* forms, culi_results** out);
+
+/* Device-resident variant for timing (bench.py "value"): the image must already be uploaded with
+ * culi_upload (done once); each call runs relocate-free dispatch + eval + export on the device and
+ * leaves records on the device.  No host copies, no host synchronisation. */
+int culi_upload(culi_ctx* ctx, const culi_image* forms, uint32_t* batch_handle);
+int culi_eval_uploaded(culi_ctx* ctx, uint32_t batch_handle);
+/* Copy the device-resident results of the last culi_eval_uploaded call to the host (synchronises). */
+int culi_fetch_results(culi_ctx* ctx, uint32_t batch_handle, culi_results** out);
+/* Release an uploaded batch (resets the heap to the post-define mark). */
+int culi_release(culi_ctx* ctx, uint32_t batch_handle);
+
+/* ---- results (host) --------------------------------------------------------------------------------- */
+uint32_t culi_results_count(const culi_results* r);
+/* tag: culi_tag (CULI_ERROR when err != 0); err: culi_err; steps: canonical eval steps (c.4). */
+int culi_result_info(const culi_results* r, uint32_t i, uint8_t* tag, uint8_t* err, uint64_t* steps);
+int culi_result_int(const culi_results* r, uint32_t i, int64_t* v);     /* CULI_E_ARG if not INT      */
+int culi_result_float(const culi_results* r, uint32_t i, double* v);    /* CULI_E_ARG if not FLOAT    */
+/* Print result i into buf[cap] (NUL-terminated).  *needed = length without the NUL,
+ * always set; if cap <= *needed the text is truncated and CULI_E_ARG is returned. */
+int culi_print(const culi_results* r, uint32_t i, char* buf, size_t cap, size_t* needed);
+/* Sum of steps over all forms, and the number of forms with err != 0. */
+int culi_results_totals(const culi_results* r, uint64_t* total_steps, uint32_t* n_errors);
+void culi_results_free(culi_results* r);
+
+/* ---- distributed hooks ------------------------------------------------------------------
+ * The collective itself is issued by the caller (torch.distributed NCCL broadcast / all_gather) on a
+ * device buffer, ordered on ctx's stream.
+ * culi_env_export: pack the global environment (global table + persistent heap segment + symbol names)
+ *   into dev_buf[cap] (device memory).  *bytes = size needed (always set); CULI_E_ARG if cap too small.
+ * culi_env_import: replace this ctx's (empty) global environment by the packed image in dev_buf; the
+ *   ctx must not have run culi_define yet (CULI_E_STATE otherwise).  Both synchronise ctx's stream. */
+int culi_env_export(culi_ctx* ctx, void* dev_buf, size_t cap, size_t* bytes);
+int culi_env_import(culi_ctx* ctx, const void* dev_buf, size_t bytes);
+/* Serialize host results into a self-contained byte blob (records + payload + symbol names) and
+ * rebuild results from per-rank blobs: form_index[rank][k] = global index of that rank's k-th form. */
+/* Pack the device-resident records of the last culi_eval_uploaded call into dev_buf (device memory, for
+ * an NCCL all_gather): [tag u8 x n][err u8 x n][pad to 8][steps u64 x n][word u64 x n].  Stream-ordered,
+ * no host synchronisation.  *bytes = size needed (always set); CULI_E_ARG if cap is too small. */
+int culi_records_device(culi_ctx* ctx, void* dev_buf, size_t cap, size_t* bytes);
+int culi_results_serialize(const culi_results* r, void* buf, size_t cap, size_t* bytes);
+int culi_results_merge(const void* const* blobs, const size_t* sizes, int nranks,
+                       const uint32_t* const* form_index, culi_results** merged);
+
+/* ---- diagnostics ---------------------------------------------------------------------------------- */
+const char* culi_status_string(int status);
+const char* culi_error_name(uint8_t err);
+/* Device time in ms of the phases of the last eval call: [0] dispatch, [1] eval, [2] export; and the
+ * number of kernels launched by that call.  Heap high-water mark in nodes. */
+int culi_last_timing(const culi_ctx* ctx, float* ms3, uint32_t* kernels, uint64_t* heap_high);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* CULI_H */

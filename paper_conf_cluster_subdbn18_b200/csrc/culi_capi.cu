@@ -1,0 +1,465 @@
+// culi_capi.cu — the C-ABI of libculi.so (include/culi.h): session state, device memory, uploads,
+// kernel launches and result copies.  No CPU fallback: every step of eval runs in the kernels of
+// culi_kernels.cu / culi_dispatch.cu.
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cstring>
+#include <memory>
+#include <new>
+#include <string>
+#include <vector>
+
+#include "../../include/culi.h"
+#include "culi_eval.cuh"
+#include "culi_host.h"
+#include "culi_ctx.h"
+
+
+
+using namespace culi;
+
+#define CK(x)                                   \
+  do {                                          \
+    cudaError_t _e = (x);                       \
+    if (_e != cudaSuccess) return CULI_E_CUDA;  \
+  } while (0)
+
+extern "C" {
+
+void culi_default_opts(culi_opts* o) {
+  if (!o) return;
+  std::memset(o, 0, sizeof *o);
+}
+
+const char* culi_status_string(int s) {
+  switch (s) {
+    case CULI_OK: return "ok";
+    case CULI_E_ARG: return "bad argument";
+    case CULI_E_PARSE: return "parse error";
+    case CULI_E_HEAP_FULL: return "device heap or stack exhausted";
+    case CULI_E_CUDA: return "CUDA error";
+    case CULI_E_NCCL: return "NCCL error";
+    case CULI_E_DEFINE: return "definition failed";
+    case CULI_E_STATE: return "invalid state";
+  }
+  return "unknown status";
+}
+
+const char* culi_error_name(uint8_t e) { return e < 10 ? kErrName[e] : "?"; }
+
+int culi_init(const culi_opts* opts, culi_ctx** out) {
+  if (!out) return CULI_E_ARG;
+  *out = nullptr;
+  culi_ctx* c = new (std::nothrow) culi_ctx;
+  if (!c) return CULI_E_ARG;
+  culi_default_opts(&c->opts);
+  if (opts) c->opts = *opts;
+  culi_opts& o = c->opts;
+  if (o.max_depth == 0) o.max_depth = 1024;
+  if (o.max_depth > 4095) { delete c; return CULI_E_ARG; }
+  if (o.fuel == 0) o.fuel = 1ull << 40;
+  if (o.heap_nodes == 0) o.heap_nodes = 64ull << 20;
+  if (o.heap_nodes > 0x7fffffffull) { delete c; return CULI_E_ARG; }
+  if (o.vstack_entries == 0) o.vstack_entries = 4096;
+  int ndev = 0;
+  if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev <= 0 || o.device >= ndev) {
+    delete c;
+    return CULI_E_CUDA;
+  }
+  if (cudaSetDevice(o.device) != cudaSuccess) { delete c; return CULI_E_CUDA; }
+  cudaDeviceGetAttribute(&c->sms, cudaDevAttrMultiProcessorCount, o.device);
+  if (o.slots == 0) o.slots = (uint32_t)c->sms * 512;
+  c->nslots = (o.slots + 127) / 128 * 128;
+  c->kcap = 2 * o.max_depth + 8;
+  c->vcap = o.vstack_entries;
+  c->stream = (cudaStream_t)o.stream;
+  bool ok = true;
+  ok &= cudaMalloc(&c->H.tag, o.heap_nodes) == cudaSuccess;
+  ok &= cudaMalloc(&c->H.word, o.heap_nodes * 8) == cudaSuccess;
+  ok &= cudaMalloc(&c->H.top, sizeof(unsigned long long)) == cudaSuccess;
+  ok &= cudaMalloc(&c->H.gtag, GCAP) == cudaSuccess;
+  ok &= cudaMalloc(&c->H.gword, (size_t)GCAP * 8) == cudaSuccess;
+  ok &= cudaMalloc((void**)&c->H.strs, c->str_cap) == cudaSuccess;
+  ok &= cudaMalloc(&c->kst, (size_t)c->nslots * c->kcap * sizeof(uint4)) == cudaSuccess;
+  ok &= cudaMalloc(&c->vst, (size_t)c->nslots * c->vcap * sizeof(uint4)) == cudaSuccess;
+  ok &= cudaMalloc(&c->next, sizeof(uint32_t)) == cudaSuccess;
+  ok &= cudaMalloc(&c->pcount, sizeof(unsigned long long)) == cudaSuccess;
+  ok &= cudaMalloc(&c->flags, 8 * sizeof(int)) == cudaSuccess;
+  for (int k = 0; k < 4 && ok; ++k) ok &= cudaEventCreate(&c->ev[k]) == cudaSuccess;
+  if (!ok) { culi_shutdown(c); return CULI_E_CUDA; }
+  c->H.cap = o.heap_nodes;
+  c->H.gcap = GCAP;
+  // nil and T nodes; every symbol unbound; builtins are resolved by id (reserved names)
+  uint8_t t01[2] = {K_NIL, K_T};
+  uint64_t w01[2] = {0, 0};
+  bool ok2 = cudaMemcpyAsync(c->H.tag, t01, 2, cudaMemcpyHostToDevice, c->stream) == cudaSuccess &&
+             cudaMemcpyAsync(c->H.word, w01, 16, cudaMemcpyHostToDevice, c->stream) == cudaSuccess &&
+             cudaMemsetAsync(c->H.gtag, K_UNBOUND, GCAP, c->stream) == cudaSuccess &&
+             cudaMemsetAsync(c->flags, 0, 8 * sizeof(int), c->stream) == cudaSuccess &&
+             cudaStreamSynchronize(c->stream) == cudaSuccess;
+  if (!ok2) { culi_shutdown(c); return CULI_E_CUDA; }
+  *out = c;
+  return CULI_OK;
+}
+
+void culi_shutdown(culi_ctx* c) {
+  if (!c) return;
+  if (c->stream || true) cudaStreamSynchronize(c->stream);
+  cudaFree(c->H.tag);
+  cudaFree(c->H.word);
+  cudaFree(c->H.top);
+  cudaFree(c->H.gtag);
+  cudaFree(c->H.gword);
+  cudaFree((void*)c->H.strs);
+  cudaFree(c->kst);
+  cudaFree(c->vst);
+  cudaFree(c->next);
+  cudaFree(c->pcount);
+  cudaFree(c->flags);
+  c->roots.release(); c->keys.release(); c->keys_alt.release(); c->perm.release();
+  c->perm_alt.release(); c->rtag.release(); c->rerr.release(); c->dtemp.release();
+  c->rsteps.release(); c->rword.release(); c->payload.release();
+  for (auto& e : c->ev) if (e) cudaEventDestroy(e);
+  delete c;
+}
+
+int culi_read(culi_ctx* c, const char* text, size_t len, culi_image** out, size_t* err_offset) {
+  if (!c || !out || (!text && len)) return CULI_E_ARG;
+  *out = nullptr;
+  culi_image* im = new (std::nothrow) culi_image;
+  if (!im) return CULI_E_ARG;
+  int rc = read_image(*c->syms, text, len, im->img, err_offset);
+  if (rc != CULI_OK) { delete im; return rc; }
+  *out = im;
+  return CULI_OK;
+}
+
+uint32_t culi_image_nforms(const culi_image* im) { return im ? (uint32_t)im->img.roots.size() : 0; }
+uint64_t culi_image_nnodes(const culi_image* im) { return im ? im->img.tag.size() : 0; }
+void culi_image_free(culi_image* im) { delete im; }
+
+}  // extern "C"
+
+// ---- internal helpers ------------------------------------------------------------------------------
+static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, int define_mode) {
+  EvalArgs A{};
+  A.H = c->H;
+  A.kst = c->kst;
+  A.vst = c->vst;
+  A.nslots = c->nslots;
+  A.kcap = c->kcap;
+  A.vcap = c->vcap;
+  A.roots = c->roots.p;
+  A.perm = perm;
+  A.nforms = nforms;
+  A.next = c->next;
+  A.rtag = c->rtag.p;
+  A.rerr = c->rerr.p;
+  A.rsteps = c->rsteps.p;
+  A.rword = c->rword.p;
+  A.max_depth = c->opts.max_depth;
+  A.fuel = c->opts.fuel;
+  A.define_mode = define_mode;
+  A.flags = c->flags;
+  A.voting = (c->opts.flags & CULI_F_NO_VOTING) ? 0 : 1;
+  return A;
+}
+
+// H2D of an image into the heap at c->mark (strings after the persistent strings) + relocation.
+static int upload_image(culi_ctx* c, const Image& img, uint32_t str_base) {
+  uint64_t n = img.tag.size();
+  if (c->mark + n > c->H.cap) return CULI_E_HEAP_FULL;
+  if (img.max_sym > c->H.gcap || c->syms->names.size() > c->H.gcap) return CULI_E_HEAP_FULL;
+  if ((uint64_t)str_base + img.strings.size() > c->str_cap) return CULI_E_HEAP_FULL;
+  uint32_t nr = (uint32_t)img.roots.size();
+  CK(c->roots.ensure(std::max<uint32_t>(nr, 1)));
+  if (n) {
+    CK(cudaMemcpyAsync(c->H.tag + c->mark, img.tag.data(), n, cudaMemcpyHostToDevice, c->stream));
+    CK(cudaMemcpyAsync(c->H.word + c->mark, img.word.data(), n * 8, cudaMemcpyHostToDevice, c->stream));
+  }
+  if (!img.strings.empty())
+    CK(cudaMemcpyAsync((char*)c->H.strs + str_base, img.strings.data(), img.strings.size(),
+                       cudaMemcpyHostToDevice, c->stream));
+  if (nr) CK(cudaMemcpyAsync(c->roots.p, img.roots.data(), nr * 4, cudaMemcpyHostToDevice, c->stream));
+  CK(launch_relocate(c->stream, c->H.tag, c->H.word, c->mark, n, str_base, c->roots.p, nr, c->sms));
+  return CULI_OK;
+}
+
+static int ensure_results(culi_ctx* c, uint32_t nforms) {
+  size_t n = std::max<uint32_t>(nforms, 1);
+  CK(c->rtag.ensure(n));
+  CK(c->rerr.ensure(n));
+  CK(c->rsteps.ensure(n));
+  CK(c->rword.ensure(n));
+  return CULI_OK;
+}
+
+extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed_index,
+                           uint8_t* failed_err) {
+  if (!c || !defs) return CULI_E_ARG;
+  const Image& img = defs->img;
+  uint32_t nf = (uint32_t)img.roots.size();
+  uint32_t str_base = (uint32_t)c->strings.size();
+  int rc = upload_image(c, img, str_base);
+  if (rc) return rc;
+  c->strings += img.strings;
+  rc = ensure_results(c, nf);
+  if (rc) return rc;
+  CK(launch_reset(c->stream, c->H.top, c->mark + img.tag.size(), c->next, c->pcount, c->flags));
+  EvalArgs A = make_args(c, nf, nullptr, 1);
+  if (nf) CK(launch_define(c->stream, A));
+  int flags[8];
+  unsigned long long top = 0;
+  CK(cudaMemcpyAsync(flags, c->flags, sizeof flags, cudaMemcpyDeviceToHost, c->stream));
+  CK(cudaMemcpyAsync(&top, c->H.top, 8, cudaMemcpyDeviceToHost, c->stream));
+  CK(cudaStreamSynchronize(c->stream));
+  c->mark = std::min<unsigned long long>(top, c->H.cap);
+  c->heap_high = std::max<uint64_t>(c->heap_high, top);
+  c->defined = true;
+  if (flags[0] && !flags[1]) return CULI_E_HEAP_FULL;
+  if (flags[1]) {
+    if (failed_index) *failed_index = (uint32_t)(flags[1] - 1);
+    if (failed_err) *failed_err = (uint8_t)flags[2];
+    if (flags[2] == E_OOM) return CULI_E_HEAP_FULL;
+    return CULI_E_DEFINE;
+  }
+  return CULI_OK;
+}
+
+// Run dispatch + eval + export for the uploaded batch (device only, stream-ordered, no host sync).
+static int run_batch_device(culi_ctx* c) {
+  uint32_t nf = c->batch_forms;
+  c->last_kernels = 0;
+  CK(cudaEventRecord(c->ev[0], c->stream));
+  CK(launch_reset(c->stream, c->H.top, c->mark + c->batch_nodes, c->next, c->pcount, c->flags));
+  ++c->last_kernels;
+  uint32_t* perm = nullptr;
+  if (!(c->opts.flags & CULI_F_NO_BINNING) && nf > 1) {
+    CK(launch_dispatch(c->stream, c->H, c->roots.p, nf, c->keys.p, c->keys_alt.p, c->perm.p,
+                       c->perm_alt.p, c->dtemp.p, c->dtemp.n, &perm, c->sms));
+    c->last_kernels += 3;
+  }
+  CK(cudaEventRecord(c->ev[1], c->stream));
+  EvalArgs A = make_args(c, nf, perm, 0);
+  uint32_t blocks = c->nslots / 128;
+  uint32_t need = (nf + 127) / 128;
+  if (need < blocks) blocks = std::max<uint32_t>(need, 1);
+  if (nf) { CK(launch_eval(c->stream, A, blocks)); ++c->last_kernels; }
+  CK(cudaEventRecord(c->ev[2], c->stream));
+  ExportArgs X{};
+  X.tag = c->H.tag;
+  X.word = c->H.word;
+  X.rtag = c->rtag.p;
+  X.rword = c->rword.p;
+  X.nforms = nf;
+  X.vst = c->vst;
+  X.nslots = c->nslots;
+  X.vcap = c->vcap;
+  X.payload = c->payload.p;
+  X.pcount = c->pcount;
+  X.pcap = c->payload.n;
+  X.flags = c->flags;
+  if (nf) { CK(launch_export(c->stream, X, blocks)); ++c->last_kernels; }
+  CK(cudaEventRecord(c->ev[3], c->stream));
+  return CULI_OK;
+}
+
+static int prepare_batch(culi_ctx* c, const Image& img) {
+  uint32_t nf = (uint32_t)img.roots.size();
+  uint32_t str_base = (uint32_t)c->strings.size();
+  int rc = upload_image(c, img, str_base);
+  if (rc) return rc;
+  rc = ensure_results(c, nf);
+  if (rc) return rc;
+  size_t n = std::max<uint32_t>(nf, 1);
+  CK(c->keys.ensure(n));
+  CK(c->keys_alt.ensure(n));
+  CK(c->perm.ensure(n));
+  CK(c->perm_alt.ensure(n));
+  CK(c->dtemp.ensure(dispatch_temp_bytes(nf)));
+  CK(c->payload.ensure(std::max<size_t>(4 * (size_t)nf, 1 << 16)));
+  c->have_batch = true;
+  c->batch_nodes = img.tag.size();
+  c->batch_forms = nf;
+  c->batch_strings = img.strings;
+  return CULI_OK;
+}
+
+static int fetch(culi_ctx* c, culi_results** out) {
+  uint32_t nf = c->batch_forms;
+  for (int attempt = 0; attempt < 3; ++attempt) {
+    int flags[8];
+    unsigned long long pc = 0, top = 0;
+    CK(cudaMemcpyAsync(flags, c->flags, sizeof flags, cudaMemcpyDeviceToHost, c->stream));
+    CK(cudaMemcpyAsync(&pc, c->pcount, 8, cudaMemcpyDeviceToHost, c->stream));
+    CK(cudaMemcpyAsync(&top, c->H.top, 8, cudaMemcpyDeviceToHost, c->stream));
+    CK(cudaStreamSynchronize(c->stream));
+    c->heap_high = std::max<uint64_t>(c->heap_high, std::min<unsigned long long>(top, c->H.cap));
+    if (flags[0] || flags[4]) return CULI_E_HEAP_FULL;
+    if (flags[3]) {                                  // payload buffer too small: grow, re-export
+      CK(c->payload.ensure((size_t)pc + 1024));
+      int zero[8] = {0};
+      CK(cudaMemcpyAsync(c->flags, zero, sizeof zero, cudaMemcpyHostToDevice, c->stream));
+      CK(cudaMemsetAsync(c->pcount, 0, 8, c->stream));
+      // results' words were partially rewritten: export reads rword as node index only for records
+      // that were not yet exported, so re-run eval + export from scratch
+      int rc = run_batch_device(c);
+      if (rc) return rc;
+      continue;
+    }
+    culi_results* r = new (std::nothrow) culi_results;
+    if (!r) return CULI_E_ARG;
+    r->r.rec.resize(nf);
+    std::vector<uint8_t> t(nf), e(nf);
+    std::vector<uint64_t> s(nf), w(nf);
+    if (nf) {
+      CK(cudaMemcpyAsync(t.data(), c->rtag.p, nf, cudaMemcpyDeviceToHost, c->stream));
+      CK(cudaMemcpyAsync(e.data(), c->rerr.p, nf, cudaMemcpyDeviceToHost, c->stream));
+      CK(cudaMemcpyAsync(s.data(), c->rsteps.p, nf * 8, cudaMemcpyDeviceToHost, c->stream));
+      CK(cudaMemcpyAsync(w.data(), c->rword.p, nf * 8, cudaMemcpyDeviceToHost, c->stream));
+    }
+    std::vector<uint4> pay(pc);
+    if (pc) CK(cudaMemcpyAsync(pay.data(), c->payload.p, pc * sizeof(uint4), cudaMemcpyDeviceToHost, c->stream));
+    CK(cudaStreamSynchronize(c->stream));
+    for (uint32_t i = 0; i < nf; ++i) r->r.rec[i] = Record{t[i], e[i], s[i], w[i]};
+    r->r.payload.resize(pc);
+    for (size_t k = 0; k < pc; ++k)
+      r->r.payload[k] = Token{((uint64_t)pay[k].y << 32) | pay[k].x, pay[k].z, 0};
+    r->r.syms = c->syms;
+    r->r.strings = c->strings + c->batch_strings;
+    *out = r;
+    return CULI_OK;
+  }
+  return CULI_E_HEAP_FULL;
+}
+
+extern "C" {
+
+int culi_eval_batch(culi_ctx* c, const culi_image* forms, culi_results** out) {
+  if (!c || !forms || !out) return CULI_E_ARG;
+  *out = nullptr;
+  int rc = prepare_batch(c, forms->img);
+  if (rc) return rc;
+  rc = run_batch_device(c);
+  if (rc) return rc;
+  rc = fetch(c, out);
+  c->have_batch = false;
+  return rc;
+}
+
+int culi_upload(culi_ctx* c, const culi_image* forms, uint32_t* handle) {
+  if (!c || !forms) return CULI_E_ARG;
+  int rc = prepare_batch(c, forms->img);
+  if (rc) return rc;
+  CK(cudaStreamSynchronize(c->stream));
+  if (handle) *handle = 1;
+  return CULI_OK;
+}
+
+int culi_eval_uploaded(culi_ctx* c, uint32_t handle) {
+  if (!c || handle != 1 || !c->have_batch) return CULI_E_STATE;
+  return run_batch_device(c);
+}
+
+int culi_fetch_results(culi_ctx* c, uint32_t handle, culi_results** out) {
+  if (!c || !out || handle != 1 || !c->have_batch) return CULI_E_STATE;
+  *out = nullptr;
+  return fetch(c, out);
+}
+
+int culi_release(culi_ctx* c, uint32_t handle) {
+  if (!c || handle != 1) return CULI_E_STATE;
+  c->have_batch = false;
+  return CULI_OK;
+}
+
+int culi_records_device(culi_ctx* c, void* dev_buf, size_t cap, size_t* bytes) {
+  if (!c) return CULI_E_ARG;
+  size_t n = c->batch_forms;
+  size_t o_steps = (2 * n + 7) & ~(size_t)7;
+  size_t total = o_steps + 16 * n;
+  if (bytes) *bytes = total;
+  if (!dev_buf) return CULI_OK;
+  if (cap < total || !c->have_batch) return CULI_E_ARG;
+  char* d = (char*)dev_buf;
+  if (n) {
+    CK(cudaMemcpyAsync(d, c->rtag.p, n, cudaMemcpyDeviceToDevice, c->stream));
+    CK(cudaMemcpyAsync(d + n, c->rerr.p, n, cudaMemcpyDeviceToDevice, c->stream));
+    CK(cudaMemcpyAsync(d + o_steps, c->rsteps.p, 8 * n, cudaMemcpyDeviceToDevice, c->stream));
+    CK(cudaMemcpyAsync(d + o_steps + 8 * n, c->rword.p, 8 * n, cudaMemcpyDeviceToDevice, c->stream));
+  }
+  return CULI_OK;
+}
+
+uint32_t culi_results_count(const culi_results* r) { return r ? (uint32_t)r->r.rec.size() : 0; }
+
+int culi_result_info(const culi_results* r, uint32_t i, uint8_t* tag, uint8_t* err, uint64_t* steps) {
+  if (!r || i >= r->r.rec.size()) return CULI_E_ARG;
+  const Record& x = r->r.rec[i];
+  if (tag) *tag = x.tag;
+  if (err) *err = x.err;
+  if (steps) *steps = x.steps;
+  return CULI_OK;
+}
+
+int culi_result_int(const culi_results* r, uint32_t i, int64_t* v) {
+  if (!r || i >= r->r.rec.size() || !v) return CULI_E_ARG;
+  const Record& x = r->r.rec[i];
+  if (x.err || x.tag != K_INT) return CULI_E_ARG;
+  *v = (int64_t)x.word;
+  return CULI_OK;
+}
+
+int culi_result_float(const culi_results* r, uint32_t i, double* v) {
+  if (!r || i >= r->r.rec.size() || !v) return CULI_E_ARG;
+  const Record& x = r->r.rec[i];
+  if (x.err || x.tag != K_FLOAT) return CULI_E_ARG;
+  std::memcpy(v, &x.word, 8);
+  return CULI_OK;
+}
+
+int culi_print(const culi_results* r, uint32_t i, char* buf, size_t cap, size_t* needed) {
+  if (!r || i >= r->r.rec.size()) return CULI_E_ARG;
+  std::string s;
+  r->r.print(i, s);
+  if (needed) *needed = s.size();
+  if (!buf || cap <= s.size()) {
+    if (buf && cap) {
+      std::memcpy(buf, s.data(), cap - 1);
+      buf[cap - 1] = 0;
+    }
+    return CULI_E_ARG;
+  }
+  std::memcpy(buf, s.data(), s.size());
+  buf[s.size()] = 0;
+  return CULI_OK;
+}
+
+int culi_results_totals(const culi_results* r, uint64_t* total_steps, uint32_t* n_errors) {
+  if (!r) return CULI_E_ARG;
+  uint64_t t = 0;
+  uint32_t ne = 0;
+  for (const Record& x : r->r.rec) {
+    t += x.steps;
+    ne += x.err != 0;
+  }
+  if (total_steps) *total_steps = t;
+  if (n_errors) *n_errors = ne;
+  return CULI_OK;
+}
+
+void culi_results_free(culi_results* r) { delete r; }
+
+int culi_last_timing(const culi_ctx* c, float* ms3, uint32_t* kernels, uint64_t* heap_high) {
+  if (!c) return CULI_E_ARG;
+  if (ms3) {
+    CK(cudaEventSynchronize(c->ev[3]));
+    for (int k = 0; k < 3; ++k) CK(cudaEventElapsedTime(&ms3[k], c->ev[k], c->ev[k + 1]));
+  }
+  if (kernels) *kernels = c->last_kernels;
+  if (heap_high) *heap_high = c->heap_high;
+  return CULI_OK;
+}
+
+}  // extern "C"

@@ -1,0 +1,87 @@
+// culi_ctx.h — session state of libculi.so (shared by culi_capi.cu and culi_dist.cu).
+#pragma once
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <memory>
+#include <string>
+#include <vector>
+
+#include "../../include/culi.h"
+#include "culi_eval.cuh"
+#include "culi_host.h"
+
+inline uint32_t lo32h(uint64_t w) { return (uint32_t)w; }
+
+using namespace culi;
+
+struct culi_image {
+  Image img;
+};
+
+struct culi_results {
+  Results r;
+};
+
+namespace culi_detail {
+
+template <typename T>
+struct DevBuf {
+  T* p = nullptr;
+  size_t n = 0;
+  cudaError_t ensure(size_t want) {
+    if (want <= n) return cudaSuccess;
+    if (p) cudaFree(p);
+    p = nullptr;
+    n = 0;
+    size_t grow = std::max(want, (size_t)1024);
+    cudaError_t e = cudaMalloc(&p, grow * sizeof(T));
+    if (e == cudaSuccess) n = grow;
+    return e;
+  }
+  void release() {
+    if (p) cudaFree(p);
+    p = nullptr;
+    n = 0;
+  }
+};
+
+constexpr uint32_t GCAP = 1u << 22;           // symbol ids supported (global table entries)
+constexpr uint64_t STR_CAP = 64ull << 20;      // string bytes
+
+}  // namespace culi_detail
+using namespace culi_detail;
+
+struct culi_ctx {
+  culi_opts opts;
+  cudaStream_t stream = nullptr;
+  int sms = 0;
+  std::shared_ptr<SymTable> syms = std::make_shared<SymTable>();
+  uint64_t str_cap = STR_CAP;
+  std::string strings;              // host mirror of the device string area (persistent part)
+  uint64_t mark = IMG_FIRST;        // first free heap node after the persistent (define) segment
+  bool defined = false;
+  // device memory
+  DevHeap H{};
+  uint4* kst = nullptr;
+  uint4* vst = nullptr;
+  uint32_t nslots = 0, kcap = 0, vcap = 0;
+  uint32_t* next = nullptr;         // work counter
+  unsigned long long* pcount = nullptr;
+  int* flags = nullptr;             // [0] oom [1] define fail idx+1 [2] define err [3] payload ovf [4] export ovf
+  DevBuf<uint32_t> roots, keys, keys_alt, perm, perm_alt;
+  DevBuf<uint8_t> rtag, rerr, dtemp;
+  DevBuf<uint64_t> rsteps, rword;
+  DevBuf<uint4> payload;
+  // uploaded batch (culi_upload)
+  bool have_batch = false;
+  uint64_t batch_nodes = 0;
+  uint32_t batch_forms = 0;
+  uint32_t* batch_perm = nullptr;
+  std::string batch_strings;
+  // timing
+  cudaEvent_t ev[4] = {nullptr, nullptr, nullptr, nullptr};
+  uint32_t last_kernels = 0;
+  uint64_t heap_high = 0;
+};
+

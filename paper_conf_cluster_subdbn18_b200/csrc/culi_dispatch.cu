@@ -1,0 +1,73 @@
+// culi_dispatch.cu — classify + bin the forms of a batch before evaluation.
+//
+// The paper notes that divergent branches of a warp are serialised (§III-D.d).  Forms are
+// independent, so their evaluation order is free: we give each form a 32-bit key
+//   (head class << 16) | (0xffff - cost hint)
+// where the head class is the form's head symbol (user functions first, then reserved builtins, then
+// atoms / data), and the cost hint is the first argument when it is an integer literal (e.g. n of
+// (fib n)), so forms whose control flow is identical land in the same warp, heaviest first.  A radix
+// sort (CUB, a plain library sort) of (key, form) gives the evaluation permutation; each warp of the
+// eval kernel then takes 32 consecutive forms of it.
+#include <cub/device/device_radix_sort.cuh>
+#include <cuda_runtime.h>
+
+#include "culi_eval.cuh"
+
+namespace culi {
+
+__global__ void culi_classify_kernel(const uint8_t* __restrict__ tag, const uint64_t* __restrict__ word,
+                                     const uint32_t* __restrict__ roots, uint32_t nforms,
+                                     uint32_t* __restrict__ keys, uint32_t* __restrict__ perm) {
+  uint32_t stride = gridDim.x * blockDim.x;
+  for (uint32_t f = blockIdx.x * blockDim.x + threadIdx.x; f < nforms; f += stride) {
+    uint32_t r = roots[f];
+    uint32_t cls = 0xffff, hint = 0;
+    if ((tag[r] & KIND_MASK) == K_CONS) {
+      uint64_t w = word[r];
+      uint32_t h = (uint32_t)w, rest = (uint32_t)(w >> 32);
+      if ((tag[h] & KIND_MASK) == K_SYM) {
+        uint32_t s = (uint32_t)word[h];
+        cls = s < N_RESERVED ? 0x8000u + s : (s < 0x7fffu ? s : 0x7fffu);
+      } else {
+        cls = 0xfffe;
+      }
+      if (rest != 0) {
+        uint32_t a = (uint32_t)word[rest];
+        uint32_t at = tag[a] & KIND_MASK;
+        if (at == K_INT) {
+          long long v = (long long)word[a];
+          hint = v < 0 ? 0 : (v > 0xffff ? 0xffff : (uint32_t)v);
+        } else if (at == K_CONS) {
+          uint32_t ah = (uint32_t)word[a];                // head symbol of a nested first argument
+          if ((tag[ah] & KIND_MASK) == K_SYM) hint = 0xff00u | ((uint32_t)word[ah] & 0xff);
+        }
+      }
+    }
+    keys[f] = (cls << 16) | (0xffffu - hint);
+    perm[f] = f;
+  }
+}
+
+size_t dispatch_temp_bytes(uint32_t nforms) {
+  size_t bytes = 0;
+  cub::DeviceRadixSort::SortPairs((void*)nullptr, bytes, (const uint32_t*)nullptr, (uint32_t*)nullptr,
+                                  (const uint32_t*)nullptr, (uint32_t*)nullptr, (int)nforms);
+  return bytes + 256;
+}
+
+cudaError_t launch_dispatch(cudaStream_t s, const DevHeap& H, const uint32_t* roots, uint32_t nforms,
+                            uint32_t* keys, uint32_t* keys_alt, uint32_t* perm, uint32_t* perm_alt,
+                            void* temp, size_t temp_bytes, uint32_t** perm_out, int sms) {
+  uint32_t blocks = (nforms + 255) / 256;
+  if (blocks > (uint32_t)sms * 8) blocks = sms * 8;
+  if (blocks == 0) blocks = 1;
+  culi_classify_kernel<<<blocks, 256, 0, s>>>(H.tag, H.word, roots, nforms, keys, perm);
+  cudaError_t e = cudaGetLastError();
+  if (e != cudaSuccess) return e;
+  size_t tb = temp_bytes;
+  e = cub::DeviceRadixSort::SortPairs(temp, tb, keys, keys_alt, perm, perm_alt, (int)nforms, 0, 32, s);
+  *perm_out = perm_alt;
+  return e;
+}
+
+}  // namespace culi

@@ -1,0 +1,96 @@
+// culi_eval.cuh — device side of libculi.so: SoA heap access, warp-aggregated bump allocator,
+// environment lookup, and the explicit-stack (non-recursive) eval/apply machine.  sm_100a only.
+//
+// The paper's evaluator is a recursive tree walk using CUDA device recursion (§III-B.c,
+// L172-175).  Here one thread runs one evaluation as a state machine over two per-thread stacks held in
+// HBM, interleaved across threads ("level-major": entry i of every thread is contiguous, so lanes that
+// run the same code at the same stack height coalesce):
+//   K-stack  (uint4 per entry) : continuation frames  {cursor, env, vsbase, depth|kind<<12|count<<16}
+//   V-stack  (uint4 per entry) : values and environment frames {w.lo, w.hi, sym, tag}
+// The machine replays the recursive definition of SURVEY §8(c).4 in the same order, so canonical step
+// counts, depths and first errors match the oracle exactly.  Tail positions (last body form, if
+// branches, macro expansions) do not keep a K-frame, but the canonical depth still increases.
+#pragma once
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+#include "culi_internal.h"
+
+namespace culi {
+
+constexpr uint32_t STACK_ENV = 0x80000000u;   // env reference into the thread's V-stack
+
+struct DevHeap {
+  uint8_t* tag;
+  uint64_t* word;
+  unsigned long long* top;     // bump pointer (node index)
+  uint64_t cap;                // node capacity
+  uint8_t* gtag;               // global frame: direct-indexed by symbol id (identity hash)
+  uint64_t* gword;
+  uint32_t gcap;
+  const char* strs;            // string bytes (offsets in STR words)
+};
+
+struct EvalArgs {
+  DevHeap H;
+  uint4* kst;                  // K-stack, level-major: kst[level * nslots + slot]
+  uint4* vst;                  // V-stack, level-major
+  uint32_t nslots;
+  uint32_t kcap;               // K-stack entries per slot
+  uint32_t vcap;               // V-stack entries per slot
+  const uint32_t* roots;       // heap index of each form's datum
+  const uint32_t* perm;        // optional evaluation order (binned dispatch), may be null
+  uint32_t nforms;
+  uint32_t* next;              // work counter (forms handed out so far)
+  uint8_t* rtag;               // results, indexed by form
+  uint8_t* rerr;
+  uint64_t* rsteps;
+  uint64_t* rword;
+  uint32_t max_depth;
+  uint64_t fuel;
+  int define_mode;
+  int* flags;                  // [0] heap/stack exhausted, [1] define: index of failing form + 1, [2] its err
+  uint32_t voting;             // warp opcode voting on/off
+  uint32_t staged_lo, staged_hi;  // node range staged in shared memory (0,0 = none)
+};
+
+struct ExportArgs {
+  const uint8_t* tag;
+  const uint64_t* word;
+  uint8_t* rtag;
+  uint64_t* rword;
+  uint32_t nforms;
+  uint4* vst;                  // DFS stack (the eval V-stack, reused)
+  uint32_t nslots, vcap;
+  uint4* payload;              // tokens {word.lo, word.hi, tag, 0}
+  unsigned long long* pcount;
+  unsigned long long pcap;
+  int* flags;                  // [3] payload overflow, [4] export stack overflow
+};
+
+// host-side launchers (culi_kernels.cu, culi_dispatch.cu)
+cudaError_t launch_relocate(cudaStream_t s, uint8_t* tag, uint64_t* word, uint64_t base, uint64_t n,
+                            uint32_t str_base, uint32_t* roots, uint32_t nroots, int sms);
+cudaError_t launch_eval(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
+cudaError_t launch_define(cudaStream_t s, const EvalArgs& A);
+cudaError_t launch_export(cudaStream_t s, const ExportArgs& X, uint32_t blocks);
+cudaError_t launch_reset(cudaStream_t s, unsigned long long* top, unsigned long long top_value,
+                         uint32_t* next, unsigned long long* pcount, int* flags);
+cudaError_t launch_dispatch(cudaStream_t s, const DevHeap& H, const uint32_t* roots, uint32_t nforms,
+                            uint32_t* keys, uint32_t* keys_alt, uint32_t* perm, uint32_t* perm_alt,
+                            void* temp, size_t temp_bytes, uint32_t** perm_out, int sms);
+size_t dispatch_temp_bytes(uint32_t nforms);
+
+struct V {
+  uint32_t t;
+  uint64_t w;
+};
+
+__device__ __forceinline__ uint32_t lo32(uint64_t w) { return (uint32_t)w; }
+__device__ __forceinline__ uint32_t hi32(uint64_t w) { return (uint32_t)(w >> 32); }
+__device__ __forceinline__ bool is_ref(uint32_t k) {
+  return k == K_CONS || k == K_STR || k == K_CLOSURE || k == K_MACRO;
+}
+__device__ __forceinline__ V mkv(uint32_t t, uint64_t w) { V v; v.t = t; v.w = w; return v; }
+
+}  // namespace culi

@@ -1,0 +1,261 @@
+// culi_host.cpp — host reader (text -> relocatable node image) and host printer of libculi.so.
+//
+// The paper reads on the device (§III-B.b) and names parsing the dominant GPU phase
+// (L785-788); north_star moves the read to the host ("host reads into a compact node array") so the
+// device runs only eval.  The reader is an iterative scanner (no recursion: inputs may nest deeply or
+// hold a 1M-element list) that allocates every list spine as consecutive cells (SURVEY c.14), so the
+// device's ||| fan-out can index list elements in O(1).
+#include <cerrno>
+#include <charconv>
+#include <cmath>
+#include <cstdlib>
+#include <cstring>
+
+#include "../../include/culi.h"
+#include "culi_host.h"
+
+namespace culi {
+
+const char* const kSpecialName[N_SPECIALS] = {"quote", "if", "define", "defun", "defmacro", "lambda",
+                                              "let", "progn"};
+const char* const kBuiltinName[N_BUILTINS] = {
+    "+", "-", "*", "/", "rem", "mod", "sqrt", "float", "trunc",
+    "=", "<", ">", "<=", ">=", "eq", "equal", "null", "not",
+    "atom", "consp", "numberp", "symbolp", "cons", "car", "cdr", "list",
+    "length", "append", "reverse", "nth", "|||"};
+const char* const kErrName[10] = {"NONE", "TYPE", "ARITY", "DIV0", "SYNTAX", "ARG", "DEPTH", "FUEL",
+                                  "DEFINE_IN_BATCH", "OOM"};
+
+SymTable::SymTable() {
+  for (uint32_t k = 0; k < N_SPECIALS; ++k) intern(kSpecialName[k], std::strlen(kSpecialName[k]));
+  for (uint32_t k = 0; k < N_BUILTINS; ++k) intern(kBuiltinName[k], std::strlen(kBuiltinName[k]));
+}
+
+uint32_t SymTable::intern(const char* s, size_t n) {
+  std::string key(s, n);
+  auto it = ids.find(key);
+  if (it != ids.end()) return it->second;
+  uint32_t id = (uint32_t)names.size();
+  names.push_back(key);
+  ids.emplace(std::move(key), id);
+  return id;
+}
+
+// ---- token classification (SURVEY c.1, c.13 #2) -------------------------------------------------------
+static inline bool is_space(char c) {
+  return c == ' ' || c == '\t' || c == '\n' || c == '\r' || c == '\f' || c == '\v';
+}
+static inline bool is_digit(char c) { return c >= '0' && c <= '9'; }
+
+// ^[+-]?[0-9]+$
+static bool classify_int(const char* s, size_t n) {
+  size_t i = (n > 0 && (s[0] == '+' || s[0] == '-')) ? 1 : 0;
+  if (i == n) return false;
+  for (; i < n; ++i)
+    if (!is_digit(s[i])) return false;
+  return true;
+}
+
+// ^[+-]?([0-9]+\.[0-9]*|\.[0-9]+)([eE][+-]?[0-9]+)?$ | ^[+-]?[0-9]+[eE][+-]?[0-9]+$
+static bool classify_float(const char* s, size_t n) {
+  size_t i = (n > 0 && (s[0] == '+' || s[0] == '-')) ? 1 : 0;
+  size_t int_digits = 0, frac_digits = 0;
+  bool dot = false;
+  while (i < n && is_digit(s[i])) { ++i; ++int_digits; }
+  if (i < n && s[i] == '.') {
+    dot = true;
+    ++i;
+    while (i < n && is_digit(s[i])) { ++i; ++frac_digits; }
+  }
+  if (int_digits + frac_digits == 0) return false;
+  bool expo = false;
+  if (i < n && (s[i] == 'e' || s[i] == 'E')) {
+    ++i;
+    if (i < n && (s[i] == '+' || s[i] == '-')) ++i;
+    size_t ed = 0;
+    while (i < n && is_digit(s[i])) { ++i; ++ed; }
+    if (ed == 0) return false;
+    expo = true;
+  }
+  if (i != n) return false;
+  return dot || expo;
+}
+
+namespace {
+struct Open {
+  bool quote;                  // a pending ' prefix (completes after one datum)
+  size_t offset;               // byte offset of '(' or '\''
+  std::vector<uint32_t> elems; // elements of an open list
+};
+
+struct Builder {
+  SymTable& st;
+  Image& img;
+  std::vector<uint32_t> sym_node;   // per-image dedupe: symbol id -> local node (0 = none yet)
+
+  uint32_t node(uint8_t tag, uint64_t word) {
+    uint32_t idx = IMG_FIRST + (uint32_t)img.tag.size();
+    img.tag.push_back(tag);
+    img.word.push_back(word);
+    return idx;
+  }
+  uint32_t symbol(uint32_t id) {
+    if (id >= sym_node.size()) sym_node.resize(id + 1, 0);
+    if (!sym_node[id]) sym_node[id] = node(K_SYM, id);
+    if (id + 1 > img.max_sym) img.max_sym = id + 1;
+    return sym_node[id];
+  }
+  // contiguous spine for a proper list (SURVEY c.14)
+  uint32_t spine(const std::vector<uint32_t>& xs) {
+    if (xs.empty()) return 0;
+    uint32_t first = IMG_FIRST + (uint32_t)img.tag.size();
+    uint32_t n = (uint32_t)xs.size();
+    for (uint32_t k = 0; k < n; ++k)
+      node(K_CONS | TAG_PROPER, pack2(xs[k], k + 1 < n ? first + k + 1 : 0));
+    return first;
+  }
+};
+}  // namespace
+
+int read_image(SymTable& st, const char* text, size_t len, Image& img, size_t* err_offset) {
+  Builder B{st, img, {}};
+  std::vector<Open> stack;
+  size_t p = 0;
+  auto fail = [&](size_t off) {
+    if (err_offset) *err_offset = off;
+    return (int)CULI_E_PARSE;
+  };
+  const uint32_t quote_id = SP_QUOTE;
+
+  // deliver a finished datum to the innermost open construct
+  auto deliver = [&](uint32_t d) {
+    for (;;) {
+      if (stack.empty()) { img.roots.push_back(d); return; }
+      Open& top = stack.back();
+      if (!top.quote) { top.elems.push_back(d); return; }
+      stack.pop_back();                              // 'x == (quote x)
+      std::vector<uint32_t> q{B.symbol(quote_id), d};
+      d = B.spine(q);
+    }
+  };
+
+  for (;;) {
+    while (p < len) {                                // whitespace and ; comments
+      if (is_space(text[p])) { ++p; continue; }
+      if (text[p] == ';') { while (p < len && text[p] != '\n') ++p; continue; }
+      break;
+    }
+    if (p >= len) break;
+    char c = text[p];
+    if (c == '(') {
+      stack.push_back(Open{false, p, {}});
+      ++p;
+    } else if (c == ')') {
+      if (stack.empty() || stack.back().quote) return fail(p);
+      std::vector<uint32_t> xs = std::move(stack.back().elems);
+      stack.pop_back();
+      ++p;
+      deliver(B.spine(xs));
+    } else if (c == '\'') {
+      stack.push_back(Open{true, p, {}});
+      ++p;
+    } else if (c == '"') {
+      const void* q = std::memchr(text + p + 1, '"', len - p - 1);
+      if (!q) return fail(p);
+      size_t e = (const char*)q - text;
+      uint64_t off = img.strings.size();
+      img.strings.append(text + p + 1, e - p - 1);
+      deliver(B.node(K_STR, pack2((uint32_t)off, (uint32_t)(e - p - 1))));
+      p = e + 1;
+    } else {
+      size_t s = p;
+      while (p < len && !is_space(text[p]) && text[p] != '(' && text[p] != ')') ++p;
+      const char* t = text + s;
+      size_t n = p - s;
+      uint32_t d;
+      if (n == 3 && std::memcmp(t, "nil", 3) == 0) {
+        d = 0;
+      } else if (n == 1 && t[0] == 'T') {
+        d = 1;
+      } else if (classify_int(t, n)) {
+        std::string tok(t, n);
+        errno = 0;
+        long long v = std::strtoll(tok.c_str(), nullptr, 10);
+        if (errno == ERANGE) return fail(s);
+        d = B.node(K_INT, (uint64_t)v);
+      } else if (classify_float(t, n)) {
+        std::string tok(t, n);
+        double v = std::strtod(tok.c_str(), nullptr);
+        uint64_t bits;
+        std::memcpy(&bits, &v, 8);
+        d = B.node(K_FLOAT, bits);
+      } else {
+        d = B.symbol(st.intern(t, n));
+      }
+      deliver(d);
+    }
+  }
+  if (!stack.empty()) return fail(stack.back().offset);
+  return CULI_OK;
+}
+
+// ---- printer (§III-B.d; SURVEY c.8) ------------------------------------------------------
+void print_float(double d, std::string& out) {
+  if (std::isnan(d)) { out += "nan"; return; }
+  if (std::isinf(d)) { out += d < 0 ? "-inf" : "inf"; return; }
+  char buf[64];
+  auto r = std::to_chars(buf, buf + sizeof buf, d);
+  bool has = false;
+  for (char* q = buf; q < r.ptr; ++q)
+    if (*q == '.' || *q == 'e') has = true;
+  out.append(buf, r.ptr);
+  if (!has) out += ".0";
+}
+
+static void print_atom(const Results& R, uint32_t tag, uint64_t w, std::string& out) {
+  switch (tag) {
+    case K_NIL: out += "nil"; break;
+    case K_T: out += "T"; break;
+    case K_INT: out += std::to_string((long long)(int64_t)w); break;
+    case K_FLOAT: { double d; std::memcpy(&d, &w, 8); print_float(d, out); break; }
+    case K_SYM: out += R.syms->names[(uint32_t)w]; break;
+    case K_STR:
+      out += '"';
+      out.append(R.strings, (uint32_t)w, (uint32_t)(w >> 32));
+      out += '"';
+      break;
+    case K_BUILTIN: out += "#<builtin "; out += kBuiltinName[w]; out += '>'; break;
+    case K_SPECIAL: out += "#<special "; out += kSpecialName[w]; out += '>'; break;
+    case K_CLOSURE: out += "#<lambda>"; break;
+    case K_MACRO: out += "#<macro>"; break;
+    default: out += "#<?>"; break;
+  }
+}
+
+void Results::print_token_range(size_t& pos, std::string& out) const {
+  const Token& t = payload[pos++];
+  if (t.tag != K_CONS) { print_atom(*this, t.tag, t.word, out); return; }
+  out += '(';
+  print_token_range(pos, out);                        // car
+  for (;;) {                                          // cdr chain iteratively
+    const Token& n = payload[pos];
+    if (n.tag == K_CONS) { ++pos; out += ' '; print_token_range(pos, out); continue; }
+    ++pos;
+    if (n.tag != K_NIL) { out += " . "; print_atom(*this, n.tag, n.word, out); }
+    break;
+  }
+  out += ')';
+}
+
+void Results::print(uint32_t i, std::string& out) const {
+  const Record& r = rec[i];
+  if (r.err) { out += "#<error "; out += kErrName[r.err < 10 ? r.err : 9]; out += '>'; return; }
+  if (r.tag == K_CONS || r.tag == K_STR) {
+    size_t pos = (uint32_t)r.word;
+    print_token_range(pos, out);
+    return;
+  }
+  print_atom(*this, r.tag, r.word, out);
+}
+
+}  // namespace culi
