@@ -62,6 +62,7 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   if (o.heap_nodes == 0) o.heap_nodes = 64ull << 20;
   if (o.heap_nodes > 0x7fffffffull) { delete c; return CULI_E_ARG; }
   if (o.vstack_entries == 0) o.vstack_entries = 4096;
+  if (o.vstack_entries > 65535) { delete c; return CULI_E_ARG; }
   int ndev = 0;
   if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev <= 0 || o.device >= ndev) {
     delete c;
@@ -163,6 +164,11 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.define_mode = define_mode;
   A.flags = c->flags;
   A.voting = (c->opts.flags & CULI_F_NO_VOTING) ? 0 : 1;
+  // stage the persistent code segment and the global frame in shared memory (batch mode only)
+  bool stage = !define_mode && !(c->opts.flags & CULI_F_NO_STAGING);
+  A.code_lo = IMG_FIRST;
+  A.code_n = stage ? (uint32_t)std::min<uint64_t>(c->mark - IMG_FIRST, 1536) : 0;
+  A.gst = stage ? (uint32_t)std::min<size_t>(c->syms->names.size(), 2048) : 0;
   return A;
 }
 

@@ -51,7 +51,8 @@ struct EvalArgs {
   int define_mode;
   int* flags;                  // [0] heap/stack exhausted, [1] define: index of failing form + 1, [2] its err
   uint32_t voting;             // warp opcode voting on/off
-  uint32_t staged_lo, staged_hi;  // node range staged in shared memory (0,0 = none)
+  uint32_t code_lo, code_n;    // node range staged in shared memory (persistent code segment)
+  uint32_t gst;                // global-frame entries staged in shared memory
 };
 
 struct ExportArgs {

@@ -110,9 +110,50 @@ struct Builder {
     if (xs.empty()) return 0;
     uint32_t first = IMG_FIRST + (uint32_t)img.tag.size();
     uint32_t n = (uint32_t)xs.size();
+    uint8_t valid = special_form_valid(xs) ? TAG_VALID : 0;
     for (uint32_t k = 0; k < n; ++k)
-      node(K_CONS | TAG_PROPER, pack2(xs[k], k + 1 < n ? first + k + 1 : 0));
+      node((uint8_t)(K_CONS | TAG_PROPER | (k == 0 ? valid : 0)), pack2(xs[k], k + 1 < n ? first + k + 1 : 0));
     return first;
+  }
+
+  // ---- syntax of special forms (SURVEY c.5), checked once at read time -----------------------------
+  uint32_t ltag(uint32_t L) const { return L < IMG_FIRST ? (L == 0 ? K_NIL : K_T) : img.tag[L - IMG_FIRST]; }
+  uint64_t lword(uint32_t L) const { return L < IMG_FIRST ? 0 : img.word[L - IMG_FIRST]; }
+  bool bindable(uint32_t L) const { return (ltag(L) & KIND_MASK) == K_SYM && lword(L) >= N_RESERVED; }
+  std::vector<uint32_t> elems(uint32_t L) const {           // reader lists are proper
+    std::vector<uint32_t> out;
+    while (L != 0) { uint64_t w = lword(L); out.push_back((uint32_t)w); L = (uint32_t)(w >> 32); }
+    return out;
+  }
+  bool is_list(uint32_t L) const { return L == 0 || (ltag(L) & KIND_MASK) == K_CONS; }
+  bool params_ok(uint32_t L) const {
+    if (!is_list(L)) return false;
+    for (uint32_t p : elems(L)) if (!bindable(p)) return false;
+    return true;
+  }
+  bool special_form_valid(const std::vector<uint32_t>& xs) const {
+    uint32_t h = xs[0];
+    if ((ltag(h) & KIND_MASK) != K_SYM || lword(h) >= N_SPECIALS) return false;
+    size_t n = xs.size() - 1;
+    switch (lword(h)) {
+      case SP_QUOTE: return n == 1;
+      case SP_IF: return n == 2 || n == 3;
+      case SP_PROGN: return true;
+      case SP_LAMBDA: return n >= 1 && params_ok(xs[1]);
+      case SP_DEFINE: return n == 2 && bindable(xs[1]);
+      case SP_DEFUN:
+      case SP_DEFMACRO: return n >= 2 && bindable(xs[1]) && params_ok(xs[2]);
+      case SP_LET: {
+        if (n < 1 || !is_list(xs[1])) return false;
+        for (uint32_t b : elems(xs[1])) {
+          if ((ltag(b) & KIND_MASK) != K_CONS) return false;
+          std::vector<uint32_t> se = elems(b);
+          if (se.size() != 2 || !bindable(se[0])) return false;
+        }
+        return true;
+      }
+    }
+    return false;
   }
 };
 }  // namespace

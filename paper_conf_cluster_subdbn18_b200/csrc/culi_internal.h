@@ -20,6 +20,11 @@ enum Kind : uint8_t {
   K_UNBOUND = 15
 };
 constexpr uint8_t TAG_PROPER = 0x10;
+// Set by the host reader on a list whose head is a special-form name (always the special form: the
+// names are reserved, c.5) and whose syntax it has already validated per c.5; the device skips the
+// checks for such lists.  Lists built at run time (macro expansions) never carry it.
+constexpr uint8_t TAG_VALID = 0x20;
+constexpr uint8_t K_AUX = 14;    // second node of a closure/macro: nparams | first param symbol << 32
 constexpr uint8_t KIND_MASK = 0x0f;
 
 enum ErrCode : uint8_t {

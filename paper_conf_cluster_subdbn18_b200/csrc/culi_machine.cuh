@@ -1,0 +1,1092 @@
+// culi_machine.cuh — the explicit-stack eval/apply machine (device code, sm_100a).
+//
+// Semantics: SURVEY.md §8(c).4-7 (§III-B.c eval, L383-413 environments, L546-589 |||),
+// replayed in exactly the recursive definition's order so that canonical step counts, depths and the
+// first error match the oracle.  Design:
+//   * control flow is a set of labels joined by gotos — no interpreter `switch` on a mode register;
+//   * atoms, symbols and reserved heads are evaluated inline where they occur, so only a nested *list*
+//     costs a continuation; ≤2-argument builtins whose arguments are all atoms/symbols are computed in
+//     registers without touching the V-stack (e.g. (- n 1), (< n 2));
+//   * K-stack (continuations, uint4) and V-stack (values / frame bindings, uint4) in HBM, level-major
+//     across threads so lock-step warps coalesce; the top continuation lives in registers with a dirty
+//     bit, so a continuation pushed and popped without an intervening push never touches memory;
+//   * environment references: heap frame node index, or STACK_ENV | n << 16 | vs_index for a frame on
+//     the thread's V-stack (n bindings), so a hit in the innermost frame costs one load;
+//   * the global frame (direct-indexed by symbol id) and the persistent code segment are staged in
+//     shared memory per block; special-form syntax of reader-produced lists is
+//     validated once on the host (TAG_VALID).
+#pragma once
+#include <cuda_runtime.h>
+#include <math.h>
+#include <stdint.h>
+
+#include "culi_eval.cuh"
+
+namespace culi {
+
+extern __shared__ __align__(16) uint4 culi_smem[];   // [code nodes][global words][global tags]
+
+struct Ctx {
+  const EvalArgs* A;         // the launch's constants (a __grid_constant__ kernel parameter)
+  uint4* kb;                 // &kst[slot]   (entry i at kb + i * nslots)
+  uint4* vb;                 // &vst[slot]
+};
+
+__device__ __forceinline__ uint4* KS(const Ctx& C, uint32_t i) { return C.kb + (size_t)i * C.A->nslots; }
+__device__ __forceinline__ uint4* VS(const Ctx& C, uint32_t i) { return C.vb + (size_t)i * C.A->nslots; }
+__device__ __forceinline__ uint4 vpack(V v, uint32_t sym) {
+  return make_uint4(lo32(v.w), hi32(v.w), sym, v.t);
+}
+__device__ __forceinline__ V vunpack(uint4 e) { return mkv(e.w, ((uint64_t)e.y << 32) | e.x); }
+__device__ __forceinline__ uint32_t kmeta(uint32_t depth, uint32_t kind, uint32_t count) {
+  return depth | (kind << 12) | (count << 16);
+}
+__device__ __forceinline__ uint32_t kdepth(uint32_t m) { return m & 0xfff; }
+__device__ __forceinline__ uint32_t kkind(uint32_t m) { return (m >> 12) & 0xf; }
+__device__ __forceinline__ uint32_t kcount(uint32_t m) { return m >> 16; }
+
+constexpr uint32_t ENV_IDX_MASK = 0xffffu;
+__device__ __forceinline__ uint32_t stack_env(uint32_t idx, uint32_t n) {
+  return STACK_ENV | (n << 16) | idx;
+}
+// reference kinds: STR, CONS, CLOSURE, MACRO (value word = node index)
+constexpr uint32_t REF_MASK = (1u << K_STR) | (1u << K_CONS) | (1u << K_CLOSURE) | (1u << K_MACRO);
+__device__ __forceinline__ bool is_ref_k(uint32_t k) { return (REF_MASK >> k) & 1u; }
+
+// ---- staged shared memory -----------------------------------------------------------------------------
+__device__ __forceinline__ const uint64_t* sm_gword(const Ctx& C) {
+  return reinterpret_cast<const uint64_t*>(culi_smem + C.A->code_n);
+}
+__device__ __forceinline__ const uint8_t* sm_gtag(const Ctx& C) {
+  return reinterpret_cast<const uint8_t*>(sm_gword(C) + C.A->gst);
+}
+
+// ---- heap access (SoA: tag u8[], word u64[]) with the staged code segment -----------
+__device__ __forceinline__ void ldnode(const Ctx& C, uint32_t n, uint32_t& t, uint64_t& w) {
+  uint32_t r = n - C.A->code_lo;
+  if (r < C.A->code_n) {
+    uint4 q = culi_smem[r];
+    t = q.z;
+    w = ((uint64_t)q.y << 32) | q.x;
+  } else {
+    t = C.A->H.tag[n];
+    w = C.A->H.word[n];
+  }
+}
+__device__ __forceinline__ uint64_t nword(const Ctx& C, uint32_t n) {
+  uint32_t r = n - C.A->code_lo;
+  if (r < C.A->code_n) { uint2 q = *reinterpret_cast<const uint2*>(&culi_smem[r]); return ((uint64_t)q.y << 32) | q.x; }
+  return C.A->H.word[n];
+}
+__device__ __forceinline__ uint32_t ntag(const Ctx& C, uint32_t n) {
+  uint32_t r = n - C.A->code_lo;
+  if (r < C.A->code_n) return culi_smem[r].z;
+  return C.A->H.tag[n];
+}
+__device__ __forceinline__ V unbox_loaded(uint32_t n, uint32_t t, uint64_t w) {
+  t &= KIND_MASK;
+  return mkv(t, is_ref_k(t) ? (uint64_t)n : w);
+}
+__device__ __forceinline__ V unbox(const Ctx& C, uint32_t n) {
+  uint32_t t;
+  uint64_t w;
+  ldnode(C, n, t, w);
+  return unbox_loaded(n, t, w);
+}
+__device__ __forceinline__ uint32_t car_of(const Ctx& C, uint32_t c) { return lo32(nword(C, c)); }
+__device__ __forceinline__ uint32_t cdr_of(const Ctx& C, uint32_t c) { return hi32(nword(C, c)); }
+
+// Warp-aggregated bump allocation (north_star; "the sequentially next free node"):
+// lanes asking for the same size in the same instruction share one atomicAdd (__match_any_sync) and
+// receive adjacent ranges, so their node stores coalesce.
+__device__ __forceinline__ bool heap_alloc(const DevHeap& H, uint32_t n, uint32_t* out) {
+  unsigned mask = __activemask();
+  unsigned peers = __match_any_sync(mask, n);
+  int lane = threadIdx.x & 31;
+  int leader = __ffs(peers) - 1;
+  unsigned rank = __popc(peers & ((1u << lane) - 1u));
+  unsigned long long base = 0;
+  if (lane == leader) base = atomicAdd(H.top, (unsigned long long)n * (unsigned)__popc(peers));
+  base = __shfl_sync(peers, base, leader);
+  unsigned long long mine = base + (unsigned long long)rank * n;
+  if (mine + n > H.cap) return false;
+  *out = (uint32_t)mine;
+  return true;
+}
+
+// store a value into a cons field: references are node indices; nil/T are nodes 0/1; immediates go to
+// the caller's preallocated box slot
+__device__ __forceinline__ uint32_t box_into(const DevHeap& H, V v, uint32_t slot_node) {
+  if (is_ref_k(v.t)) return (uint32_t)v.w;
+  if (v.t == K_NIL) return 0;
+  if (v.t == K_T) return 1;
+  H.tag[slot_node] = (uint8_t)v.t;
+  H.word[slot_node] = v.w;
+  return slot_node;
+}
+__device__ __forceinline__ bool proper_value(const Ctx& C, V v) {
+  return v.t == K_NIL || (v.t == K_CONS && (ntag(C, (uint32_t)v.w) & TAG_PROPER));
+}
+
+// ---- environments (§III-B.a; SURVEY c.3) ------------------------------------------------
+__device__ __forceinline__ V reserved_value(uint32_t sym) {
+  return sym < N_SPECIALS ? mkv(K_SPECIAL, sym) : mkv(K_BUILTIN, sym - N_SPECIALS);
+}
+__device__ __forceinline__ V global_value(const Ctx& C, uint32_t sym) {
+  uint32_t gt;
+  uint64_t gw;
+  if (sym < C.A->gst) {
+    gt = sm_gtag(C)[sym];
+    gw = sm_gword(C)[sym];
+  } else {
+    gt = C.A->H.gtag[sym];
+    gw = C.A->H.gword[sym];
+  }
+  if (gt == K_UNBOUND) return mkv(K_SYM, sym);
+  return mkv(gt, gw);
+}
+
+// full walk: innermost frame first, leftmost binding first, then the global frame; unbound -> itself
+__device__ __noinline__ V lookup_slow(const Ctx& C, uint32_t sym, uint32_t env) {
+  while (env != 0) {
+    if (env & STACK_ENV) {
+      uint32_t h = env & ENV_IDX_MASK, n = (env >> 16) & 0x7fffu;
+      for (uint32_t i = 1; i <= n; ++i) {
+        uint4 e = *VS(C, h + i);
+        if (e.z == sym) return vunpack(e);
+      }
+      env = VS(C, h)->x;
+    } else {
+      uint64_t hw = nword(C, env);
+      uint32_t n = hi32(hw);
+      for (uint32_t i = 1; i <= n; ++i) {
+        uint64_t bw = nword(C, env + i);
+        if (lo32(bw) == sym) return unbox(C, hi32(bw));
+      }
+      env = lo32(hw);
+    }
+  }
+  return global_value(C, sym);
+}
+
+// fast path: reserved names; the innermost stack frame's first binding; a one-binding stack frame
+// whose parent is the global frame (both loads issued together)
+__device__ __forceinline__ V lookup(const Ctx& C, uint32_t sym, uint32_t env) {
+  if (sym < N_RESERVED) return reserved_value(sym);
+  if (env == 0) return global_value(C, sym);
+  if (env & STACK_ENV) {
+    uint32_t h = env & ENV_IDX_MASK, n = (env >> 16) & 0x7fffu;
+    uint4 e = make_uint4(0, 0, 0xffffffffu, 0);
+    if (n >= 1) e = *VS(C, h + 1);
+    uint32_t parent = VS(C, h)->x;
+    if (n >= 1 && e.z == sym) return vunpack(e);
+    if (n <= 1 && parent == 0) return global_value(C, sym);
+  }
+  return lookup_slow(C, sym, env);
+}
+
+// Copy the stack frames a closure captures into the heap (frames are immutable, c.3, so a copy is
+// indistinguishable from the original).  Memoised in the stack header's .y field.
+__device__ __noinline__ bool promote(const Ctx& C, uint32_t env, uint32_t* out) {
+  const DevHeap& H = C.A->H;
+  if (!(env & STACK_ENV)) { *out = env; return true; }
+  for (;;) {
+    uint32_t topp = VS(C, env & ENV_IDX_MASK)->y;
+    if (topp) { *out = topp; return true; }
+    uint32_t e = env;
+    for (;;) {
+      uint32_t h = e & ENV_IDX_MASK;
+      uint4 hd = *VS(C, h);
+      uint32_t p = hd.x, ph = 0;
+      bool ready = true;
+      if (p & STACK_ENV) {
+        uint32_t pp = VS(C, p & ENV_IDX_MASK)->y;
+        if (pp) ph = pp; else ready = false;
+      } else {
+        ph = p;
+      }
+      if (ready) {
+        uint32_t n = hd.z, a;
+        if (!heap_alloc(H, 1 + 2 * n, &a)) return false;
+        H.tag[a] = K_FRAME;
+        H.word[a] = pack2(ph, n);
+        for (uint32_t i = 0; i < n; ++i) {
+          uint4 ent = *VS(C, h + 1 + i);
+          uint32_t vn = box_into(H, vunpack(ent), a + 1 + n + i);
+          H.tag[a + 1 + i] = K_BIND;
+          H.word[a + 1 + i] = pack2(ent.z, vn);
+        }
+        VS(C, h)->y = a;
+        break;
+      }
+      e = p;
+    }
+  }
+}
+
+// A closure / macro is two nodes: {kind: code | env << 32} and {K_AUX: nparams | first param << 32}
+// (code = the cons (params . body); env = heap frame or 0).
+__device__ __noinline__ bool make_closure(const Ctx& C, uint32_t kind, uint32_t code, uint32_t env,
+                                          V* out) {
+  uint32_t henv, a;
+  if (!promote(C, env, &henv)) return false;
+  uint32_t np = 0, first = 0;
+  for (uint32_t p = car_of(C, code); p != 0; p = cdr_of(C, p)) {
+    if (np == 0) first = (uint32_t)nword(C, car_of(C, p));
+    ++np;
+  }
+  if (!heap_alloc(C.A->H, 2, &a)) return false;
+  C.A->H.tag[a] = (uint8_t)kind;
+  C.A->H.word[a] = pack2(code, henv);
+  C.A->H.tag[a + 1] = K_AUX;
+  C.A->H.word[a + 1] = pack2(np, first);
+  *out = mkv(kind, a);
+  return true;
+}
+
+// c.5: a parameter list is a proper list of non-reserved symbols
+__device__ __noinline__ bool valid_params(const Ctx& C, uint32_t ps) {
+  if (ps == 0) return true;
+  uint32_t t = ntag(C, ps);
+  if ((t & KIND_MASK) != K_CONS || !(t & TAG_PROPER)) return false;
+  while (ps != 0) {
+    uint64_t w = nword(C, ps);
+    uint32_t at;
+    uint64_t aw;
+    ldnode(C, lo32(w), at, aw);
+    if ((at & KIND_MASK) != K_SYM || aw < N_RESERVED) return false;
+    ps = hi32(w);
+  }
+  return true;
+}
+__device__ __forceinline__ bool bindable_node(const Ctx& C, uint32_t n) {
+  uint32_t t;
+  uint64_t w;
+  ldnode(C, n, t, w);
+  return (t & KIND_MASK) == K_SYM && w >= N_RESERVED;
+}
+
+// ---- builtins (SURVEY c.6): arity, then types left to right, then compute --------------------------
+__device__ __forceinline__ bool is_num(uint32_t t) { return t == K_INT || t == K_FLOAT; }
+__device__ __forceinline__ double as_f64(V v) {
+  return v.t == K_INT ? __ll2double_rn((long long)v.w) : __longlong_as_double((long long)v.w);
+}
+__device__ __forceinline__ V mkf(double d) { return mkv(K_FLOAT, (uint64_t)__double_as_longlong(d)); }
+__device__ __forceinline__ V mkb(bool b) { return mkv(b ? K_T : K_NIL, 0); }
+__device__ __forceinline__ V arg(const Ctx& C, uint32_t base, uint32_t i) {
+  return vunpack(*VS(C, base + 1 + i));
+}
+__device__ __forceinline__ bool eq_values(V a, V b) {
+  if (a.t != b.t) return false;
+  if (a.t == K_NIL || a.t == K_T) return true;
+  return a.w == b.w;   // INT value, FLOAT bits, SYM id, op, or node identity for references
+}
+
+// one step of a numeric fold (types already checked); returns false on integer division by zero
+__device__ __noinline__ bool fold_float(uint32_t op, V& acc, V b) {
+  double x = as_f64(acc), y = as_f64(b), r;
+  switch (op) {
+    case BI_ADD: r = __dadd_rn(x, y); break;
+    case BI_SUB: r = __dsub_rn(x, y); break;
+    case BI_MUL: r = __dmul_rn(x, y); break;
+    default: r = __ddiv_rn(x, y); break;
+  }
+  acc = mkf(r);
+  return true;
+}
+__device__ __forceinline__ bool fold_step(uint32_t op, V& acc, V b) {
+  if (acc.t == K_INT && b.t == K_INT) {
+    switch (op) {
+      case BI_ADD: acc.w = acc.w + b.w; return true;
+      case BI_SUB: acc.w = acc.w - b.w; return true;
+      case BI_MUL: acc.w = acc.w * b.w; return true;
+      default: {
+        long long x = (long long)acc.w, y = (long long)b.w;
+        if (y == 0) return false;
+        acc.w = (y == -1) ? (0ull - acc.w) : (uint64_t)(x / y);   // INT64_MIN / -1 wraps
+        return true;
+      }
+    }
+  }
+  return fold_float(op, acc, b);
+}
+__device__ __forceinline__ bool cmp_values(uint32_t op, V a, V b) {
+  if (a.t == K_INT && b.t == K_INT) {
+    long long x = (long long)a.w, y = (long long)b.w;
+    return op == BI_NUMEQ ? x == y : op == BI_LT ? x < y : op == BI_GT ? x > y : op == BI_LE ? x <= y : x >= y;
+  }
+  double x = as_f64(a), y = as_f64(b);
+  return op == BI_NUMEQ ? x == y : op == BI_LT ? x < y : op == BI_GT ? x > y : op == BI_LE ? x <= y : x >= y;
+}
+
+// Builtins that the register fast path handles when they get at most two arguments.
+constexpr uint64_t FAST_OPS =
+    (1ull << BI_ADD) | (1ull << BI_SUB) | (1ull << BI_MUL) | (1ull << BI_DIV) | (1ull << BI_REM) |
+    (1ull << BI_MOD) | (1ull << BI_NUMEQ) | (1ull << BI_LT) | (1ull << BI_GT) | (1ull << BI_LE) |
+    (1ull << BI_GE) | (1ull << BI_EQ) | (1ull << BI_NULL) | (1ull << BI_NOT) | (1ull << BI_ATOM) |
+    (1ull << BI_CONSP) | (1ull << BI_NUMBERP) | (1ull << BI_SYMBOLP) | (1ull << BI_CAR) | (1ull << BI_CDR);
+
+// (op a0 [a1]) with argc <= 2 evaluated arguments in registers; same checks as the general path
+__device__ __forceinline__ uint8_t fast2(const Ctx& C, uint32_t op, uint32_t argc, V a0, V a1, V* out) {
+  switch (op) {
+    case BI_ADD: case BI_SUB: case BI_MUL: case BI_DIV: {
+      if (argc == 0) {
+        if (op == BI_SUB || op == BI_DIV) return E_ARITY;
+        *out = mkv(K_INT, op == BI_MUL ? 1 : 0);
+        return 0;
+      }
+      if (!is_num(a0.t) || (argc == 2 && !is_num(a1.t))) return E_TYPE;
+      if (argc == 1) {
+        if (op == BI_SUB) {
+          *out = a0.t == K_INT ? mkv(K_INT, 0ull - a0.w) : mkf(-__longlong_as_double((long long)a0.w));
+          return 0;
+        }
+        if (op != BI_DIV) { *out = a0; return 0; }
+        a1 = a0;                                     // (/ a) = (/ 1 a)
+        a0 = mkv(K_INT, 1);
+      }
+      if (!fold_step(op, a0, a1)) return E_DIV0;
+      *out = a0;
+      return 0;
+    }
+    case BI_REM: case BI_MOD: {
+      if (argc != 2) return E_ARITY;
+      if (a0.t != K_INT || a1.t != K_INT) return E_TYPE;
+      long long x = (long long)a0.w, y = (long long)a1.w;
+      if (y == 0) return E_DIV0;
+      long long r = (y == -1) ? 0 : x % y;
+      if (op == BI_MOD && r != 0 && ((r < 0) != (y < 0))) r += y;
+      *out = mkv(K_INT, (uint64_t)r);
+      return 0;
+    }
+    case BI_NUMEQ: case BI_LT: case BI_GT: case BI_LE: case BI_GE:
+      if (argc != 2) return E_ARITY;
+      if (!is_num(a0.t) || !is_num(a1.t)) return E_TYPE;
+      *out = mkb(cmp_values(op, a0, a1));
+      return 0;
+    case BI_EQ:
+      if (argc != 2) return E_ARITY;
+      *out = mkb(eq_values(a0, a1));
+      return 0;
+    case BI_CAR: case BI_CDR: {
+      if (argc != 1) return E_ARITY;
+      if (a0.t == K_NIL) { *out = a0; return 0; }
+      if (a0.t != K_CONS) return E_TYPE;
+      uint64_t w = nword(C, (uint32_t)a0.w);
+      *out = unbox(C, op == BI_CAR ? lo32(w) : hi32(w));
+      return 0;
+    }
+    default: {                                       // one-argument predicates
+      if (argc != 1) return E_ARITY;
+      uint32_t t = a0.t;
+      bool r = op == BI_NULL || op == BI_NOT ? t == K_NIL
+             : op == BI_ATOM ? t != K_CONS
+             : op == BI_CONSP ? t == K_CONS
+             : op == BI_NUMBERP ? is_num(t)
+             : (t == K_SYM || t == K_NIL || t == K_T);
+      *out = mkb(r);
+      return 0;
+    }
+  }
+}
+
+// equal: recursive on cons cells, with the V-stack above vtop as the explicit work stack
+__device__ __noinline__ uint8_t equal_values(const Ctx& C, uint32_t vtop, V a, V b, bool* res) {
+  uint32_t sp = vtop;
+  for (;;) {
+    bool same;
+    if (a.t == K_CONS && b.t == K_CONS) {
+      uint64_t wa = nword(C, (uint32_t)a.w), wb = nword(C, (uint32_t)b.w);
+      if (sp + 1 >= C.A->vcap) return E_OOM;
+      *VS(C, sp) = make_uint4(hi32(wa), hi32(wb), 0, 0);
+      ++sp;
+      a = unbox(C, lo32(wa));
+      b = unbox(C, lo32(wb));
+      continue;
+    }
+    if (a.t == K_STR && b.t == K_STR) {
+      uint64_t wa = nword(C, (uint32_t)a.w), wb = nword(C, (uint32_t)b.w);
+      uint32_t la = hi32(wa), lb = hi32(wb);
+      same = la == lb;
+      for (uint32_t i = 0; same && i < la; ++i) same = C.A->H.strs[lo32(wa) + i] == C.A->H.strs[lo32(wb) + i];
+    } else {
+      same = eq_values(a, b);
+    }
+    if (!same) { *res = false; return 0; }
+    if (sp == vtop) { *res = true; return 0; }
+    --sp;
+    uint4 pr = *VS(C, sp);
+    a = unbox(C, pr.x);
+    b = unbox(C, pr.y);
+  }
+}
+
+// general builtin application over vs[base+1 .. base+cnt] (any arity)
+__device__ __noinline__ uint8_t apply_builtin(const Ctx& C, uint32_t op, uint32_t base, uint32_t cnt,
+                                              uint32_t vtop, V* out) {
+  const DevHeap& H = C.A->H;
+  if (((FAST_OPS >> op) & 1) && cnt <= 2) {
+    V a0 = cnt > 0 ? arg(C, base, 0) : mkv(K_NIL, 0), a1 = cnt > 1 ? arg(C, base, 1) : mkv(K_NIL, 0);
+    return fast2(C, op, cnt, a0, a1, out);
+  }
+  switch (op) {
+    case BI_ADD: case BI_SUB: case BI_MUL: case BI_DIV: {       // cnt >= 3: left fold (c.13 #29)
+      bool type_err = false, div0 = false;
+      for (uint32_t i = 0; i < cnt; ++i) type_err |= !is_num(arg(C, base, i).t);
+      if (type_err) return E_TYPE;
+      V acc = arg(C, base, 0);
+      for (uint32_t i = 1; i < cnt && !div0; ++i) div0 = !fold_step(op, acc, arg(C, base, i));
+      if (div0) return E_DIV0;
+      *out = acc;
+      return 0;
+    }
+    case BI_REM: case BI_MOD: case BI_NUMEQ: case BI_LT: case BI_GT: case BI_LE: case BI_GE:
+    case BI_EQ: case BI_EQUAL: case BI_NULL: case BI_NOT: case BI_ATOM: case BI_CONSP:
+    case BI_NUMBERP: case BI_SYMBOLP: case BI_CAR: case BI_CDR: case BI_CONS: case BI_LENGTH:
+    case BI_REVERSE: case BI_NTH: case BI_SQRT: case BI_FLOAT: case BI_TRUNC: {
+      uint32_t need = (op == BI_REM || op == BI_MOD || op == BI_NUMEQ || op == BI_LT || op == BI_GT ||
+                       op == BI_LE || op == BI_GE || op == BI_EQ || op == BI_EQUAL || op == BI_CONS ||
+                       op == BI_NTH) ? 2 : 1;
+      if (cnt != need) return E_ARITY;
+      break;
+    }
+  }
+  switch (op) {
+    case BI_SQRT: case BI_FLOAT: case BI_TRUNC: {
+      V a = arg(C, base, 0);
+      if (!is_num(a.t)) return E_TYPE;
+      if (op == BI_SQRT) { *out = mkf(__dsqrt_rn(as_f64(a))); return 0; }
+      if (op == BI_FLOAT) { *out = mkf(as_f64(a)); return 0; }
+      if (a.t == K_INT) { *out = a; return 0; }
+      double x = __longlong_as_double((long long)a.w);
+      if (isnan(x) || fabs(x) >= 9223372036854775808.0) return E_ARG;
+      *out = mkv(K_INT, (uint64_t)__double2ll_rz(x));
+      return 0;
+    }
+    case BI_EQUAL: {
+      bool r;
+      uint8_t e = equal_values(C, vtop, arg(C, base, 0), arg(C, base, 1), &r);
+      if (e) return e;
+      *out = mkb(r);
+      return 0;
+    }
+    case BI_CONS: {
+      V a = arg(C, base, 0), b = arg(C, base, 1);
+      uint32_t c;
+      if (!heap_alloc(H, 3, &c)) return E_OOM;
+      uint32_t ca = box_into(H, a, c + 1), cd = box_into(H, b, c + 2);
+      H.tag[c] = (uint8_t)(K_CONS | (proper_value(C, b) ? TAG_PROPER : 0));
+      H.word[c] = pack2(ca, cd);
+      *out = mkv(K_CONS, c);
+      return 0;
+    }
+    case BI_LIST: {
+      if (cnt == 0) { *out = mkv(K_NIL, 0); return 0; }
+      uint32_t c;
+      if (!heap_alloc(H, 2 * cnt, &c)) return E_OOM;
+      for (uint32_t i = 0; i < cnt; ++i) {
+        uint32_t ca = box_into(H, arg(C, base, i), c + cnt + i);
+        H.tag[c + i] = K_CONS | TAG_PROPER;
+        H.word[c + i] = pack2(ca, i + 1 < cnt ? c + i + 1 : 0);
+      }
+      *out = mkv(K_CONS, c);
+      return 0;
+    }
+    case BI_LENGTH: {
+      V a = arg(C, base, 0);
+      if (!proper_value(C, a)) return E_TYPE;
+      uint64_t n = 0;
+      for (uint32_t c = a.t == K_NIL ? 0 : (uint32_t)a.w; c != 0; c = cdr_of(C, c)) ++n;
+      *out = mkv(K_INT, n);
+      return 0;
+    }
+    case BI_APPEND: {
+      if (cnt == 0) { *out = mkv(K_NIL, 0); return 0; }
+      uint32_t total = 0;
+      for (uint32_t i = 0; i + 1 < cnt; ++i) {
+        V a = arg(C, base, i);
+        if (!proper_value(C, a)) return E_TYPE;
+        for (uint32_t c = a.t == K_NIL ? 0 : (uint32_t)a.w; c != 0; c = cdr_of(C, c)) ++total;
+      }
+      V last = arg(C, base, cnt - 1);
+      if (total == 0) { *out = last; return 0; }
+      uint32_t c;
+      if (!heap_alloc(H, total + 1, &c)) return E_OOM;
+      uint32_t tail = box_into(H, last, c + total);
+      uint8_t tg = (uint8_t)(K_CONS | (proper_value(C, last) ? TAG_PROPER : 0));
+      uint32_t k = 0;
+      for (uint32_t i = 0; i + 1 < cnt; ++i) {
+        V a = arg(C, base, i);
+        for (uint32_t x = a.t == K_NIL ? 0 : (uint32_t)a.w; x != 0;) {
+          uint64_t w = nword(C, x);
+          H.tag[c + k] = tg;
+          H.word[c + k] = pack2(lo32(w), k + 1 < total ? c + k + 1 : tail);
+          ++k;
+          x = hi32(w);
+        }
+      }
+      *out = mkv(K_CONS, c);
+      return 0;
+    }
+    case BI_REVERSE: {
+      V a = arg(C, base, 0);
+      if (!proper_value(C, a)) return E_TYPE;
+      if (a.t == K_NIL) { *out = a; return 0; }
+      uint32_t n = 0;
+      for (uint32_t x = (uint32_t)a.w; x != 0; x = cdr_of(C, x)) ++n;
+      uint32_t c;
+      if (!heap_alloc(H, n, &c)) return E_OOM;
+      uint32_t k = 0;
+      for (uint32_t x = (uint32_t)a.w; x != 0; ++k) {
+        uint64_t w = nword(C, x);
+        uint32_t j = n - 1 - k;
+        H.tag[c + j] = K_CONS | TAG_PROPER;
+        H.word[c + j] = pack2(lo32(w), j + 1 < n ? c + j + 1 : 0);
+        x = hi32(w);
+      }
+      *out = mkv(K_CONS, c);
+      return 0;
+    }
+    case BI_NTH: {
+      V i = arg(C, base, 0), l = arg(C, base, 1);
+      if (i.t != K_INT || !proper_value(C, l)) return E_TYPE;
+      long long k = (long long)i.w;
+      if (k < 0) return E_ARG;
+      uint32_t x = l.t == K_NIL ? 0 : (uint32_t)l.w;
+      for (; k > 0 && x != 0; --k) x = cdr_of(C, x);
+      *out = x == 0 ? mkv(K_NIL, 0) : unbox(C, car_of(C, x));
+      return 0;
+    }
+    default: {                                       // fast ops with arity errors (cnt > 2)
+      V a0 = arg(C, base, 0), a1 = arg(C, base, 1);
+      return fast2(C, op, cnt > 2 ? 3 : cnt, a0, a1, out);
+    }
+  }
+}
+
+// (||| n f l1 .. lm) argument checks (c.7): arity, types left to right, then n >= 0 and every list
+// proper with >= n elements.  Returns 0 and fills n, or an error.
+__device__ __noinline__ uint8_t par_check(const Ctx& C, uint32_t base, uint32_t cnt, uint32_t* n_out) {
+  if (cnt < 3) return E_ARITY;
+  V nv = arg(C, base, 0), f = arg(C, base, 1);
+  if (nv.t != K_INT) return E_TYPE;
+  if (f.t != K_BUILTIN && f.t != K_CLOSURE) return E_TYPE;
+  long long n = (long long)nv.w;
+  if (n < 0) return E_ARG;
+  for (uint32_t j = 2; j < cnt; ++j) {
+    V l = arg(C, base, j);
+    if (!proper_value(C, l)) return E_ARG;
+    uint32_t c = l.t == K_NIL ? 0 : (uint32_t)l.w;
+    long long q = 0;
+    for (; q < n && c != 0; ++q) c = cdr_of(C, c);
+    if (q < n) return E_ARG;
+  }
+  if (n > 0x3fffffffll) return E_OOM;
+  *n_out = (uint32_t)n;
+  return 0;
+}
+
+// runtime syntax checks of special forms without TAG_VALID (c.5); cur = the argument list
+__device__ __noinline__ bool special_syntax_ok(const Ctx& C, uint32_t op, uint32_t cur) {
+  uint32_t n = 0;
+  for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
+  switch (op) {
+    case SP_QUOTE: return n == 1;
+    case SP_IF: return n == 2 || n == 3;
+    case SP_PROGN: return true;
+    case SP_LAMBDA: return n >= 1 && valid_params(C, car_of(C, cur));
+    case SP_DEFINE: return n == 2 && bindable_node(C, car_of(C, cur));
+    case SP_DEFUN: case SP_DEFMACRO:
+      return n >= 2 && bindable_node(C, car_of(C, cur)) && valid_params(C, car_of(C, cdr_of(C, cur)));
+    case SP_LET: {
+      if (n < 1) return false;
+      uint32_t bl = car_of(C, cur);
+      if (bl != 0) {
+        uint32_t bt = ntag(C, bl);
+        if ((bt & KIND_MASK) != K_CONS || !(bt & TAG_PROPER)) return false;
+        for (uint32_t c = bl; c != 0; c = cdr_of(C, c)) {
+          uint32_t b = car_of(C, c);
+          uint32_t tb = ntag(C, b);
+          if ((tb & KIND_MASK) != K_CONS || !(tb & TAG_PROPER)) return false;
+          uint64_t bw = nword(C, b);
+          if (!bindable_node(C, lo32(bw))) return false;
+          uint32_t r = hi32(bw);
+          if (r == 0 || cdr_of(C, r) != 0) return false;
+        }
+      }
+      return true;
+    }
+  }
+  return false;
+}
+
+// ---- the machine ---------------------------------------------------------------------------------------
+enum KKind : uint32_t { KF_HEAD = 1, KF_ARGS, KF_BODY, KF_IF, KF_LET, KF_DEFINE, KF_MACRO, KF_PAR, KF_DATA };
+
+struct FormOut {
+  uint32_t t;
+  uint64_t w;
+  uint64_t steps;
+  uint8_t err;
+};
+
+__device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root) {
+  const DevHeap& H = C.A->H;
+  const uint32_t kcap = C.A->kcap, vcap = C.A->vcap, maxd = C.A->max_depth;
+  const uint64_t fuel = C.A->fuel;
+  V v = mkv(K_NIL, 0), a0 = mkv(K_NIL, 0), a1 = mkv(K_NIL, 0);
+  uint32_t x = root, t = 0, env = 0, d = 1, cur = 0, base = 0, cnt = 0, sp = 0, vtop = 0;
+  uint32_t a = 0, at = 0, nxt = 0, kd = 0, hop = 0;
+  uint64_t w = 0, aw = 0, w0 = 0;
+  uint64_t steps = 0;
+  uint8_t err = 0;
+  uint4 k, ktop = make_uint4(0, 0, 0, 0);
+  bool kdirty = false;                      // ktop holds frame sp-1 not yet written to memory
+
+#define FAIL(e) do { err = (e); goto done; } while (0)
+#define STEP(depth)                                     \
+  do {                                                  \
+    ++steps;                                            \
+    if (steps > fuel || (depth) > maxd) {               \
+      err = steps > fuel ? E_FUEL : E_DEPTH;            \
+      goto done;                                        \
+    }                                                   \
+  } while (0)
+#define KPUSH(kind, cursor, envv, vsb, depth, count)                                  \
+  do {                                                                                \
+    if (sp >= kcap) FAIL(E_OOM);                                                      \
+    if (kdirty) *KS(C, sp - 1) = ktop;                                                \
+    ktop = make_uint4((cursor), (envv), (vsb), kmeta((depth), (kind), (count)));      \
+    kdirty = true;                                                                    \
+    ++sp;                                                                             \
+  } while (0)
+#define ATOMVAL(n, tt, ww) (((tt) & KIND_MASK) == K_SYM ? lookup(C, (uint32_t)(ww), env) : unbox_loaded((n), (tt), (ww)))
+
+  // ======================================================== EVAL a code node x in env at depth d
+EVAL_NODE:
+  ldnode(C, x, t, w);
+EVAL_NODE_LOADED:
+  STEP(d);                                                      // one canonical step (c.4 step 1)
+  if ((t & KIND_MASK) != K_CONS) { v = ATOMVAL(x, t, w); goto RET; }   // symbol / self-evaluating
+  // ======================================================== a list x (its step already counted)
+EVAL_CONS:
+  if (__builtin_expect(!(t & TAG_PROPER), 0)) FAIL(E_SYNTAX);
+  a = lo32(w);
+  cur = hi32(w);
+  ldnode(C, a, at, aw);
+  STEP(d + 1);                                                  // the head is always evaluated first
+  if ((at & KIND_MASK) != K_CONS) { v = ATOMVAL(a, at, aw); goto HEAD; }   // (L440-441)
+  KPUSH(KF_HEAD, cur, env, vtop, d, 0);
+  x = a; t = at; w = aw; d = d + 1;
+  goto EVAL_CONS;
+
+  // ======================================================== EVAL a value (a macro expansion)
+EVAL_VALUE:
+  STEP(d);
+  if (v.t == K_SYM) { v = lookup(C, (uint32_t)v.w, env); goto RET; }
+  if (v.t != K_CONS) goto RET;
+  x = (uint32_t)v.w;
+  ldnode(C, x, t, w);
+  goto EVAL_CONS;
+
+  // ======================================================== head value v, unevaluated args `cur`
+HEAD:
+  if (v.t == K_BUILTIN && ((FAST_OPS >> v.w) & 1)) {            // register fast path
+    hop = (uint32_t)v.w;
+    cnt = 0;
+    while (cur != 0) {
+      w0 = nword(C, cur);
+      a = lo32(w0);
+      nxt = hi32(w0);
+      ldnode(C, a, at, aw);
+      STEP(d + 1);
+      if ((at & KIND_MASK) == K_CONS || cnt == 2) {             // spill to the general path
+        if (vtop + 3 >= vcap) FAIL(E_OOM);
+        base = vtop;
+        *VS(C, base) = vpack(mkv(K_BUILTIN, hop), 0);
+        if (cnt > 0) *VS(C, base + 1) = vpack(a0, 0);
+        if (cnt > 1) *VS(C, base + 2) = vpack(a1, 0);
+        if ((at & KIND_MASK) == K_CONS) {
+          vtop = base + 1 + cnt;
+          KPUSH(KF_ARGS, nxt, env, base, d, cnt);
+          x = a; t = at; w = aw; d = d + 1;
+          goto EVAL_CONS;
+        }
+        *VS(C, base + 1 + cnt) = vpack(ATOMVAL(a, at, aw), 0);
+        ++cnt;
+        cur = nxt;
+        goto ARGS;
+      }
+      if (cnt == 0) a0 = ATOMVAL(a, at, aw); else a1 = ATOMVAL(a, at, aw);
+      ++cnt;
+      cur = nxt;
+    }
+    {
+      uint8_t e = fast2(C, hop, cnt, a0, a1, &v);
+      if (e) FAIL(e);
+    }
+    goto RET;
+  }
+  if (v.t == K_SPECIAL) {
+    uint32_t op = (uint32_t)v.w;
+    if (op == SP_DEFINE || op == SP_DEFUN || op == SP_DEFMACRO) {
+      if (!C.A->define_mode) FAIL(E_DEFINE_IN_BATCH);
+    }
+    if (!(t & TAG_VALID) && !special_syntax_ok(C, op, cur)) FAIL(E_SYNTAX);
+    switch (op) {
+      case SP_IF: {
+        w0 = nword(C, cur);
+        uint32_t c1 = hi32(w0);
+        a = lo32(w0);
+        ldnode(C, a, at, aw);
+        STEP(d + 1);
+        if ((at & KIND_MASK) == K_CONS) {
+          KPUSH(KF_IF, c1, env, vtop, d, 0);
+          x = a; t = at; w = aw; d = d + 1;
+          goto EVAL_CONS;
+        }
+        v = ATOMVAL(a, at, aw);
+        cur = c1;
+        goto IF_BRANCH;
+      }
+      case SP_QUOTE:
+        v = unbox(C, car_of(C, cur));
+        goto RET;
+      case SP_PROGN:
+        goto BODY;
+      case SP_LAMBDA:
+        if (!make_closure(C, K_CLOSURE, cur, env, &v)) FAIL(E_OOM);
+        goto RET;
+      case SP_LET: {
+        w0 = nword(C, cur);
+        uint32_t bl = lo32(w0), body = hi32(w0);
+        if (bl == 0) { cur = body; goto BODY; }
+        if (vtop >= vcap) FAIL(E_OOM);
+        base = vtop;
+        *VS(C, base) = make_uint4(body, 0, 0, K_FRAME);         // header (holds the body for now)
+        cnt = 0;
+        cur = bl;
+        goto LET_LOOP;
+      }
+      case SP_DEFINE: {
+        w0 = nword(C, cur);
+        KPUSH(KF_DEFINE, (uint32_t)nword(C, lo32(w0)), env, vtop, d, 0);
+        x = car_of(C, hi32(w0));
+        d = d + 1;
+        goto EVAL_NODE;
+      }
+      default: {                                                // defun / defmacro
+        w0 = nword(C, cur);
+        uint32_t s = (uint32_t)nword(C, lo32(w0));
+        V clo;
+        if (!make_closure(C, op == SP_DEFUN ? K_CLOSURE : K_MACRO, hi32(w0), env, &clo)) FAIL(E_OOM);
+        H.gtag[s] = (uint8_t)clo.t;
+        H.gword[s] = clo.w;
+        v = mkv(K_SYM, s);
+        goto RET;
+      }
+    }
+  }
+  if (__builtin_expect(v.t == K_MACRO, 0)) {                    // c.4 MACRO branch (c.13 #13)
+    uint64_t mw = nword(C, (uint32_t)v.w);
+    uint32_t menv = hi32(mw);
+    uint64_t cw = nword(C, lo32(mw));
+    uint32_t ps = lo32(cw), body = hi32(cw);
+    uint32_t hdr = vtop, n = 0;
+    a = cur;
+    while (ps != 0 && a != 0) {                                 // bind params to UNevaluated forms
+      uint64_t pw = nword(C, ps), aw2 = nword(C, a);
+      if (hdr + 1 + n >= vcap) FAIL(E_OOM);
+      *VS(C, hdr + 1 + n) = vpack(unbox(C, lo32(aw2)), (uint32_t)nword(C, lo32(pw)));
+      ++n;
+      ps = hi32(pw);
+      a = hi32(aw2);
+    }
+    if (ps != 0 || a != 0) FAIL(E_ARITY);
+    if (n >= 0x8000u) FAIL(E_OOM);
+    *VS(C, hdr) = make_uint4(menv, 0, n, K_FRAME);
+    KPUSH(KF_MACRO, 0, env, hdr, d, 0);
+    env = stack_env(hdr, n);
+    vtop = hdr + 1 + n;
+    cur = body;
+    goto BODY;
+  }
+  // data list (L443-444) or (list ...): elements stream into a preallocated contiguous spine (c.14)
+  if ((v.t != K_BUILTIN && v.t != K_CLOSURE) || (v.t == K_BUILTIN && v.w == BI_LIST)) {
+    bool data = v.t != K_BUILTIN;
+    uint32_t n = data ? 1 : 0;
+    for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
+    if (n == 0) { v = mkv(K_NIL, 0); goto RET; }
+    uint32_t s;
+    if (!heap_alloc(H, 2 * n, &s)) FAIL(E_OOM);
+    if (data) {
+      uint32_t ca = box_into(H, v, s + n);
+      H.tag[s] = K_CONS | TAG_PROPER;
+      H.word[s] = pack2(ca, n > 1 ? s + 1 : 0);
+    }
+    if (vtop >= vcap) FAIL(E_OOM);
+    base = vtop;
+    *VS(C, base) = make_uint4(s, n, 0, 0);                      // {spine, n}
+    cnt = data ? 1 : 0;                                         // next element index
+    goto DATA_LOOP;
+  }
+  // BUILTIN or CLOSURE: evaluate the args left to right at depth d+1 onto the V-stack
+  if (vtop >= vcap) FAIL(E_OOM);
+  base = vtop;
+  *VS(C, base) = vpack(v, 0);
+  cnt = 0;
+  // fallthrough
+ARGS:
+  while (cur != 0) {
+    w0 = nword(C, cur);
+    a = lo32(w0);
+    nxt = hi32(w0);
+    ldnode(C, a, at, aw);
+    STEP(d + 1);
+    if ((at & KIND_MASK) == K_CONS) {
+      vtop = base + 1 + cnt;
+      KPUSH(KF_ARGS, nxt, env, base, d, cnt);
+      x = a; t = at; w = aw; d = d + 1;
+      goto EVAL_CONS;
+    }
+    if (base + 1 + cnt >= vcap) FAIL(E_OOM);
+    *VS(C, base + 1 + cnt) = vpack(ATOMVAL(a, at, aw), 0);
+    ++cnt;
+    cur = nxt;
+  }
+  vtop = base + 1 + cnt;
+  // fallthrough
+APPLY: {                                                        // apply vs[base] to cnt args
+  V h = vunpack(*VS(C, base));
+  if (h.t == K_CLOSURE) {                                       // PAPER L456-460, c.4 CLOSURE
+    uint64_t cwd = nword(C, (uint32_t)h.w);
+    uint64_t aux = nword(C, (uint32_t)h.w + 1);
+    uint32_t np = lo32(aux);
+    if (np != cnt) FAIL(E_ARITY);
+    uint32_t code = lo32(cwd);
+    uint32_t body = cdr_of(C, code);
+    if (np == 1) {
+      VS(C, base + 1)->z = hi32(aux);
+    } else {
+      uint32_t ps = car_of(C, code);
+      for (uint32_t i = 0; i < cnt; ++i) {
+        uint64_t pw = nword(C, ps);
+        VS(C, base + 1 + i)->z = (uint32_t)nword(C, lo32(pw));
+        ps = hi32(pw);
+      }
+    }
+    if (cnt >= 0x8000u) FAIL(E_OOM);
+    *VS(C, base) = make_uint4(hi32(cwd), 0, cnt, K_FRAME);
+    env = stack_env(base, cnt);
+    vtop = base + 1 + cnt;
+    cur = body;
+    goto BODY;
+  }
+  if (h.t != K_BUILTIN) FAIL(E_SYNTAX);
+  if ((uint32_t)h.w == BI_PAR) {                                // (||| n f l1 ... lm), c.7
+    uint32_t n;
+    uint8_t e = par_check(C, base, cnt, &n);
+    if (e) FAIL(e);
+    if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
+    uint32_t m = cnt - 2, spine;
+    if (!heap_alloc(H, 2 * n, &spine)) FAIL(E_OOM);
+    // state: vs[base] = {spine, n}, vs[base+1] = f, vs[base+2+j] = list cursor j
+    V f = arg(C, base, 1);
+    for (uint32_t j = 0; j < m; ++j) *VS(C, base + 2 + j) = *VS(C, base + 3 + j);
+    *VS(C, base + 1) = vpack(f, 0);
+    *VS(C, base) = make_uint4(spine, n, 0, 0);
+    KPUSH(KF_PAR, 0, 0, base, d, m);
+    goto PAR_NEXT;
+  }
+  {
+    uint8_t e = apply_builtin(C, (uint32_t)h.w, base, cnt, vtop, &v);
+    if (e) FAIL(e);
+  }
+  vtop = base;
+  goto RET;
+}
+
+  // ======================================================== implicit progn of the forms `cur`
+BODY:
+  if (cur == 0) { v = mkv(K_NIL, 0); goto RET; }
+  for (;;) {
+    w0 = nword(C, cur);
+    a = lo32(w0);
+    nxt = hi32(w0);
+    ldnode(C, a, at, aw);
+    if (nxt == 0) { x = a; t = at; w = aw; d = d + 1; goto EVAL_NODE_LOADED; }   // tail position
+    STEP(d + 1);
+    if ((at & KIND_MASK) == K_CONS) {
+      KPUSH(KF_BODY, nxt, env, vtop, d, 0);
+      x = a; t = at; w = aw; d = d + 1;
+      goto EVAL_CONS;
+    }
+    cur = nxt;                                                  // an atom's value is discarded
+  }
+
+  // ======================================================== if: cond value v, `cur` = then cell
+IF_BRANCH:
+  w0 = nword(C, cur);
+  if (v.t != K_NIL) { x = lo32(w0); d = d + 1; goto EVAL_NODE; }   // only nil is false (L300-305)
+  if (hi32(w0) != 0) { x = car_of(C, hi32(w0)); d = d + 1; goto EVAL_NODE; }
+  v = mkv(K_NIL, 0);
+  goto RET;
+
+  // ======================================================== let: binding `cur` next (parallel let)
+LET_LOOP:
+  while (cur != 0) {
+    w0 = nword(C, cur);
+    uint64_t bw = nword(C, lo32(w0));
+    uint32_t e = car_of(C, hi32(bw));
+    ldnode(C, e, at, aw);
+    STEP(d + 1);
+    if ((at & KIND_MASK) == K_CONS) {
+      vtop = base + 1 + cnt;
+      KPUSH(KF_LET, cur, env, base, d, cnt);
+      x = e; t = at; w = aw; d = d + 1;
+      goto EVAL_CONS;
+    }
+    if (base + 1 + cnt >= vcap || cnt >= 0x7fffu) FAIL(E_OOM);
+    *VS(C, base + 1 + cnt) = vpack(ATOMVAL(e, at, aw), (uint32_t)nword(C, lo32(bw)));
+    ++cnt;
+    cur = hi32(w0);
+  }
+  cur = VS(C, base)->x;                                         // body list stored in the header
+  *VS(C, base) = make_uint4(env, 0, cnt, K_FRAME);
+  env = stack_env(base, cnt);
+  vtop = base + 1 + cnt;
+  goto BODY;
+
+  // ======================================================== data list / list: element `cnt` next
+DATA_LOOP: {
+  uint4 st = *VS(C, base);
+  uint32_t s = st.x, n = st.y;
+  while (cur != 0) {
+    w0 = nword(C, cur);
+    a = lo32(w0);
+    nxt = hi32(w0);
+    ldnode(C, a, at, aw);
+    STEP(d + 1);
+    if ((at & KIND_MASK) == K_CONS) {
+      VS(C, base)->z = cnt;
+      vtop = base + 1;
+      KPUSH(KF_DATA, nxt, env, base, d, 0);
+      x = a; t = at; w = aw; d = d + 1;
+      goto EVAL_CONS;
+    }
+    v = ATOMVAL(a, at, aw);
+    uint32_t ca = box_into(H, v, s + n + cnt);
+    H.tag[s + cnt] = K_CONS | TAG_PROPER;
+    H.word[s + cnt] = pack2(ca, cnt + 1 < n ? s + cnt + 1 : 0);
+    ++cnt;
+    cur = nxt;
+  }
+  vtop = base;
+  v = mkv(K_CONS, s);
+  goto RET;
+}
+
+  // ======================================================== ||| : start element i (frame in ktop)
+PAR_NEXT: {
+  uint32_t m = kcount(ktop.w), pb = ktop.z;
+  V f = vunpack(*VS(C, pb + 1));
+  base = pb + 2 + m;
+  if (base + 1 + m >= vcap) FAIL(E_OOM);
+  *VS(C, base) = vpack(f, 0);
+  for (uint32_t j = 0; j < m; ++j) {
+    uint4* cj = VS(C, pb + 2 + j);
+    uint64_t wj = nword(C, cj->x);
+    *VS(C, base + 1 + j) = vpack(unbox(C, lo32(wj)), 0);
+    cj->x = hi32(wj);
+  }
+  cnt = m;
+  vtop = base + 1 + m;
+  d = kdepth(ktop.w);
+  goto APPLY;
+}
+
+  // ======================================================== return v to the top continuation
+RET:
+  if (sp == 0) goto done;
+  k = ktop;
+  --sp;
+  if (sp > 0) ktop = *KS(C, sp - 1);                            // consumed at the next return
+  kdirty = false;
+  kd = kdepth(k.w);
+  switch (kkind(k.w)) {
+    case KF_ARGS:
+      base = k.z; cnt = kcount(k.w);
+      if (base + 1 + cnt >= vcap) FAIL(E_OOM);
+      *VS(C, base + 1 + cnt) = vpack(v, 0);
+      ++cnt;
+      cur = k.x; env = k.y; d = kd;
+      goto ARGS;
+    case KF_IF:
+      vtop = k.z; cur = k.x; env = k.y; d = kd;
+      goto IF_BRANCH;
+    case KF_BODY:
+      vtop = k.z; cur = k.x; env = k.y; d = kd;
+      goto BODY;
+    case KF_HEAD:
+      cur = k.x; env = k.y; vtop = k.z; d = kd;
+      t = 0;                                                    // a computed head: no TAG_VALID
+      goto HEAD;
+    case KF_LET: {
+      base = k.z; cnt = kcount(k.w);
+      w0 = nword(C, k.x);
+      uint32_t sym = (uint32_t)nword(C, car_of(C, lo32(w0)));
+      if (base + 1 + cnt >= vcap || cnt >= 0x7fffu) FAIL(E_OOM);
+      *VS(C, base + 1 + cnt) = vpack(v, sym);
+      ++cnt;
+      cur = hi32(w0); env = k.y; d = kd;
+      goto LET_LOOP;
+    }
+    case KF_DEFINE:
+      H.gtag[k.x] = (uint8_t)v.t;
+      H.gword[k.x] = v.w;
+      v = mkv(K_SYM, k.x);
+      vtop = k.z;
+      goto RET;
+    case KF_MACRO:                                              // evaluate the expansion
+      vtop = k.z; env = k.y; d = kd + 1;
+      goto EVAL_VALUE;
+    case KF_PAR: {                                              // element i finished
+      uint32_t m = kcount(k.w), i = k.x, pb = k.z;
+      uint4 st = *VS(C, pb);
+      uint32_t spine = st.x, n = st.y;
+      uint32_t ca = box_into(H, v, spine + n + i);
+      H.tag[spine + i] = K_CONS | TAG_PROPER;
+      H.word[spine + i] = pack2(ca, i + 1 < n ? spine + i + 1 : 0);
+      if (i + 1 == n) { v = mkv(K_CONS, spine); vtop = pb; goto RET; }
+      KPUSH(KF_PAR, i + 1, 0, pb, kd, m);
+      goto PAR_NEXT;
+    }
+    case KF_DATA: {
+      base = k.z;
+      uint4 st = *VS(C, base);
+      uint32_t s = st.x, n = st.y, i = st.z;
+      uint32_t ca = box_into(H, v, s + n + i);
+      H.tag[s + i] = K_CONS | TAG_PROPER;
+      H.word[s + i] = pack2(ca, i + 1 < n ? s + i + 1 : 0);
+      cnt = i + 1;
+      cur = k.x; env = k.y; d = kd;
+      goto DATA_LOOP;
+    }
+    default:
+      FAIL(E_SYNTAX);
+  }
+
+done:
+#undef FAIL
+#undef STEP
+#undef KPUSH
+#undef ATOMVAL
+  FormOut o;
+  o.t = v.t;
+  o.w = v.w;
+  o.steps = steps;
+  o.err = err;
+  return o;
+}
+
+}  // namespace culi

@@ -15,3 +15,8 @@ if [ -z "$SKIP_NCU" ]; then
   timeout 900 ncu --set full --clock-control none --import-source on -k regex:culi_eval_kernel -s 1 -c 1 -o $OUT/prof_$WL -f python bench.py --workload $WL --steps 1 --warmup 1 --e2e-steps 1 --no-cpu-baseline > $OUT/ncu_full.log 2>&1
   tail -3 $OUT/ncu_full.log
 fi
+if [ -f $OUT/prof_$WL.ncu-rep ]; then
+  python tools/ncu_summary.py full $OUT/prof_$WL.ncu-rep --json $OUT/eval_inst_$(echo $WL | tr A-Z a-z).json > $OUT/prof_${WL}_summary.txt 2>&1
+  python tools/ncu_summary.py launches $OUT/launches_$WL.csv > $OUT/launches_${WL}.md 2>&1
+  cat $OUT/eval_inst_$(echo $WL | tr A-Z a-z).json
+fi
