@@ -218,24 +218,14 @@ def culi_arm(args):
         if wl.defs:
             ctx.define(wl.defs)
     else:
-        size = torch.zeros(1, dtype=torch.int64, device=dev)
-        if rank == 0:
-            if wl.defs:
-                ctx.define(wl.defs)
-            size[0] = ctx.env_export_size()
-        dist.broadcast(size, 0)
-        buf = torch.empty(int(size.item()), dtype=torch.uint8, device=dev)
-        if rank == 0:
-            ctx.env_export(buf.data_ptr(), buf.numel())
+        from paper_conf_cluster_subdbn18_b200 import dist as D
+        if rank == 0 and wl.defs:
+            ctx.define(wl.defs)
         torch.cuda.synchronize()
-        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-        e0.record()
-        dist.broadcast(buf, 0)
-        e1.record()
+        t0 = time.perf_counter()
+        env_bytes = D.broadcast_env(ctx, src=0)
         torch.cuda.synchronize()
-        t_env = e0.elapsed_time(e1)
-        if rank != 0:
-            ctx.env_import(buf.data_ptr(), buf.numel())
+        t_env = {"ms": 1e3 * (time.perf_counter() - t0), "bytes": env_bytes}
 
     # ---- read (host, outside the timed region) + upload (a1, a2)
     t0 = time.perf_counter()
@@ -305,22 +295,10 @@ def culi_arm(args):
             dist.barrier()
         a.record(stream)
         r = ctx.eval_batch(img)
+        d2h = len(r.serialize())
         if world > 1:
-            blob = r.serialize()
-            t = torch.frombuffer(bytearray(blob), dtype=torch.uint8).to(dev)
-            sizes = [torch.zeros(1, dtype=torch.int64, device=dev) for _ in range(world)]
-            dist.all_gather(sizes, torch.tensor([t.numel()], dtype=torch.int64, device=dev))
-            mx = int(max(s.item() for s in sizes))
-            pad = torch.zeros(mx, dtype=torch.uint8, device=dev)
-            pad[: t.numel()] = t
-            outs = [torch.empty(mx, dtype=torch.uint8, device=dev) for _ in range(world)]
-            dist.all_gather(outs, pad)
-            if rank == 0:
-                blobs = [o[: int(s.item())].cpu().numpy().tobytes() for o, s in zip(outs, sizes)]
-                idx = [list(range(q, wl.nforms, world)) for q in range(world)]
-                culi.merge_results(blobs, idx)
-        else:
-            d2h = len(r.serialize())
+            from paper_conf_cluster_subdbn18_b200 import dist as D
+            D.gather_results(r, wl.nforms)
         b.record(stream)
         torch.cuda.synchronize()
         e2e_ms.append(a.elapsed_time(b))

@@ -87,6 +87,9 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   ok &= cudaMalloc(&c->next, sizeof(uint32_t)) == cudaSuccess;
   ok &= cudaMalloc(&c->pcount, sizeof(unsigned long long)) == cudaSuccess;
   ok &= cudaMalloc(&c->flags, 8 * sizeof(int)) == cudaSuccess;
+  ok &= cudaMalloc(&c->desc, (size_t)c->maxdesc * sizeof(FanDesc)) == cudaSuccess;
+  ok &= cudaMalloc(&c->npend, sizeof(uint32_t)) == cudaSuccess;
+  ok &= cudaMalloc(&c->nfallback, sizeof(uint32_t)) == cudaSuccess;
   for (int k = 0; k < 4 && ok; ++k) ok &= cudaEventCreate(&c->ev[k]) == cudaSuccess;
   if (!ok) { culi_shutdown(c); return CULI_E_CUDA; }
   c->H.cap = o.heap_nodes;
@@ -118,6 +121,10 @@ void culi_shutdown(culi_ctx* c) {
   cudaFree(c->next);
   cudaFree(c->pcount);
   cudaFree(c->flags);
+  cudaFree(c->desc);
+  cudaFree(c->npend);
+  cudaFree(c->nfallback);
+  c->fallback.release();
   c->roots.release(); c->keys.release(); c->keys_alt.release(); c->perm.release();
   c->perm_alt.release(); c->rtag.release(); c->rerr.release(); c->dtemp.release();
   c->rsteps.release(); c->rword.release(); c->payload.release();
@@ -164,6 +171,15 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.define_mode = define_mode;
   A.flags = c->flags;
   A.voting = (c->opts.flags & CULI_F_NO_VOTING) ? 0 : 1;
+  A.fanout = (!define_mode && !(c->opts.flags & CULI_F_NO_FANOUT)) ? 1 : 0;
+  A.desc = c->desc;
+  A.npend = c->npend;
+  A.maxdesc = c->maxdesc;
+  A.fallback = c->fallback.p;
+  A.nfallback = c->nfallback;
+  A.payload = c->payload.p;
+  A.pcount = c->pcount;
+  A.pcap = c->payload.n;
   // stage the persistent code segment and the global frame in shared memory (batch mode only)
   bool stage = !define_mode && !(c->opts.flags & CULI_F_NO_STAGING);
   A.code_lo = IMG_FIRST;
@@ -212,7 +228,8 @@ extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed
   c->strings += img.strings;
   rc = ensure_results(c, nf);
   if (rc) return rc;
-  CK(launch_reset(c->stream, c->H.top, c->mark + img.tag.size(), c->next, c->pcount, c->flags));
+  CK(launch_reset(c->stream, c->H.top, c->mark + img.tag.size(), c->next, c->pcount, c->flags, c->npend,
+                  c->nfallback));
   EvalArgs A = make_args(c, nf, nullptr, 1);
   if (nf) CK(launch_define(c->stream, A));
   int flags[8];
@@ -238,7 +255,8 @@ static int run_batch_device(culi_ctx* c) {
   uint32_t nf = c->batch_forms;
   c->last_kernels = 0;
   CK(cudaEventRecord(c->ev[0], c->stream));
-  CK(launch_reset(c->stream, c->H.top, c->mark + c->batch_nodes, c->next, c->pcount, c->flags));
+  CK(launch_reset(c->stream, c->H.top, c->mark + c->batch_nodes, c->next, c->pcount, c->flags, c->npend,
+                  c->nfallback));
   ++c->last_kernels;
   uint32_t* perm = nullptr;
   if (!(c->opts.flags & CULI_F_NO_BINNING) && nf > 1) {
@@ -252,6 +270,10 @@ static int run_batch_device(culi_ctx* c) {
   uint32_t need = (nf + 127) / 128;
   if (need < blocks) blocks = std::max<uint32_t>(need, 1);
   if (nf) { CK(launch_eval(c->stream, A, blocks)); ++c->last_kernels; }
+  if (nf && A.fanout && c->batch_has_par) {            // ||| fan-out (a6) + finalize (a8)
+    CK(launch_fanout(c->stream, A, c->nslots / 128));
+    c->last_kernels += 2;
+  }
   CK(cudaEventRecord(c->ev[2], c->stream));
   ExportArgs X{};
   X.tag = c->H.tag;
@@ -266,7 +288,13 @@ static int run_batch_device(culi_ctx* c) {
   X.pcount = c->pcount;
   X.pcap = c->payload.n;
   X.flags = c->flags;
+  X.list = nullptr;
+  X.nlist = 0;
   if (nf) { CK(launch_export(c->stream, X, blocks)); ++c->last_kernels; }
+  if (nf && A.fanout && c->batch_has_par) {
+    CK(launch_flat_export(c->stream, A, c->sms * 8));
+    c->last_kernels += 2;
+  }
   CK(cudaEventRecord(c->ev[3], c->stream));
   return CULI_OK;
 }
@@ -284,25 +312,71 @@ static int prepare_batch(culi_ctx* c, const Image& img) {
   CK(c->perm.ensure(n));
   CK(c->perm_alt.ensure(n));
   CK(c->dtemp.ensure(dispatch_temp_bytes(nf)));
-  CK(c->payload.ensure(std::max<size_t>(4 * (size_t)nf, 1 << 16)));
+  // tokens: ~4 per form; a ||| result list can be as long as the persistent segment (2 tokens per cell)
+  CK(c->payload.ensure(std::max<size_t>(4 * (size_t)nf + 2 * (size_t)(c->mark + img.tag.size()), 1 << 16)));
   c->have_batch = true;
   c->batch_nodes = img.tag.size();
   c->batch_forms = nf;
   c->batch_strings = img.strings;
+  CK(c->fallback.ensure(std::max<size_t>(c->maxdesc, 1)));
+  c->batch_has_par = false;                          // does any form start with the ||| symbol?
+  for (uint32_t r : img.roots) {
+    if (r < IMG_FIRST || (img.tag[r - IMG_FIRST] & KIND_MASK) != K_CONS) continue;
+    uint32_t h = (uint32_t)img.word[r - IMG_FIRST];
+    if (h >= IMG_FIRST && (img.tag[h - IMG_FIRST] & KIND_MASK) == K_SYM &&
+        img.word[h - IMG_FIRST] == N_SPECIALS + BI_PAR) {
+      c->batch_has_par = true;
+      break;
+    }
+  }
+  return CULI_OK;
+}
+
+// ||| forms the fan-out could not decide (an element error, fuel overflow, a short or non-contiguous
+// list) are re-evaluated exactly, one thread per form, without fan-out; then exported.
+static int rerun_fallback(culi_ctx* c, uint32_t nfb) {
+  CK(cudaMemsetAsync(c->next, 0, sizeof(uint32_t), c->stream));
+  EvalArgs A = make_args(c, nfb, c->fallback.p, 0);
+  A.fanout = 0;
+  CK(launch_eval(c->stream, A, std::max<uint32_t>(1, std::min<uint32_t>(c->nslots / 128, (nfb + 127) / 128))));
+  ExportArgs X{};
+  X.tag = c->H.tag;
+  X.word = c->H.word;
+  X.rtag = c->rtag.p;
+  X.rword = c->rword.p;
+  X.nforms = c->batch_forms;
+  X.vst = c->vst;
+  X.nslots = c->nslots;
+  X.vcap = c->vcap;
+  X.payload = c->payload.p;
+  X.pcount = c->pcount;
+  X.pcap = c->payload.n;
+  X.flags = c->flags;
+  X.list = c->fallback.p;
+  X.nlist = nfb;
+  CK(launch_export(c->stream, X, std::max<uint32_t>(1, (nfb + 127) / 128)));
+  CK(cudaMemsetAsync(c->nfallback, 0, sizeof(uint32_t), c->stream));
   return CULI_OK;
 }
 
 static int fetch(culi_ctx* c, culi_results** out) {
   uint32_t nf = c->batch_forms;
-  for (int attempt = 0; attempt < 3; ++attempt) {
+  for (int attempt = 0; attempt < 4; ++attempt) {
     int flags[8];
     unsigned long long pc = 0, top = 0;
+    uint32_t nfb = 0;
     CK(cudaMemcpyAsync(flags, c->flags, sizeof flags, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(&pc, c->pcount, 8, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(&top, c->H.top, 8, cudaMemcpyDeviceToHost, c->stream));
+    CK(cudaMemcpyAsync(&nfb, c->nfallback, 4, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaStreamSynchronize(c->stream));
     c->heap_high = std::max<uint64_t>(c->heap_high, std::min<unsigned long long>(top, c->H.cap));
     if (flags[0] || flags[4]) return CULI_E_HEAP_FULL;
+    if (nfb && !flags[3]) {
+      int rc = rerun_fallback(c, nfb);
+      if (rc) return rc;
+      continue;
+    }
     if (flags[3]) {                                  // payload buffer too small: grow, re-export
       CK(c->payload.ensure((size_t)pc + 1024));
       int zero[8] = {0};

@@ -73,6 +73,13 @@ struct culi_ctx {
   DevBuf<uint8_t> rtag, rerr, dtemp;
   DevBuf<uint64_t> rsteps, rword;
   DevBuf<uint4> payload;
+  // ||| fan-out state
+  FanDesc* desc = nullptr;
+  uint32_t maxdesc = 4096;
+  uint32_t* npend = nullptr;
+  uint32_t* nfallback = nullptr;
+  DevBuf<uint32_t> fallback;
+  bool batch_has_par = false;
   // uploaded batch (culi_upload)
   bool have_batch = false;
   uint64_t batch_nodes = 0;

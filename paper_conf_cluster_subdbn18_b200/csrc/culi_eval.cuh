@@ -51,9 +51,35 @@ struct EvalArgs {
   int define_mode;
   int* flags;                  // [0] heap/stack exhausted, [1] define: index of failing form + 1, [2] its err
   uint32_t voting;             // warp opcode voting on/off
+  uint32_t fanout;             // top-level ||| forms fan out over threads (batch eval kernel only)
+  struct FanDesc* desc;        // fan-out descriptors (device)
+  uint32_t* npend;             // number of descriptors written
+  uint32_t maxdesc;
+  uint32_t* fallback;          // forms to re-evaluate sequentially (fan-out could not decide them)
+  uint32_t* nfallback;
+  uint4* payload;              // export tokens (flat ||| results are written by the fan-out stage)
+  unsigned long long* pcount;
+  unsigned long long pcap;
   uint32_t code_lo, code_n;    // node range staged in shared memory (persistent code segment)
   uint32_t gst;                // global-frame entries staged in shared memory
 };
+
+// One top-level (||| n f l1 .. lm) form whose arguments have been evaluated.
+constexpr uint32_t FANOUT_MAXM = 6;
+constexpr uint8_t E_PENDING = 0xfe;          // internal: record filled in by the fan-out finalizer
+struct FanDesc {
+  uint32_t form, n, m, spine;                // spine: 2n nodes (n cells, then n box slots)
+  uint32_t ftag, depth;
+  uint64_t fword;
+  uint64_t steps0;                           // canonical steps before the first element
+  uint64_t top;                              // heap top when the descriptor was written
+  uint32_t heads[FANOUT_MAXM];               // first cell of each list
+  unsigned long long total;                  // sum of element steps (atomic)
+  uint32_t bad;                              // bit 0: non-contiguous list, bit 1: an element errored
+  uint32_t nonflat;                          // some element value is a cons (export walks it)
+  unsigned long long flat_off;               // payload offset of a flat result list
+};
+constexpr uint8_t K_FLATREC = 12;            // internal record tag: flat ||| result awaiting export
 
 struct ExportArgs {
   const uint8_t* tag;
@@ -67,6 +93,8 @@ struct ExportArgs {
   unsigned long long* pcount;
   unsigned long long pcap;
   int* flags;                  // [3] payload overflow, [4] export stack overflow
+  const uint32_t* list;        // optional: export only these forms
+  uint32_t nlist;
 };
 
 // host-side launchers (culi_kernels.cu, culi_dispatch.cu)
@@ -76,7 +104,10 @@ cudaError_t launch_eval(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
 cudaError_t launch_define(cudaStream_t s, const EvalArgs& A);
 cudaError_t launch_export(cudaStream_t s, const ExportArgs& X, uint32_t blocks);
 cudaError_t launch_reset(cudaStream_t s, unsigned long long* top, unsigned long long top_value,
-                         uint32_t* next, unsigned long long* pcount, int* flags);
+                         uint32_t* next, unsigned long long* pcount, int* flags, uint32_t* npend,
+                         uint32_t* nfallback);
+cudaError_t launch_fanout(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
+cudaError_t launch_flat_export(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
 cudaError_t launch_dispatch(cudaStream_t s, const DevHeap& H, const uint32_t* roots, uint32_t nforms,
                             uint32_t* keys, uint32_t* keys_alt, uint32_t* perm, uint32_t* perm_alt,
                             void* temp, size_t temp_bytes, uint32_t** perm_out, int sms);

@@ -37,7 +37,7 @@ __device__ __forceinline__ void write_result(const EvalArgs& A, uint32_t f, cons
   A.rerr[f] = o.err;
   A.rsteps[f] = o.steps;
   A.rword[f] = o.w;
-  if (o.err == E_OOM) atomicExch(&A.flags[0], 1);
+  if (o.err == E_OOM) atomicExch(&A.flags[0], 1);   // (E_PENDING: filled in by the fan-out finalizer)
 }
 
 __device__ __forceinline__ Ctx make_ctx(const EvalArgs& A, uint32_t slot) {
@@ -75,7 +75,7 @@ __global__ void __launch_bounds__(128) culi_eval_kernel(const __grid_constant__ 
     uint32_t i = b + lane;
     if (i < A.nforms) {
       uint32_t f = A.perm ? A.perm[i] : i;
-      FormOut o = eval_form(C, A.roots[f]);
+      FormOut o = eval_form(C, A.roots[f], f, 0, 0, A.fuel);
       write_result(A, f, o);
     }
   }
@@ -87,7 +87,7 @@ __global__ void culi_define_kernel(const __grid_constant__ EvalArgs A) {
   if (blockIdx.x != 0 || threadIdx.x != 0) return;
   Ctx C = make_ctx(A, 0);
   for (uint32_t f = 0; f < A.nforms; ++f) {
-    FormOut o = eval_form(C, A.roots[f]);
+    FormOut o = eval_form(C, A.roots[f], f, 0, 0, A.fuel);
     write_result(A, f, o);
     if (o.err) {
       A.flags[1] = (int)f + 1;
@@ -102,7 +102,9 @@ __global__ void culi_define_kernel(const __grid_constant__ EvalArgs A) {
 __global__ void __launch_bounds__(128) culi_export_kernel(ExportArgs X) {
   uint32_t slot = blockIdx.x * blockDim.x + threadIdx.x;
   uint32_t nthreads = gridDim.x * blockDim.x;
-  for (uint32_t f = slot; f < X.nforms; f += nthreads) {
+  uint32_t total = X.list ? X.nlist : X.nforms;
+  for (uint32_t q = slot; q < total; q += nthreads) {
+    uint32_t f = X.list ? X.list[q] : q;
     uint32_t t = X.rtag[f];
     if (t != K_CONS && t != K_STR) continue;
     uint32_t root = (uint32_t)X.rword[f];
@@ -148,11 +150,145 @@ __global__ void __launch_bounds__(128) culi_export_kernel(ExportArgs X) {
 }
 
 __global__ void culi_reset_kernel(unsigned long long* top, unsigned long long top_value, uint32_t* next,
-                                  unsigned long long* pcount, int* flags) {
+                                  unsigned long long* pcount, int* flags, uint32_t* npend,
+                                  uint32_t* nfallback) {
   *top = top_value;
   *next = 0;
   *pcount = 0;
+  *npend = 0;
+  *nfallback = 0;
   for (int k = 0; k < 8; ++k) flags[k] = 0;
+}
+
+// ---- ||| fan-out ------------------------------------------------
+// Element i of every pending descriptor is applied by one thread: f applied to (l1[i] .. lm[i]) at the
+// depth of the ||| form + 1, with the fuel left after the ||| arguments.  Lists are indexed in O(1)
+// through their contiguous spines (SURVEY c.14): cell i of list j is heads[j] + i, which the thread
+// verifies (cons, inside the heap as it was when the descriptor was written, linked to cell i+1); a
+// failed check or an element error marks the form for exact sequential re-evaluation.  Results go to
+// the preallocated spine (cells [spine, spine+n), boxes [spine+n, spine+2n)): coalesced stores.
+__global__ void __launch_bounds__(128) culi_fanout_kernel(const __grid_constant__ EvalArgs A) {
+  uint4* scode = culi_smem;
+  uint64_t* sgword = reinterpret_cast<uint64_t*>(culi_smem + A.code_n);
+  uint8_t* sgtag = reinterpret_cast<uint8_t*>(sgword + A.gst);
+  for (uint32_t i = threadIdx.x; i < A.code_n; i += blockDim.x) {
+    uint64_t w = A.H.word[A.code_lo + i];
+    scode[i] = make_uint4(lo32(w), hi32(w), A.H.tag[A.code_lo + i], 0);
+  }
+  for (uint32_t i = threadIdx.x; i < A.gst; i += blockDim.x) {
+    sgword[i] = A.H.gword[i];
+    sgtag[i] = A.H.gtag[i];
+  }
+  __syncthreads();
+  uint32_t slot = blockIdx.x * blockDim.x + threadIdx.x;
+  uint32_t nthreads = gridDim.x * blockDim.x;
+  Ctx C = make_ctx(A, slot);
+  uint32_t npend = *A.npend;
+  if (npend > A.maxdesc) npend = A.maxdesc;
+  const DevHeap& H = A.H;
+  for (uint32_t k = 0; k < npend; ++k) {
+    FanDesc* D = A.desc + k;
+    uint32_t n = D->n, m = D->m, spine = D->spine;
+    uint64_t top = D->top;
+    V f = mkv(D->ftag, D->fword);
+    uint64_t budget = A.fuel - D->steps0;
+    unsigned long long my_steps = 0;
+    uint32_t bad = 0, nonflat = 0;
+    for (uint32_t i = slot; i < n; i += nthreads) {
+      bool ok = true;
+      *VS(C, 0) = vpack(f, 0);
+      for (uint32_t j = 0; j < m; ++j) {
+        uint32_t c = D->heads[j] + i;
+        if ((uint64_t)c >= top) { ok = false; break; }
+        uint32_t tc = H.tag[c];
+        uint64_t wc = H.word[c];
+        if ((tc & KIND_MASK) != K_CONS || (i + 1 < n && hi32(wc) != c + 1)) { ok = false; break; }
+        *VS(C, 1 + j) = vpack(unbox(C, lo32(wc)), 0);
+      }
+      if (!ok) { bad |= 1; continue; }
+      FormOut o = eval_form(C, 0, D->form, 1, m, budget);
+      if (o.err) { bad |= 2; continue; }
+      my_steps += o.steps;
+      nonflat |= (o.t == K_CONS);
+      uint32_t ca = box_into(H, mkv(o.t, o.w), spine + n + i);
+      H.tag[spine + i] = K_CONS | TAG_PROPER;
+      H.word[spine + i] = pack2(ca, i + 1 < n ? spine + i + 1 : 0);
+    }
+    // warp-reduce, one atomic per warp
+    for (int o = 16; o > 0; o >>= 1) {
+      my_steps += __shfl_down_sync(0xffffffffu, my_steps, o);
+      bad |= __shfl_down_sync(0xffffffffu, bad, o);
+      nonflat |= __shfl_down_sync(0xffffffffu, nonflat, o);
+    }
+    if ((threadIdx.x & 31) == 0) {
+      if (my_steps) atomicAdd(&D->total, my_steps);
+      if (bad) atomicOr(&D->bad, bad);
+      if (nonflat) atomicOr(&D->nonflat, 1u);
+    }
+  }
+}
+
+// One thread per descriptor: write the ||| form's record, or queue it for sequential re-evaluation.
+__global__ void culi_fanout_finalize_kernel(const __grid_constant__ EvalArgs A) {
+  uint32_t npend = *A.npend;
+  if (npend > A.maxdesc) npend = A.maxdesc;
+  for (uint32_t k = blockIdx.x * blockDim.x + threadIdx.x; k < npend; k += gridDim.x * blockDim.x) {
+    const FanDesc* D = A.desc + k;
+    uint64_t steps = D->steps0 + D->total;
+    if (D->bad || steps > A.fuel) {
+      A.fallback[atomicAdd(A.nfallback, 1u)] = D->form;
+      continue;
+    }
+    A.rerr[D->form] = 0;
+    A.rsteps[D->form] = steps;
+    if (!D->nonflat && A.payload) {
+      // a flat list (no element is a cons): 2n+1 tokens written in parallel by culi_flat_export_kernel
+      unsigned long long ntok = 2ull * D->n + 1;
+      unsigned long long off = atomicAdd(A.pcount, ntok);
+      if (off + ntok > A.pcap) {
+        atomicExch(&A.flags[3], 1);
+        A.rtag[D->form] = K_CONS;
+        A.rword[D->form] = D->spine;
+        continue;
+      }
+      A.desc[k].flat_off = off;
+      A.rtag[D->form] = K_FLATREC;
+      A.rword[D->form] = (off & 0xffffffffull) | (ntok << 32);
+    } else {
+      A.rtag[D->form] = K_CONS;
+      A.rword[D->form] = D->spine;
+    }
+  }
+}
+
+// Export of flat ||| result lists (SURVEY §8(a)9 for the a6/a8 output): token 2i = the cons of cell i,
+// token 2i+1 = element i, token 2n = nil.  Grid-stride over all elements of all flat descriptors.
+__global__ void __launch_bounds__(256) culi_flat_export_kernel(const __grid_constant__ EvalArgs A) {
+  uint32_t npend = *A.npend;
+  if (npend > A.maxdesc) npend = A.maxdesc;
+  uint32_t tid = blockIdx.x * blockDim.x + threadIdx.x, nth = gridDim.x * blockDim.x;
+  for (uint32_t k = 0; k < npend; ++k) {
+    const FanDesc* D = A.desc + k;
+    if (A.rtag[D->form] != K_FLATREC) continue;
+    uint32_t n = D->n, spine = D->spine;
+    uint4* out = A.payload + D->flat_off;
+    for (uint32_t i = tid; i < n; i += nth) {
+      uint64_t cw = A.H.word[spine + i];
+      uint32_t e = lo32(cw);
+      uint32_t et = A.H.tag[e] & KIND_MASK;
+      uint64_t ew = A.H.word[e];
+      out[2 * i] = make_uint4(lo32(cw), hi32(cw), K_CONS, 0);
+      out[2 * i + 1] = make_uint4(lo32(ew), hi32(ew), et, 0);
+    }
+    if (tid == 0) out[2 * n] = make_uint4(0, 0, K_NIL, 0);
+  }
+}
+
+__global__ void culi_flat_commit_kernel(const __grid_constant__ EvalArgs A) {
+  uint32_t npend = *A.npend;
+  if (npend > A.maxdesc) npend = A.maxdesc;
+  for (uint32_t k = threadIdx.x; k < npend; k += blockDim.x)
+    if (A.rtag[A.desc[k].form] == K_FLATREC) A.rtag[A.desc[k].form] = K_CONS;
 }
 
 // ---- host launchers ----------------------------------------------------------------------------------
@@ -192,8 +328,31 @@ cudaError_t launch_export(cudaStream_t s, const ExportArgs& X, uint32_t blocks) 
 }
 
 cudaError_t launch_reset(cudaStream_t s, unsigned long long* top, unsigned long long top_value,
-                         uint32_t* next, unsigned long long* pcount, int* flags) {
-  culi_reset_kernel<<<1, 1, 0, s>>>(top, top_value, next, pcount, flags);
+                         uint32_t* next, unsigned long long* pcount, int* flags, uint32_t* npend,
+                         uint32_t* nfallback) {
+  culi_reset_kernel<<<1, 1, 0, s>>>(top, top_value, next, pcount, flags, npend, nfallback);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_fanout(cudaStream_t s, const EvalArgs& A, uint32_t blocks) {
+  size_t smem = eval_smem_bytes(A);
+  if (smem > 48 * 1024) {
+    cudaError_t e = cudaFuncSetAttribute(culi_fanout_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                         (int)smem);
+    if (e != cudaSuccess) return e;
+  }
+  culi_fanout_kernel<<<blocks, 128, smem, s>>>(A);
+  cudaError_t e = cudaGetLastError();
+  if (e != cudaSuccess) return e;
+  culi_fanout_finalize_kernel<<<1, 128, 0, s>>>(A);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_flat_export(cudaStream_t s, const EvalArgs& A, uint32_t blocks) {
+  culi_flat_export_kernel<<<blocks, 256, 0, s>>>(A);
+  cudaError_t e = cudaGetLastError();
+  if (e != cudaSuccess) return e;
+  culi_flat_commit_kernel<<<1, 128, 0, s>>>(A);
   return cudaGetLastError();
 }
 

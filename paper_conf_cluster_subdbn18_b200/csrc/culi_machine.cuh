@@ -24,6 +24,10 @@
 
 namespace culi {
 
+#ifndef CULI_COLD
+#define CULI_COLD __noinline__
+#endif
+
 extern __shared__ __align__(16) uint4 culi_smem[];   // [code nodes][global words][global tags]
 
 struct Ctx {
@@ -147,7 +151,7 @@ __device__ __forceinline__ V global_value(const Ctx& C, uint32_t sym) {
 }
 
 // full walk: innermost frame first, leftmost binding first, then the global frame; unbound -> itself
-__device__ __noinline__ V lookup_slow(const Ctx& C, uint32_t sym, uint32_t env) {
+__device__ CULI_COLD V lookup_slow(const Ctx& C, uint32_t sym, uint32_t env) {
   while (env != 0) {
     if (env & STACK_ENV) {
       uint32_t h = env & ENV_IDX_MASK, n = (env >> 16) & 0x7fffu;
@@ -187,7 +191,7 @@ __device__ __forceinline__ V lookup(const Ctx& C, uint32_t sym, uint32_t env) {
 
 // Copy the stack frames a closure captures into the heap (frames are immutable, c.3, so a copy is
 // indistinguishable from the original).  Memoised in the stack header's .y field.
-__device__ __noinline__ bool promote(const Ctx& C, uint32_t env, uint32_t* out) {
+__device__ CULI_COLD bool promote(const Ctx& C, uint32_t env, uint32_t* out) {
   const DevHeap& H = C.A->H;
   if (!(env & STACK_ENV)) { *out = env; return true; }
   for (;;) {
@@ -226,7 +230,7 @@ __device__ __noinline__ bool promote(const Ctx& C, uint32_t env, uint32_t* out) 
 
 // A closure / macro is two nodes: {kind: code | env << 32} and {K_AUX: nparams | first param << 32}
 // (code = the cons (params . body); env = heap frame or 0).
-__device__ __noinline__ bool make_closure(const Ctx& C, uint32_t kind, uint32_t code, uint32_t env,
+__device__ CULI_COLD bool make_closure(const Ctx& C, uint32_t kind, uint32_t code, uint32_t env,
                                           V* out) {
   uint32_t henv, a;
   if (!promote(C, env, &henv)) return false;
@@ -245,7 +249,7 @@ __device__ __noinline__ bool make_closure(const Ctx& C, uint32_t kind, uint32_t 
 }
 
 // c.5: a parameter list is a proper list of non-reserved symbols
-__device__ __noinline__ bool valid_params(const Ctx& C, uint32_t ps) {
+__device__ CULI_COLD bool valid_params(const Ctx& C, uint32_t ps) {
   if (ps == 0) return true;
   uint32_t t = ntag(C, ps);
   if ((t & KIND_MASK) != K_CONS || !(t & TAG_PROPER)) return false;
@@ -283,7 +287,7 @@ __device__ __forceinline__ bool eq_values(V a, V b) {
 }
 
 // one step of a numeric fold (types already checked); returns false on integer division by zero
-__device__ __noinline__ bool fold_float(uint32_t op, V& acc, V b) {
+__device__ CULI_COLD bool fold_float(uint32_t op, V& acc, V b) {
   double x = as_f64(acc), y = as_f64(b), r;
   switch (op) {
     case BI_ADD: r = __dadd_rn(x, y); break;
@@ -391,7 +395,7 @@ __device__ __forceinline__ uint8_t fast2(const Ctx& C, uint32_t op, uint32_t arg
 }
 
 // equal: recursive on cons cells, with the V-stack above vtop as the explicit work stack
-__device__ __noinline__ uint8_t equal_values(const Ctx& C, uint32_t vtop, V a, V b, bool* res) {
+__device__ CULI_COLD uint8_t equal_values(const Ctx& C, uint32_t vtop, V a, V b, bool* res) {
   uint32_t sp = vtop;
   for (;;) {
     bool same;
@@ -422,7 +426,7 @@ __device__ __noinline__ uint8_t equal_values(const Ctx& C, uint32_t vtop, V a, V
 }
 
 // general builtin application over vs[base+1 .. base+cnt] (any arity)
-__device__ __noinline__ uint8_t apply_builtin(const Ctx& C, uint32_t op, uint32_t base, uint32_t cnt,
+__device__ CULI_COLD uint8_t apply_builtin(const Ctx& C, uint32_t op, uint32_t base, uint32_t cnt,
                                               uint32_t vtop, V* out) {
   const DevHeap& H = C.A->H;
   if (((FAST_OPS >> op) & 1) && cnt <= 2) {
@@ -566,7 +570,7 @@ __device__ __noinline__ uint8_t apply_builtin(const Ctx& C, uint32_t op, uint32_
 
 // (||| n f l1 .. lm) argument checks (c.7): arity, types left to right, then n >= 0 and every list
 // proper with >= n elements.  Returns 0 and fills n, or an error.
-__device__ __noinline__ uint8_t par_check(const Ctx& C, uint32_t base, uint32_t cnt, uint32_t* n_out) {
+__device__ CULI_COLD uint8_t par_check(const Ctx& C, uint32_t base, uint32_t cnt, uint32_t* n_out) {
   if (cnt < 3) return E_ARITY;
   V nv = arg(C, base, 0), f = arg(C, base, 1);
   if (nv.t != K_INT) return E_TYPE;
@@ -586,8 +590,26 @@ __device__ __noinline__ uint8_t par_check(const Ctx& C, uint32_t base, uint32_t 
   return 0;
 }
 
+// The O(1) part of par_check: arity, types, n >= 0, every list proper, and no empty list when n > 0.
+__device__ CULI_COLD uint8_t par_check_light(const Ctx& C, uint32_t base, uint32_t cnt, uint32_t* n_out) {
+  if (cnt < 3) return E_ARITY;
+  V nv = arg(C, base, 0), f = arg(C, base, 1);
+  if (nv.t != K_INT) return E_TYPE;
+  if (f.t != K_BUILTIN && f.t != K_CLOSURE) return E_TYPE;
+  long long n = (long long)nv.w;
+  if (n < 0) return E_ARG;
+  for (uint32_t j = 2; j < cnt; ++j) {
+    V l = arg(C, base, j);
+    if (!proper_value(C, l)) return E_ARG;
+    if (n > 0 && l.t == K_NIL) return E_ARG;
+  }
+  if (n > 0x3fffffffll) return E_OOM;
+  *n_out = (uint32_t)n;
+  return 0;
+}
+
 // runtime syntax checks of special forms without TAG_VALID (c.5); cur = the argument list
-__device__ __noinline__ bool special_syntax_ok(const Ctx& C, uint32_t op, uint32_t cur) {
+__device__ CULI_COLD bool special_syntax_ok(const Ctx& C, uint32_t op, uint32_t cur) {
   uint32_t n = 0;
   for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
   switch (op) {
@@ -630,10 +652,14 @@ struct FormOut {
   uint8_t err;
 };
 
-__device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root) {
+// eval_form(C, root, form, 0, 0, fuel): evaluate the datum at node `root` at depth 1.
+// eval_form(C, 0, form, 1, m, budget): apply vs[0] to the m values vs[1..m] as the body of a top-level
+//   (||| ...) form (depth 1) — one fan-out element (c.7); `budget` = fuel left after the ||| arguments.
+__device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32_t form, int apply_mode,
+                                             uint32_t apply_cnt, uint64_t fuel) {
   const DevHeap& H = C.A->H;
   const uint32_t kcap = C.A->kcap, vcap = C.A->vcap, maxd = C.A->max_depth;
-  const uint64_t fuel = C.A->fuel;
+  const bool fanout = C.A->fanout && !apply_mode;
   V v = mkv(K_NIL, 0), a0 = mkv(K_NIL, 0), a1 = mkv(K_NIL, 0);
   uint32_t x = root, t = 0, env = 0, d = 1, cur = 0, base = 0, cnt = 0, sp = 0, vtop = 0;
   uint32_t a = 0, at = 0, nxt = 0, kd = 0, hop = 0;
@@ -662,6 +688,12 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root) {
   } while (0)
 #define ATOMVAL(n, tt, ww) (((tt) & KIND_MASK) == K_SYM ? lookup(C, (uint32_t)(ww), env) : unbox_loaded((n), (tt), (ww)))
 
+  if (apply_mode) {
+    base = 0;
+    cnt = apply_cnt;
+    vtop = 1 + cnt;
+    goto APPLY;
+  }
   // ======================================================== EVAL a code node x in env at depth d
 EVAL_NODE:
   ldnode(C, x, t, w);
@@ -885,6 +917,35 @@ APPLY: {                                                        // apply vs[base
   if (h.t != K_BUILTIN) FAIL(E_SYNTAX);
   if ((uint32_t)h.w == BI_PAR) {                                // (||| n f l1 ... lm), c.7
     uint32_t n;
+    if (fanout && sp == 0 && d == 1 && cnt >= 3 && cnt - 2 <= FANOUT_MAXM) {
+      // top-level ||| form: its arguments are evaluated; hand the elements to the fan-out kernel
+      // (SURVEY §8(a)6).  Errors decidable now are raised exactly; list lengths are verified by the
+      // element kernel (a short or non-contiguous list sends the form to sequential re-evaluation).
+      uint8_t e = par_check_light(C, base, cnt, &n);
+      if (e) FAIL(e);
+      if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
+      uint32_t slot = atomicAdd(C.A->npend, 1u);
+      if (slot < C.A->maxdesc) {
+        uint32_t spine;
+        if (!heap_alloc(H, 2 * n, &spine)) FAIL(E_OOM);
+        FanDesc* D = C.A->desc + slot;
+        V f = arg(C, base, 1);
+        D->form = form;
+        D->n = n;
+        D->m = cnt - 2;
+        D->spine = spine;
+        D->ftag = f.t;
+        D->depth = d;
+        D->fword = f.w;
+        D->steps0 = steps;
+        D->top = atomicAdd(H.top, 0ull);
+        for (uint32_t j = 0; j < cnt - 2; ++j) D->heads[j] = (uint32_t)arg(C, base, 2 + j).w;
+        D->total = 0;
+        D->bad = 0;
+        err = E_PENDING;
+        goto done;
+      }
+    }
     uint8_t e = par_check(C, base, cnt, &n);
     if (e) FAIL(e);
     if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
