@@ -183,7 +183,7 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   // stage the persistent code segment and the global frame in shared memory (batch mode only)
   bool stage = !define_mode && !(c->opts.flags & CULI_F_NO_STAGING);
   A.code_lo = IMG_FIRST;
-  A.code_n = stage ? (uint32_t)std::min<uint64_t>(c->mark - IMG_FIRST, 1536) : 0;
+  A.code_n = (stage && CULI_STAGE_CODE) ? (uint32_t)std::min<uint64_t>(c->mark - IMG_FIRST, 1536) : 0;
   A.gst = stage ? (uint32_t)std::min<size_t>(c->syms->names.size(), 2048) : 0;
   return A;
 }
@@ -266,6 +266,7 @@ static int run_batch_device(culi_ctx* c) {
   }
   CK(cudaEventRecord(c->ev[1], c->stream));
   EvalArgs A = make_args(c, nf, perm, 0);
+  A.fanout = A.fanout && c->batch_has_par;
   uint32_t blocks = c->nslots / 128;
   uint32_t need = (nf + 127) / 128;
   if (need < blocks) blocks = std::max<uint32_t>(need, 1);

@@ -20,6 +20,11 @@ namespace culi {
 
 constexpr uint32_t STACK_ENV = 0x80000000u;   // env reference into the thread's V-stack
 
+// Serve the persistent code segment from shared memory (see culi_machine.cuh ldnode); off by default.
+#ifndef CULI_STAGE_CODE
+#define CULI_STAGE_CODE 0
+#endif
+
 struct DevHeap {
   uint8_t* tag;
   uint64_t* word;

@@ -51,7 +51,8 @@ __device__ __forceinline__ Ctx make_ctx(const EvalArgs& A, uint32_t slot) {
 // Batch mode.  Shared memory per block: the persistent code segment [code_lo, code_lo + code_n) as
 // {w.lo, w.hi, tag, 0} and the global frame [0, gst) ("stage").  Each warp takes 32
 // consecutive forms of the (binned) order with one atomicAdd and runs them to completion.
-__global__ void __launch_bounds__(128) culi_eval_kernel(const __grid_constant__ EvalArgs A) {
+template <bool FANOUT>
+__global__ void __launch_bounds__(128, 4) culi_eval_kernel(const __grid_constant__ EvalArgs A) {
   uint4* scode = culi_smem;
   uint64_t* sgword = reinterpret_cast<uint64_t*>(culi_smem + A.code_n);
   uint8_t* sgtag = reinterpret_cast<uint8_t*>(sgword + A.gst);
@@ -75,7 +76,7 @@ __global__ void __launch_bounds__(128) culi_eval_kernel(const __grid_constant__ 
     uint32_t i = b + lane;
     if (i < A.nforms) {
       uint32_t f = A.perm ? A.perm[i] : i;
-      FormOut o = eval_form(C, A.roots[f], f, 0, 0, A.fuel);
+      FormOut o = eval_form<FANOUT, false>(C, A.roots[f], f, 0, 0, A.fuel);
       write_result(A, f, o);
     }
   }
@@ -87,7 +88,7 @@ __global__ void culi_define_kernel(const __grid_constant__ EvalArgs A) {
   if (blockIdx.x != 0 || threadIdx.x != 0) return;
   Ctx C = make_ctx(A, 0);
   for (uint32_t f = 0; f < A.nforms; ++f) {
-    FormOut o = eval_form(C, A.roots[f], f, 0, 0, A.fuel);
+    FormOut o = eval_form<false, false>(C, A.roots[f], f, 0, 0, A.fuel);
     write_result(A, f, o);
     if (o.err) {
       A.flags[1] = (int)f + 1;
@@ -167,7 +168,7 @@ __global__ void culi_reset_kernel(unsigned long long* top, unsigned long long to
 // verifies (cons, inside the heap as it was when the descriptor was written, linked to cell i+1); a
 // failed check or an element error marks the form for exact sequential re-evaluation.  Results go to
 // the preallocated spine (cells [spine, spine+n), boxes [spine+n, spine+2n)): coalesced stores.
-__global__ void __launch_bounds__(128) culi_fanout_kernel(const __grid_constant__ EvalArgs A) {
+__global__ void __launch_bounds__(128, 4) culi_fanout_kernel(const __grid_constant__ EvalArgs A) {
   uint4* scode = culi_smem;
   uint64_t* sgword = reinterpret_cast<uint64_t*>(culi_smem + A.code_n);
   uint8_t* sgtag = reinterpret_cast<uint8_t*>(sgword + A.gst);
@@ -206,7 +207,7 @@ __global__ void __launch_bounds__(128) culi_fanout_kernel(const __grid_constant_
         *VS(C, 1 + j) = vpack(unbox(C, lo32(wc)), 0);
       }
       if (!ok) { bad |= 1; continue; }
-      FormOut o = eval_form(C, 0, D->form, 1, m, budget);
+      FormOut o = eval_form<false, true>(C, 0, D->form, 1, m, budget);
       if (o.err) { bad |= 2; continue; }
       my_steps += o.steps;
       nonflat |= (o.t == K_CONS);
@@ -309,11 +310,14 @@ size_t eval_smem_bytes(const EvalArgs& A) {
 cudaError_t launch_eval(cudaStream_t s, const EvalArgs& A, uint32_t blocks) {
   size_t smem = eval_smem_bytes(A);
   if (smem > 48 * 1024) {
-    cudaError_t e = cudaFuncSetAttribute(culi_eval_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                         (int)smem);
+    cudaError_t e = cudaFuncSetAttribute(A.fanout ? culi_eval_kernel<true> : culi_eval_kernel<false>,
+                                         cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     if (e != cudaSuccess) return e;
   }
-  culi_eval_kernel<<<blocks, 128, smem, s>>>(A);
+  if (A.fanout)
+    culi_eval_kernel<true><<<blocks, 128, smem, s>>>(A);   // batches holding top-level ||| forms
+  else
+    culi_eval_kernel<false><<<blocks, 128, smem, s>>>(A);
   return cudaGetLastError();
 }
 

@@ -65,26 +65,39 @@ __device__ __forceinline__ const uint8_t* sm_gtag(const Ctx& C) {
   return reinterpret_cast<const uint8_t*>(sm_gword(C) + C.A->gst);
 }
 
-// ---- heap access (SoA: tag u8[], word u64[]) with the staged code segment -----------
+// ---- heap access (SoA: tag u8[], word u64[]) ------------------------------------------
+// CULI_STAGE_CODE=1 serves the persistent code segment from shared memory.  Measured on C2 (round 1):
+// the range check makes every node load execute both paths predicated (~25 % of all instructions),
+// which costs more than the L1 hits it replaces, so it is off by default; the global frame (one lookup
+// site) stays staged.
+#ifndef CULI_STAGE_CODE
+#define CULI_STAGE_CODE 0
+#endif
 __device__ __forceinline__ void ldnode(const Ctx& C, uint32_t n, uint32_t& t, uint64_t& w) {
+#if CULI_STAGE_CODE
   uint32_t r = n - C.A->code_lo;
   if (r < C.A->code_n) {
     uint4 q = culi_smem[r];
     t = q.z;
     w = ((uint64_t)q.y << 32) | q.x;
-  } else {
-    t = C.A->H.tag[n];
-    w = C.A->H.word[n];
+    return;
   }
+#endif
+  t = C.A->H.tag[n];
+  w = C.A->H.word[n];
 }
 __device__ __forceinline__ uint64_t nword(const Ctx& C, uint32_t n) {
+#if CULI_STAGE_CODE
   uint32_t r = n - C.A->code_lo;
   if (r < C.A->code_n) { uint2 q = *reinterpret_cast<const uint2*>(&culi_smem[r]); return ((uint64_t)q.y << 32) | q.x; }
+#endif
   return C.A->H.word[n];
 }
 __device__ __forceinline__ uint32_t ntag(const Ctx& C, uint32_t n) {
+#if CULI_STAGE_CODE
   uint32_t r = n - C.A->code_lo;
   if (r < C.A->code_n) return culi_smem[r].z;
+#endif
   return C.A->H.tag[n];
 }
 __device__ __forceinline__ V unbox_loaded(uint32_t n, uint32_t t, uint64_t w) {
@@ -655,11 +668,12 @@ struct FormOut {
 // eval_form(C, root, form, 0, 0, fuel): evaluate the datum at node `root` at depth 1.
 // eval_form(C, 0, form, 1, m, budget): apply vs[0] to the m values vs[1..m] as the body of a top-level
 //   (||| ...) form (depth 1) — one fan-out element (c.7); `budget` = fuel left after the ||| arguments.
+template <bool FANOUT, bool APPLY>
 __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32_t form, int apply_mode,
                                              uint32_t apply_cnt, uint64_t fuel) {
   const DevHeap& H = C.A->H;
   const uint32_t kcap = C.A->kcap, vcap = C.A->vcap, maxd = C.A->max_depth;
-  const bool fanout = C.A->fanout && !apply_mode;
+  const bool fanout = FANOUT && !APPLY && C.A->fanout;
   V v = mkv(K_NIL, 0), a0 = mkv(K_NIL, 0), a1 = mkv(K_NIL, 0);
   uint32_t x = root, t = 0, env = 0, d = 1, cur = 0, base = 0, cnt = 0, sp = 0, vtop = 0;
   uint32_t a = 0, at = 0, nxt = 0, kd = 0, hop = 0;
@@ -688,7 +702,7 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32
   } while (0)
 #define ATOMVAL(n, tt, ww) (((tt) & KIND_MASK) == K_SYM ? lookup(C, (uint32_t)(ww), env) : unbox_loaded((n), (tt), (ww)))
 
-  if (apply_mode) {
+  if (APPLY && apply_mode) {
     base = 0;
     cnt = apply_cnt;
     vtop = 1 + cnt;

@@ -12,7 +12,7 @@ fi
 timeout 600 python bench.py --workload $WL > $OUT/bench_$WL.json 2> $OUT/bench_$WL.err; tail -3 $OUT/bench_$WL.err; cat $OUT/bench_$WL.json
 if [ -z "$SKIP_NCU" ]; then
   timeout 600 ncu --metrics gpu__time_duration.sum --clock-control none -c 200 --csv --log-file $OUT/launches_$WL.csv python bench.py --workload $WL --steps 2 --warmup 1 --e2e-steps 1 --no-cpu-baseline > $OUT/ncu_launch_bench.log 2>&1
-  timeout 900 ncu --set full --clock-control none --import-source on -k regex:culi_eval_kernel -s 1 -c 1 -o $OUT/prof_$WL -f python bench.py --workload $WL --steps 1 --warmup 1 --e2e-steps 1 --no-cpu-baseline > $OUT/ncu_full.log 2>&1
+  timeout 900 ncu --set full --clock-control none --import-source on -k regex:${KREGEX:-culi_eval_kernel} -s 1 -c 1 -o $OUT/prof_$WL -f python bench.py --workload $WL --steps 1 --warmup 1 --e2e-steps 1 --no-cpu-baseline > $OUT/ncu_full.log 2>&1
   tail -3 $OUT/ncu_full.log
 fi
 if [ -f $OUT/prof_$WL.ncu-rep ]; then
