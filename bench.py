@@ -193,9 +193,17 @@ def culi_arm(args):
     local = int(os.environ.get("LOCAL_RANK", "0"))
     if world != args.gpus:
         args.gpus = world
+    # CULI_SHARE_DEVICE=1 + CULI_DIST_BACKEND=gloo: every rank on cuda:0 (exercises the N>1 path on one GPU)
+    if os.environ.get("CULI_SHARE_DEVICE") == "1":
+        local = 0
+    backend = os.environ.get("CULI_DIST_BACKEND", "nccl")
     torch.cuda.set_device(local)
     if world > 1:
-        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        if backend == "nccl":
+            dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        else:
+            dist.init_process_group(backend)
+    cdev = torch.device("cuda", local) if backend == "nccl" else torch.device("cpu")   # collective buffers
     B.build()
     culi.load()
     stream = torch.cuda.current_stream()
@@ -241,7 +249,12 @@ def culi_arm(args):
         ctx.eval_uploaded(h)
         if world > 1:
             ctx.records_device(rec.data_ptr(), rec.numel())
-            dist.all_gather_into_tensor(gathered, rec)
+            if cdev.type == "cuda":
+                dist.all_gather_into_tensor(gathered, rec)
+            else:
+                g = torch.empty(world * rec.numel(), dtype=torch.uint8)
+                dist.all_gather_into_tensor(g, rec.cpu())
+                gathered.copy_(g)
 
     for _ in range(args.warmup):
         step()
@@ -274,10 +287,10 @@ def culi_arm(args):
     t_rank = sum(step_ms) / 1e3
     t_max = t_rank
     if world > 1:
-        tt = torch.tensor([t_rank], dtype=torch.float64, device=dev)
+        tt = torch.tensor([t_rank], dtype=torch.float64, device=cdev)
         dist.all_reduce(tt, op=dist.ReduceOp.MAX)
         t_max = float(tt.item())
-        agg = torch.tensor([units_rank, total_steps], dtype=torch.float64, device=dev)
+        agg = torch.tensor([units_rank, total_steps], dtype=torch.float64, device=cdev)
         dist.all_reduce(agg)
         units_all, steps_all = float(agg[0].item()), float(agg[1].item())
     else:
@@ -305,7 +318,7 @@ def culi_arm(args):
         del r
     t_e2e = sum(e2e_ms) / 1e3
     if world > 1:
-        tt = torch.tensor([t_e2e], dtype=torch.float64, device=dev)
+        tt = torch.tensor([t_e2e], dtype=torch.float64, device=cdev)
         dist.all_reduce(tt, op=dist.ReduceOp.MAX)
         t_e2e = float(tt.item())
     e2e_value = units_all * len(e2e_ms) / t_e2e
