@@ -655,6 +655,55 @@ __device__ CULI_COLD bool special_syntax_ok(const Ctx& C, uint32_t op, uint32_t 
   return false;
 }
 
+// ---- leaf forms ------------------------------------------------------------------------------------------
+// x (tag xt, word xw) is a list whose own eval step was already counted at depth dx.  If x is a *leaf*
+// (op a [b]) — op a reserved builtin of FAST_OPS, a and b atoms or symbols — evaluate it right here:
+// the head step, then each argument step (all at depth dx + 1, with the fuel/depth checks in the same
+// order as the recursive definition, c.4), then the builtin.  Returns 1 with *out, 2 with *err, or 0
+// (not a leaf: nothing counted, nothing changed).  Saves the continuation push/pop of the common
+// arithmetic leaves, e.g. (- n 1), (< n 2), (* k x).
+__device__ __forceinline__ int try_leaf(const Ctx& C, uint32_t xt, uint64_t xw, uint32_t dx, uint32_t env,
+                                        uint64_t& steps, uint64_t fuel, uint32_t maxd, V* out, uint8_t* err) {
+  if (!(xt & TAG_PROPER)) return 0;
+  uint32_t ht;
+  uint64_t hw;
+  ldnode(C, lo32(xw), ht, hw);
+  if ((ht & KIND_MASK) != K_SYM || hw < N_SPECIALS || hw >= N_RESERVED) return 0;
+  uint32_t op = (uint32_t)hw - N_SPECIALS;
+  if (!((FAST_OPS >> op) & 1)) return 0;
+  uint32_t c1 = hi32(xw), argc = 0, n1 = 0, n2 = 0, t1 = 0, t2 = 0;
+  uint64_t w1 = 0, w2 = 0;
+  if (c1 != 0) {
+    uint64_t cw1 = nword(C, c1);
+    n1 = lo32(cw1);
+    uint32_t c2 = hi32(cw1);
+    ldnode(C, n1, t1, w1);
+    if ((t1 & KIND_MASK) == K_CONS) return 0;
+    argc = 1;
+    if (c2 != 0) {
+      uint64_t cw2 = nword(C, c2);
+      if (hi32(cw2) != 0) return 0;
+      n2 = lo32(cw2);
+      ldnode(C, n2, t2, w2);
+      if ((t2 & KIND_MASK) == K_CONS) return 0;
+      argc = 2;
+    }
+  }
+  for (uint32_t i = 0; i <= argc; ++i) {              // head step, then one step per argument
+    ++steps;
+    if (__builtin_expect(steps > fuel || dx + 1 > maxd, 0)) {
+      *err = steps > fuel ? E_FUEL : E_DEPTH;
+      return 2;
+    }
+  }
+  V a0 = mkv(K_NIL, 0), a1 = mkv(K_NIL, 0);
+  if (argc > 0) a0 = (t1 & KIND_MASK) == K_SYM ? lookup(C, (uint32_t)w1, env) : unbox_loaded(n1, t1, w1);
+  if (argc > 1) a1 = (t2 & KIND_MASK) == K_SYM ? lookup(C, (uint32_t)w2, env) : unbox_loaded(n2, t2, w2);
+  uint8_t e = fast2(C, op, argc, a0, a1, out);
+  if (__builtin_expect(e != 0, 0)) { *err = e; return 2; }
+  return 1;
+}
+
 // ---- the machine ---------------------------------------------------------------------------------------
 enum KKind : uint32_t { KF_HEAD = 1, KF_ARGS, KF_BODY, KF_IF, KF_LET, KF_DEFINE, KF_MACRO, KF_PAR, KF_DATA };
 
@@ -687,14 +736,14 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32
 #define STEP(depth)                                     \
   do {                                                  \
     ++steps;                                            \
-    if (steps > fuel || (depth) > maxd) {               \
+    if (__builtin_expect(steps > fuel || (depth) > maxd, 0)) { \
       err = steps > fuel ? E_FUEL : E_DEPTH;            \
       goto done;                                        \
     }                                                   \
   } while (0)
 #define KPUSH(kind, cursor, envv, vsb, depth, count)                                  \
   do {                                                                                \
-    if (sp >= kcap) FAIL(E_OOM);                                                      \
+    if (__builtin_expect(!!(sp >= kcap), 0)) FAIL(E_OOM);                                                      \
     if (kdirty) *KS(C, sp - 1) = ktop;                                                \
     ktop = make_uint4((cursor), (envv), (vsb), kmeta((depth), (kind), (count)));      \
     kdirty = true;                                                                    \
@@ -746,39 +795,47 @@ HEAD:
       nxt = hi32(w0);
       ldnode(C, a, at, aw);
       STEP(d + 1);
-      if ((at & KIND_MASK) == K_CONS || cnt == 2) {             // spill to the general path
-        if (vtop + 3 >= vcap) FAIL(E_OOM);
+      int leaf = 0;
+      V av;
+      if ((at & KIND_MASK) == K_CONS) {
+        leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &av, &err);
+        if (__builtin_expect(leaf == 2, 0)) goto done;
+      } else {
+        av = ATOMVAL(a, at, aw);
+      }
+      if ((at & KIND_MASK) == K_CONS && leaf == 0 || cnt == 2) {   // spill to the general path
+        if (__builtin_expect(!!(vtop + 3 >= vcap), 0)) FAIL(E_OOM);
         base = vtop;
         *VS(C, base) = vpack(mkv(K_BUILTIN, hop), 0);
         if (cnt > 0) *VS(C, base + 1) = vpack(a0, 0);
         if (cnt > 1) *VS(C, base + 2) = vpack(a1, 0);
-        if ((at & KIND_MASK) == K_CONS) {
+        if ((at & KIND_MASK) == K_CONS && leaf == 0) {
           vtop = base + 1 + cnt;
           KPUSH(KF_ARGS, nxt, env, base, d, cnt);
           x = a; t = at; w = aw; d = d + 1;
           goto EVAL_CONS;
         }
-        *VS(C, base + 1 + cnt) = vpack(ATOMVAL(a, at, aw), 0);
+        *VS(C, base + 1 + cnt) = vpack(av, 0);
         ++cnt;
         cur = nxt;
         goto ARGS;
       }
-      if (cnt == 0) a0 = ATOMVAL(a, at, aw); else a1 = ATOMVAL(a, at, aw);
+      if (cnt == 0) a0 = av; else a1 = av;
       ++cnt;
       cur = nxt;
     }
     {
       uint8_t e = fast2(C, hop, cnt, a0, a1, &v);
-      if (e) FAIL(e);
+      if (__builtin_expect(!!(e), 0)) FAIL(e);
     }
     goto RET;
   }
   if (v.t == K_SPECIAL) {
     uint32_t op = (uint32_t)v.w;
     if (op == SP_DEFINE || op == SP_DEFUN || op == SP_DEFMACRO) {
-      if (!C.A->define_mode) FAIL(E_DEFINE_IN_BATCH);
+      if (__builtin_expect(!!(!C.A->define_mode), 0)) FAIL(E_DEFINE_IN_BATCH);
     }
-    if (!(t & TAG_VALID) && !special_syntax_ok(C, op, cur)) FAIL(E_SYNTAX);
+    if (__builtin_expect(!!(!(t & TAG_VALID) && !special_syntax_ok(C, op, cur)), 0)) FAIL(E_SYNTAX);
     switch (op) {
       case SP_IF: {
         w0 = nword(C, cur);
@@ -787,11 +844,16 @@ HEAD:
         ldnode(C, a, at, aw);
         STEP(d + 1);
         if ((at & KIND_MASK) == K_CONS) {
-          KPUSH(KF_IF, c1, env, vtop, d, 0);
-          x = a; t = at; w = aw; d = d + 1;
-          goto EVAL_CONS;
+          int leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &v, &err);
+          if (__builtin_expect(leaf == 2, 0)) goto done;
+          if (leaf == 0) {
+            KPUSH(KF_IF, c1, env, vtop, d, 0);
+            x = a; t = at; w = aw; d = d + 1;
+            goto EVAL_CONS;
+          }
+        } else {
+          v = ATOMVAL(a, at, aw);
         }
-        v = ATOMVAL(a, at, aw);
         cur = c1;
         goto IF_BRANCH;
       }
@@ -801,13 +863,13 @@ HEAD:
       case SP_PROGN:
         goto BODY;
       case SP_LAMBDA:
-        if (!make_closure(C, K_CLOSURE, cur, env, &v)) FAIL(E_OOM);
+        if (__builtin_expect(!!(!make_closure(C, K_CLOSURE, cur, env, &v)), 0)) FAIL(E_OOM);
         goto RET;
       case SP_LET: {
         w0 = nword(C, cur);
         uint32_t bl = lo32(w0), body = hi32(w0);
         if (bl == 0) { cur = body; goto BODY; }
-        if (vtop >= vcap) FAIL(E_OOM);
+        if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
         base = vtop;
         *VS(C, base) = make_uint4(body, 0, 0, K_FRAME);         // header (holds the body for now)
         cnt = 0;
@@ -825,7 +887,7 @@ HEAD:
         w0 = nword(C, cur);
         uint32_t s = (uint32_t)nword(C, lo32(w0));
         V clo;
-        if (!make_closure(C, op == SP_DEFUN ? K_CLOSURE : K_MACRO, hi32(w0), env, &clo)) FAIL(E_OOM);
+        if (__builtin_expect(!!(!make_closure(C, op == SP_DEFUN ? K_CLOSURE : K_MACRO, hi32(w0), env, &clo)), 0)) FAIL(E_OOM);
         H.gtag[s] = (uint8_t)clo.t;
         H.gword[s] = clo.w;
         v = mkv(K_SYM, s);
@@ -842,14 +904,14 @@ HEAD:
     a = cur;
     while (ps != 0 && a != 0) {                                 // bind params to UNevaluated forms
       uint64_t pw = nword(C, ps), aw2 = nword(C, a);
-      if (hdr + 1 + n >= vcap) FAIL(E_OOM);
+      if (__builtin_expect(!!(hdr + 1 + n >= vcap), 0)) FAIL(E_OOM);
       *VS(C, hdr + 1 + n) = vpack(unbox(C, lo32(aw2)), (uint32_t)nword(C, lo32(pw)));
       ++n;
       ps = hi32(pw);
       a = hi32(aw2);
     }
-    if (ps != 0 || a != 0) FAIL(E_ARITY);
-    if (n >= 0x8000u) FAIL(E_OOM);
+    if (__builtin_expect(!!(ps != 0 || a != 0), 0)) FAIL(E_ARITY);
+    if (__builtin_expect(!!(n >= 0x8000u), 0)) FAIL(E_OOM);
     *VS(C, hdr) = make_uint4(menv, 0, n, K_FRAME);
     KPUSH(KF_MACRO, 0, env, hdr, d, 0);
     env = stack_env(hdr, n);
@@ -864,20 +926,20 @@ HEAD:
     for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
     if (n == 0) { v = mkv(K_NIL, 0); goto RET; }
     uint32_t s;
-    if (!heap_alloc(H, 2 * n, &s)) FAIL(E_OOM);
+    if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &s)), 0)) FAIL(E_OOM);
     if (data) {
       uint32_t ca = box_into(H, v, s + n);
       H.tag[s] = K_CONS | TAG_PROPER;
       H.word[s] = pack2(ca, n > 1 ? s + 1 : 0);
     }
-    if (vtop >= vcap) FAIL(E_OOM);
+    if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
     base = vtop;
     *VS(C, base) = make_uint4(s, n, 0, 0);                      // {spine, n}
     cnt = data ? 1 : 0;                                         // next element index
     goto DATA_LOOP;
   }
   // BUILTIN or CLOSURE: evaluate the args left to right at depth d+1 onto the V-stack
-  if (vtop >= vcap) FAIL(E_OOM);
+  if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
   base = vtop;
   *VS(C, base) = vpack(v, 0);
   cnt = 0;
@@ -889,14 +951,21 @@ ARGS:
     nxt = hi32(w0);
     ldnode(C, a, at, aw);
     STEP(d + 1);
+    V av;
     if ((at & KIND_MASK) == K_CONS) {
-      vtop = base + 1 + cnt;
-      KPUSH(KF_ARGS, nxt, env, base, d, cnt);
-      x = a; t = at; w = aw; d = d + 1;
-      goto EVAL_CONS;
+      int leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &av, &err);
+      if (__builtin_expect(leaf == 2, 0)) goto done;
+      if (leaf == 0) {
+        vtop = base + 1 + cnt;
+        KPUSH(KF_ARGS, nxt, env, base, d, cnt);
+        x = a; t = at; w = aw; d = d + 1;
+        goto EVAL_CONS;
+      }
+    } else {
+      av = ATOMVAL(a, at, aw);
     }
-    if (base + 1 + cnt >= vcap) FAIL(E_OOM);
-    *VS(C, base + 1 + cnt) = vpack(ATOMVAL(a, at, aw), 0);
+    if (__builtin_expect(!!(base + 1 + cnt >= vcap), 0)) FAIL(E_OOM);
+    *VS(C, base + 1 + cnt) = vpack(av, 0);
     ++cnt;
     cur = nxt;
   }
@@ -908,7 +977,7 @@ APPLY: {                                                        // apply vs[base
     uint64_t cwd = nword(C, (uint32_t)h.w);
     uint64_t aux = nword(C, (uint32_t)h.w + 1);
     uint32_t np = lo32(aux);
-    if (np != cnt) FAIL(E_ARITY);
+    if (__builtin_expect(!!(np != cnt), 0)) FAIL(E_ARITY);
     uint32_t code = lo32(cwd);
     uint32_t body = cdr_of(C, code);
     if (np == 1) {
@@ -921,14 +990,14 @@ APPLY: {                                                        // apply vs[base
         ps = hi32(pw);
       }
     }
-    if (cnt >= 0x8000u) FAIL(E_OOM);
+    if (__builtin_expect(!!(cnt >= 0x8000u), 0)) FAIL(E_OOM);
     *VS(C, base) = make_uint4(hi32(cwd), 0, cnt, K_FRAME);
     env = stack_env(base, cnt);
     vtop = base + 1 + cnt;
     cur = body;
     goto BODY;
   }
-  if (h.t != K_BUILTIN) FAIL(E_SYNTAX);
+  if (__builtin_expect(!!(h.t != K_BUILTIN), 0)) FAIL(E_SYNTAX);
   if ((uint32_t)h.w == BI_PAR) {                                // (||| n f l1 ... lm), c.7
     uint32_t n;
     if (fanout && sp == 0 && d == 1 && cnt >= 3 && cnt - 2 <= FANOUT_MAXM) {
@@ -936,12 +1005,12 @@ APPLY: {                                                        // apply vs[base
       // (SURVEY §8(a)6).  Errors decidable now are raised exactly; list lengths are verified by the
       // element kernel (a short or non-contiguous list sends the form to sequential re-evaluation).
       uint8_t e = par_check_light(C, base, cnt, &n);
-      if (e) FAIL(e);
+      if (__builtin_expect(!!(e), 0)) FAIL(e);
       if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
       uint32_t slot = atomicAdd(C.A->npend, 1u);
       if (slot < C.A->maxdesc) {
         uint32_t spine;
-        if (!heap_alloc(H, 2 * n, &spine)) FAIL(E_OOM);
+        if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
         FanDesc* D = C.A->desc + slot;
         V f = arg(C, base, 1);
         D->form = form;
@@ -961,10 +1030,10 @@ APPLY: {                                                        // apply vs[base
       }
     }
     uint8_t e = par_check(C, base, cnt, &n);
-    if (e) FAIL(e);
+    if (__builtin_expect(!!(e), 0)) FAIL(e);
     if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
     uint32_t m = cnt - 2, spine;
-    if (!heap_alloc(H, 2 * n, &spine)) FAIL(E_OOM);
+    if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
     // state: vs[base] = {spine, n}, vs[base+1] = f, vs[base+2+j] = list cursor j
     V f = arg(C, base, 1);
     for (uint32_t j = 0; j < m; ++j) *VS(C, base + 2 + j) = *VS(C, base + 3 + j);
@@ -975,7 +1044,7 @@ APPLY: {                                                        // apply vs[base
   }
   {
     uint8_t e = apply_builtin(C, (uint32_t)h.w, base, cnt, vtop, &v);
-    if (e) FAIL(e);
+    if (__builtin_expect(!!(e), 0)) FAIL(e);
   }
   vtop = base;
   goto RET;
@@ -1015,14 +1084,21 @@ LET_LOOP:
     uint32_t e = car_of(C, hi32(bw));
     ldnode(C, e, at, aw);
     STEP(d + 1);
+    V lv;
     if ((at & KIND_MASK) == K_CONS) {
-      vtop = base + 1 + cnt;
-      KPUSH(KF_LET, cur, env, base, d, cnt);
-      x = e; t = at; w = aw; d = d + 1;
-      goto EVAL_CONS;
+      int leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &lv, &err);
+      if (__builtin_expect(leaf == 2, 0)) goto done;
+      if (leaf == 0) {
+        vtop = base + 1 + cnt;
+        KPUSH(KF_LET, cur, env, base, d, cnt);
+        x = e; t = at; w = aw; d = d + 1;
+        goto EVAL_CONS;
+      }
+    } else {
+      lv = ATOMVAL(e, at, aw);
     }
-    if (base + 1 + cnt >= vcap || cnt >= 0x7fffu) FAIL(E_OOM);
-    *VS(C, base + 1 + cnt) = vpack(ATOMVAL(e, at, aw), (uint32_t)nword(C, lo32(bw)));
+    if (__builtin_expect(!!(base + 1 + cnt >= vcap || cnt >= 0x7fffu), 0)) FAIL(E_OOM);
+    *VS(C, base + 1 + cnt) = vpack(lv, (uint32_t)nword(C, lo32(bw)));
     ++cnt;
     cur = hi32(w0);
   }
@@ -1066,7 +1142,7 @@ PAR_NEXT: {
   uint32_t m = kcount(ktop.w), pb = ktop.z;
   V f = vunpack(*VS(C, pb + 1));
   base = pb + 2 + m;
-  if (base + 1 + m >= vcap) FAIL(E_OOM);
+  if (__builtin_expect(!!(base + 1 + m >= vcap), 0)) FAIL(E_OOM);
   *VS(C, base) = vpack(f, 0);
   for (uint32_t j = 0; j < m; ++j) {
     uint4* cj = VS(C, pb + 2 + j);
@@ -1091,7 +1167,7 @@ RET:
   switch (kkind(k.w)) {
     case KF_ARGS:
       base = k.z; cnt = kcount(k.w);
-      if (base + 1 + cnt >= vcap) FAIL(E_OOM);
+      if (__builtin_expect(!!(base + 1 + cnt >= vcap), 0)) FAIL(E_OOM);
       *VS(C, base + 1 + cnt) = vpack(v, 0);
       ++cnt;
       cur = k.x; env = k.y; d = kd;
@@ -1110,7 +1186,7 @@ RET:
       base = k.z; cnt = kcount(k.w);
       w0 = nword(C, k.x);
       uint32_t sym = (uint32_t)nword(C, car_of(C, lo32(w0)));
-      if (base + 1 + cnt >= vcap || cnt >= 0x7fffu) FAIL(E_OOM);
+      if (__builtin_expect(!!(base + 1 + cnt >= vcap || cnt >= 0x7fffu), 0)) FAIL(E_OOM);
       *VS(C, base + 1 + cnt) = vpack(v, sym);
       ++cnt;
       cur = hi32(w0); env = k.y; d = kd;
