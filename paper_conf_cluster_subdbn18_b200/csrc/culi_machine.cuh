@@ -241,7 +241,8 @@ __device__ CULI_COLD bool promote(const Ctx& C, uint32_t env, uint32_t* out) {
   }
 }
 
-// A closure / macro is two nodes: {kind: code | env << 32} and {K_AUX: nparams | first param << 32}
+// A closure / macro is three nodes: {kind: code | env << 32}, {K_AUX: nparams | first param << 32} and
+// {K_AUX: body | params << 32}, so a call reads all it needs with three independent loads
 // (code = the cons (params . body); env = heap frame or 0).
 __device__ CULI_COLD bool make_closure(const Ctx& C, uint32_t kind, uint32_t code, uint32_t env,
                                           V* out) {
@@ -252,11 +253,13 @@ __device__ CULI_COLD bool make_closure(const Ctx& C, uint32_t kind, uint32_t cod
     if (np == 0) first = (uint32_t)nword(C, car_of(C, p));
     ++np;
   }
-  if (!heap_alloc(C.A->H, 2, &a)) return false;
+  if (!heap_alloc(C.A->H, 3, &a)) return false;
   C.A->H.tag[a] = (uint8_t)kind;
   C.A->H.word[a] = pack2(code, henv);
   C.A->H.tag[a + 1] = K_AUX;
   C.A->H.word[a + 1] = pack2(np, first);
+  C.A->H.tag[a + 2] = K_AUX;                            // body list | parameter list
+  C.A->H.word[a + 2] = pack2(cdr_of(C, code), car_of(C, code));
   *out = mkv(kind, a);
   return true;
 }
@@ -665,26 +668,31 @@ __device__ CULI_COLD bool special_syntax_ok(const Ctx& C, uint32_t op, uint32_t 
 __device__ __forceinline__ int try_leaf(const Ctx& C, uint32_t xt, uint64_t xw, uint32_t dx, uint32_t env,
                                         uint64_t& steps, uint64_t fuel, uint32_t maxd, V* out, uint8_t* err) {
   if (!(xt & TAG_PROPER)) return 0;
+  // round 1 (independent loads): the head node, the first argument cell and — speculatively, since
+  // reader spines are contiguous (c.14) — the cell after it
+  uint32_t c1 = hi32(xw);
   uint32_t ht;
   uint64_t hw;
   ldnode(C, lo32(xw), ht, hw);
+  uint64_t cw1 = C.A->H.word[c1];                     // c1 == 0 reads the nil node: harmless
+  uint64_t cw2s = C.A->H.word[c1 + 1 < C.A->H.cap ? c1 + 1 : 0];
   if ((ht & KIND_MASK) != K_SYM || hw < N_SPECIALS || hw >= N_RESERVED) return 0;
   uint32_t op = (uint32_t)hw - N_SPECIALS;
   if (!((FAST_OPS >> op) & 1)) return 0;
-  uint32_t c1 = hi32(xw), argc = 0, n1 = 0, n2 = 0, t1 = 0, t2 = 0;
+  uint32_t argc = 0, n1 = 0, n2 = 0, t1 = 0, t2 = 0;
   uint64_t w1 = 0, w2 = 0;
   if (c1 != 0) {
-    uint64_t cw1 = nword(C, c1);
     n1 = lo32(cw1);
     uint32_t c2 = hi32(cw1);
+    uint64_t cw2 = c2 == c1 + 1 ? cw2s : C.A->H.word[c2];
+    // round 2: both argument nodes
     ldnode(C, n1, t1, w1);
+    if (c2 != 0) ldnode(C, lo32(cw2), t2, w2);
     if ((t1 & KIND_MASK) == K_CONS) return 0;
     argc = 1;
     if (c2 != 0) {
-      uint64_t cw2 = nword(C, c2);
       if (hi32(cw2) != 0) return 0;
       n2 = lo32(cw2);
-      ldnode(C, n2, t2, w2);
       if ((t2 & KIND_MASK) == K_CONS) return 0;
       argc = 2;
     }
@@ -730,6 +738,7 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32
   uint64_t steps = 0;
   uint8_t err = 0;
   uint4 k, ktop = make_uint4(0, 0, 0, 0);
+  uint4 hv = make_uint4(0, 0, 0, 0);      // the value being applied (copy of vs[base])
   bool kdirty = false;                      // ktop holds frame sp-1 not yet written to memory
 
 #define FAIL(e) do { err = (e); goto done; } while (0)
@@ -753,6 +762,7 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32
 
   if (APPLY && apply_mode) {
     base = 0;
+    hv = *VS(C, 0);
     cnt = apply_cnt;
     vtop = 1 + cnt;
     goto APPLY;
@@ -806,7 +816,8 @@ HEAD:
       if ((at & KIND_MASK) == K_CONS && leaf == 0 || cnt == 2) {   // spill to the general path
         if (__builtin_expect(!!(vtop + 3 >= vcap), 0)) FAIL(E_OOM);
         base = vtop;
-        *VS(C, base) = vpack(mkv(K_BUILTIN, hop), 0);
+        hv = vpack(mkv(K_BUILTIN, hop), 0);
+        *VS(C, base) = hv;
         if (cnt > 0) *VS(C, base + 1) = vpack(a0, 0);
         if (cnt > 1) *VS(C, base + 2) = vpack(a1, 0);
         if ((at & KIND_MASK) == K_CONS && leaf == 0) {
@@ -941,7 +952,8 @@ HEAD:
   // BUILTIN or CLOSURE: evaluate the args left to right at depth d+1 onto the V-stack
   if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
   base = vtop;
-  *VS(C, base) = vpack(v, 0);
+  hv = vpack(v, 0);
+  *VS(C, base) = hv;
   cnt = 0;
   // fallthrough
 ARGS:
@@ -972,18 +984,18 @@ ARGS:
   vtop = base + 1 + cnt;
   // fallthrough
 APPLY: {                                                        // apply vs[base] to cnt args
-  V h = vunpack(*VS(C, base));
+  V h = vunpack(hv);
   if (h.t == K_CLOSURE) {                                       // PAPER L456-460, c.4 CLOSURE
-    uint64_t cwd = nword(C, (uint32_t)h.w);
+    uint64_t cwd = nword(C, (uint32_t)h.w);                     // three independent loads
     uint64_t aux = nword(C, (uint32_t)h.w + 1);
+    uint64_t aux2 = nword(C, (uint32_t)h.w + 2);
     uint32_t np = lo32(aux);
     if (__builtin_expect(!!(np != cnt), 0)) FAIL(E_ARITY);
-    uint32_t code = lo32(cwd);
-    uint32_t body = cdr_of(C, code);
+    uint32_t body = lo32(aux2);
     if (np == 1) {
       VS(C, base + 1)->z = hi32(aux);
     } else {
-      uint32_t ps = car_of(C, code);
+      uint32_t ps = hi32(aux2);
       for (uint32_t i = 0; i < cnt; ++i) {
         uint64_t pw = nword(C, ps);
         VS(C, base + 1 + i)->z = (uint32_t)nword(C, lo32(pw));
@@ -1143,7 +1155,8 @@ PAR_NEXT: {
   V f = vunpack(*VS(C, pb + 1));
   base = pb + 2 + m;
   if (__builtin_expect(!!(base + 1 + m >= vcap), 0)) FAIL(E_OOM);
-  *VS(C, base) = vpack(f, 0);
+  hv = vpack(f, 0);
+  *VS(C, base) = hv;
   for (uint32_t j = 0; j < m; ++j) {
     uint4* cj = VS(C, pb + 2 + j);
     uint64_t wj = nword(C, cj->x);
@@ -1167,6 +1180,7 @@ RET:
   switch (kkind(k.w)) {
     case KF_ARGS:
       base = k.z; cnt = kcount(k.w);
+      hv = *VS(C, base);                                        // needed at APPLY: load early
       if (__builtin_expect(!!(base + 1 + cnt >= vcap), 0)) FAIL(E_OOM);
       *VS(C, base + 1 + cnt) = vpack(v, 0);
       ++cnt;
