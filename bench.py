@@ -334,24 +334,26 @@ def culi_arm(args):
     eval_s = statistics.mean(eval_ms) / 1e3
     clocks = clk.summary()
     prof = load_inst_profile(args.workload)
-    if args.workload == "C3":
-        # algorithmic bytes per element: read cons + float node, write cons + float node (9 B each)
-        traffic_alg = 36.0 * wl.units
-        ach = traffic_alg / eval_s / 1e9
-        roof = {"bound": "hbm", "achieved": ach, "peak": peaks["hbm_gbs"], "unit": "GB/s",
-                "frac": ach / peaks["hbm_gbs"], "traffic": prof.get("dram_bytes") if prof else None,
-                "peak_source": peak_src}
-    else:
-        sm_mhz = peaks.get("sm_max_mhz", 1965.0)
-        peak_inst = 148 * 4 * sm_mhz * 1e6 / 1e9          # warp instructions / ns -> G warp-inst/s
-        inst = prof.get("warp_inst_per_launch") if prof else None
-        ach = inst / eval_s / 1e9 if inst else None
-        roof = {"bound": "alu", "achieved": ach, "peak": peak_inst, "unit": "Gwarp-inst/s",
-                "frac": (ach / peak_inst) if ach else None,
-                "traffic": prof.get("dram_bytes") if prof else None,
-                "peak_source": "148 SMs x 4 SMSP x 1 warp-inst/clk x %.0f MHz (B200_PROFILING.md)" % sm_mhz,
-                "achieved_source": ("ncu smsp__inst_executed.sum of profiles/eval_inst_%s.json / live "
-                                    "eval-kernel time" % args.workload.lower()) if inst else None}
+    # The dominant kernel is the eval phase (culi_eval_kernel; for ||| workloads plus the fan-out element
+    # kernel).  It is bound by instruction issue/latency (an interpreter: plain int64/f64 ALU + branches),
+    # so the roofline is the warp-instruction issue rate; the HBM view is reported beside it.
+    sm_mhz = peaks.get("sm_max_mhz", 1965.0)
+    peak_inst = 148 * 4 * sm_mhz * 1e6 / 1e9          # G warp-instructions / s
+    inst = prof.get("warp_inst_per_launch") if prof else None
+    ach = inst / eval_s / 1e9 if inst else None
+    alg_bytes = {"C3": 36.0 * wl.units,                # per element: read cons + float, write cons + box
+                 "C2": 52.0 * len(shard_idx), "C1": 190.0 * len(shard_idx),
+                 "C4": 120.0 * len(shard_idx), "C5": 120.0 * len(shard_idx)}.get(args.workload, 0.0)
+    hbm_ach = alg_bytes / eval_s / 1e9
+    roof = {"bound": "alu", "achieved": ach, "peak": peak_inst, "unit": "Gwarp-inst/s",
+            "frac": (ach / peak_inst) if ach else None,
+            "traffic": prof.get("dram_bytes") if prof else None,
+            "peak_source": "148 SMs x 4 SMSP x 1 warp-inst/clk x %.0f MHz (B200_PROFILING.md, "
+                           "MEASURED_PEAKS sm_max_mhz)" % sm_mhz,
+            "achieved_source": ("ncu smsp__inst_executed.sum per launch (profiles/eval_inst_%s.json) / live "
+                                "eval-phase CUDA-event time" % args.workload.lower()) if inst else None,
+            "hbm_view": {"algorithmic_bytes": alg_bytes, "achieved_gbs": hbm_ach, "peak_gbs": peaks["hbm_gbs"],
+                         "frac": hbm_ach / peaks["hbm_gbs"], "peak_source": peak_src}}
 
     cpu = None
     if world == 1 and not args.no_cpu_baseline:
