@@ -12,6 +12,7 @@ from __future__ import annotations
 
 import dataclasses
 import hashlib
+import os
 
 import numpy as np
 
@@ -110,92 +111,127 @@ def c3(n: int = 1 << 20, seed: int = 1003) -> Workload:
     return Workload("C3", defs, forms, 1, n, seed)
 
 
-# ---- C4: macro-heavy control forms (BASELINE configs[3]) ------------------------------------------
-def c4(n: int = 262144, seed: int = 1004) -> Workload:
-    rng = _rng(seed)
+# ---- fast chunked drawing (C4, C5) ------------------------------------------------------------------
+# Big batches are generated in chunks of CHUNK forms; chunk c draws from PCG64(SeedSequence(seed).spawn)
+# [c], so the text is identical however many processes generate it.  Draws come from a pre-generated
+# block of uniforms: integers(lo, hi) = lo + floor(u * (hi - lo)).
+CHUNK = 1 << 15
 
+
+class _Draw:
+    def __init__(self, seq: np.random.SeedSequence):
+        self.g = np.random.Generator(np.random.PCG64(seq))
+        self.buf = self.g.random(1 << 16).tolist()
+        self.i = 0
+
+    def u(self) -> float:
+        if self.i >= len(self.buf):
+            self.buf = self.g.random(1 << 16).tolist()
+            self.i = 0
+        x = self.buf[self.i]
+        self.i += 1
+        return x
+
+    def int(self, lo: int, hi: int) -> int:          # uniform in [lo, hi)
+        return lo + int(self.u() * (hi - lo))
+
+
+def _chunked(fn, n: int, seed: int, procs: int | None = None) -> list[str]:
+    nchunks = (n + CHUNK - 1) // CHUNK
+    seqs = np.random.SeedSequence(seed).spawn(max(nchunks, 1))
+    jobs = [(fn, seqs[c], min(CHUNK, n - c * CHUNK)) for c in range(nchunks)]
+    if nchunks <= 2 or procs == 1:
+        parts = [_run_chunk(j) for j in jobs]
+    else:
+        import multiprocessing as mp
+        with mp.get_context("fork").Pool(procs or min(16, os.cpu_count() or 1)) as pool:
+            parts = pool.map(_run_chunk, jobs, chunksize=1)
+    return [line for part in parts for line in part]
+
+
+def _run_chunk(job):
+    fn, seq, count = job
+    r = _Draw(seq)
+    return [fn(r) for _ in range(count)]
+
+
+# ---- C4: macro-heavy control forms (BASELINE configs[3]) ------------------------------------------
+def _c4_form(r: _Draw) -> str:
     def leaf() -> str:
-        return str(int(rng.integers(-20, 21)))
+        return str(r.int(-20, 21))
 
     def I(d: int) -> str:
         if d == 0:
             return leaf()
-        u = rng.random()
+        u = r.u()
         if u < 0.35:
-            m = ["inc", "dec", "square"][int(rng.integers(0, 3))]
-            return "(%s %s)" % (m, I(d - 1))
+            return "(%s %s)" % (("inc", "dec", "square")[r.int(0, 3)], I(d - 1))
         if u < 0.60:
-            op = ["+", "-", "*"][int(rng.integers(0, 3))]
+            op = "+-*"[r.int(0, 3)]
             a = I(d - 1)
-            b = I(d - 1)
-            return "(%s %s %s)" % (op, a, b)
+            return "(%s %s %s)" % (op, a, I(d - 1))
         return leaf()
 
     def B(d: int) -> str:
-        cmp_ = ["<", "=", ">"]
         if d == 0:
-            c = cmp_[int(rng.integers(0, 3))]
+            c = "<=>"[r.int(0, 3)]
             a = leaf()
-            b = leaf()
-            return "(%s %s %s)" % (c, a, b)
-        if rng.random() < 0.3:
-            m = ["my-and", "my-or"][int(rng.integers(0, 2))]
+            return "(%s %s %s)" % (c, a, leaf())
+        if r.u() < 0.3:
+            m = ("my-and", "my-or")[r.int(0, 2)]
             a = B(d - 1)
-            b = B(d - 1)
-            return "(%s %s %s)" % (m, a, b)
-        c = cmp_[int(rng.integers(0, 3))]
+            return "(%s %s %s)" % (m, a, B(d - 1))
+        c = "<=>"[r.int(0, 3)]
         a = I(d - 1)
-        b = I(d - 1)
-        return "(%s %s %s)" % (c, a, b)
+        return "(%s %s %s)" % (c, a, I(d - 1))
 
-    lines = []
-    for _ in range(n):
-        k = int(rng.integers(0, 5))
-        if k == 0:
-            lines.append("(when %s %s)" % (B(2), I(2)))
-        elif k == 1:
-            lines.append("(unless %s %s)" % (B(2), I(2)))
-        elif k == 2:
-            b1 = B(2); i1 = I(2); b2 = B(2); i2 = I(2); i3 = I(2)
-            lines.append("(cond3 %s %s %s %s %s)" % (b1, i1, b2, i2, i3))
-        elif k == 3:
-            m = ["my-and", "my-or"][int(rng.integers(0, 2))]
-            a = B(2)
-            b = B(2)
-            lines.append("(%s %s %s)" % (m, a, b))
-        else:
-            m = ["inc", "dec", "square"][int(rng.integers(0, 3))]
-            lines.append("(%s %s)" % (m, I(2)))
+    k = r.int(0, 5)
+    if k == 0:
+        b = B(2)
+        return "(when %s %s)" % (b, I(2))
+    if k == 1:
+        b = B(2)
+        return "(unless %s %s)" % (b, I(2))
+    if k == 2:
+        b1 = B(2); i1 = I(2); b2 = B(2); i2 = I(2); i3 = I(2)
+        return "(cond3 %s %s %s %s %s)" % (b1, i1, b2, i2, i3)
+    if k == 3:
+        m = ("my-and", "my-or")[r.int(0, 2)]
+        a = B(2)
+        return "(%s %s %s)" % (m, a, B(2))
+    return "(%s %s)" % (("inc", "dec", "square")[r.int(0, 3)], I(2))
+
+
+def c4(n: int = 262144, seed: int = 1004, procs: int | None = None) -> Workload:
+    lines = _chunked(_c4_form, n, seed, procs)
     return Workload("C4", "\n".join(C4_MACROS) + "\n", "\n".join(lines) + "\n", n, n, seed)
 
 
 # ---- C5: 16M mixed forms (fib / fact / list ops), sharded over 1/2/4/8 GPUs --------------------------
-def _c5_list(rng: np.random.Generator, d: int) -> str:
-    if d == 0 or rng.random() < 0.4:
-        k = int(rng.integers(0, 9))
-        ints = [str(int(v)) for v in rng.integers(-50, 51, size=k)]
-        return "(list%s)" % "".join(" " + s for s in ints)
-    c = int(rng.integers(0, 4))
+def _c5_list(r: _Draw, d: int) -> str:
+    if d == 0 or r.u() < 0.4:
+        k = r.int(0, 9)
+        return "(list%s)" % "".join(" %d" % r.int(-50, 51) for _ in range(k))
+    c = r.int(0, 4)
     if c == 0:
-        i = str(int(rng.integers(-50, 51)))
-        return "(cons %s %s)" % (i, _c5_list(rng, d - 1))
+        i = r.int(-50, 51)
+        return "(cons %d %s)" % (i, _c5_list(r, d - 1))
     if c == 1:
-        return "(cdr %s)" % _c5_list(rng, d - 1)
+        return "(cdr %s)" % _c5_list(r, d - 1)
     if c == 2:
-        return "(reverse %s)" % _c5_list(rng, d - 1)
-    a = _c5_list(rng, d - 1)
-    b = _c5_list(rng, d - 1)
-    return "(append %s %s)" % (a, b)
+        return "(reverse %s)" % _c5_list(r, d - 1)
+    a = _c5_list(r, d - 1)
+    return "(append %s %s)" % (a, _c5_list(r, d - 1))
 
 
-def c5_form(rng: np.random.Generator) -> str:
-    kind = int(rng.integers(0, 3))
+def _c5_form(r: _Draw) -> str:
+    kind = r.int(0, 3)
     if kind == 0:
-        return "(fib %d)" % int(rng.integers(5, 16))
+        return "(fib %d)" % r.int(5, 16)
     if kind == 1:
-        return "(fact %d)" % int(rng.integers(1, 21))
-    root = int(rng.integers(0, 6))
-    L = _c5_list(rng, 2)
+        return "(fact %d)" % r.int(1, 21)
+    root = r.int(0, 6)
+    L = _c5_list(r, 2)
     if root == 0:
         return "(length %s)" % L
     if root == 1:
@@ -203,16 +239,15 @@ def c5_form(rng: np.random.Generator) -> str:
     if root == 2:
         return "(sum-list %s)" % L
     if root == 3:
-        return "(nth %d %s)" % (int(rng.integers(0, 9)), L)
+        return "(nth %d %s)" % (r.int(0, 9), L)
     if root == 4:
         return L
-    L2 = L if rng.random() < 0.5 else _c5_list(rng, 2)
+    L2 = L if r.u() < 0.5 else _c5_list(r, 2)
     return "(equal %s %s)" % (L, L2)
 
 
-def c5(n: int = 16777216, seed: int = 1005) -> Workload:
-    rng = _rng(seed)
-    lines = [c5_form(rng) for _ in range(n)]
+def c5(n: int = 16777216, seed: int = 1005, procs: int | None = None) -> Workload:
+    lines = _chunked(_c5_form, n, seed, procs)
     defs = "\n".join([FIB_DEF, FACT_DEF, SUM_LIST_DEF]) + "\n"
     return Workload("C5", defs, "\n".join(lines) + "\n", n, n, seed)
 

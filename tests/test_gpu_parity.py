@@ -36,7 +36,7 @@ def run_both(culi, oracle_mod, defs, forms, ctx_kw=None, oracle_kw=None):
     s = oracle_mod.Session(**(oracle_kw or {}))
     if defs:
         s.define(defs)
-    o = s.eval(forms)
+    o = s.eval_batch(forms, nthreads=os.cpu_count() or 1).results
     return res.printed(), res.steps(), o
 
 
@@ -136,14 +136,19 @@ def test_c3_full(culi, oracle_mod):
     assert_parity(culi, oracle_mod, wl.defs, wl.forms, ctx_kw=dict(heap_nodes=1 << 26))
 
 
-def test_c4(culi, oracle_mod):
-    wl = W.c4(20000)
-    assert_parity(culi, oracle_mod, wl.defs, wl.forms)
+def test_c4_full(culi, oracle_mod):
+    wl = W.c4()                                   # configs[3] at full size: 262,144 forms
+    assert_parity(culi, oracle_mod, wl.defs, wl.forms, ctx_kw=dict(heap_nodes=1 << 27))
 
 
 def test_c5_small(culi, oracle_mod):
     wl = W.c5(20000)
     assert_parity(culi, oracle_mod, wl.defs, wl.forms)
+
+
+def test_c5_large(culi, oracle_mod):
+    wl = W.c5(1 << 18)                            # 262,144 mixed forms, every one checked
+    assert_parity(culi, oracle_mod, wl.defs, wl.forms, ctx_kw=dict(heap_nodes=1 << 27))
 
 
 def test_c0(culi, oracle_mod):
