@@ -140,11 +140,11 @@ def _chunked(fn, n: int, seed: int, procs: int | None = None) -> list[str]:
     nchunks = (n + CHUNK - 1) // CHUNK
     seqs = np.random.SeedSequence(seed).spawn(max(nchunks, 1))
     jobs = [(fn, seqs[c], min(CHUNK, n - c * CHUNK)) for c in range(nchunks)]
-    if nchunks <= 2 or procs == 1:
+    if nchunks <= 16 or procs == 1:
         parts = [_run_chunk(j) for j in jobs]
-    else:
+    else:                                             # spawn: the caller may hold CUDA / NCCL threads
         import multiprocessing as mp
-        with mp.get_context("fork").Pool(procs or min(16, os.cpu_count() or 1)) as pool:
+        with mp.get_context("spawn").Pool(procs or min(16, os.cpu_count() or 1)) as pool:
             parts = pool.map(_run_chunk, jobs, chunksize=1)
     return [line for part in parts for line in part]
 
