@@ -40,6 +40,16 @@ WORKLOADS = {
 SCALING = {"C1": "weak", "C2": "weak", "C3": "replicas", "C4": "weak", "C5": "strong"}
 
 
+def bench_config(workload: str, world: int) -> dict:
+    """The `config` object shared by the culi arm and the reference (oracle) arm."""
+    idx = {"C1": 0, "C2": 1, "C3": 2, "C4": 3, "C5": 4}[workload]
+    what = {"C1": "1,024 integer arithmetic forms", "C2": "65,536 (fib n) forms, n in 15..22",
+            "C3": "(||| 1048576 f xs), closure + let + float", "C4": "262,144 macro forms",
+            "C5": "16.8M mixed forms"}[workload]
+    return {"workload": "%s (BASELINE configs[%d]): %s" % (workload, idx, what),
+            "parallelism": "dp%d" % world, "l2": "flushed between timed steps (512 MB write)"}
+
+
 def parse():
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
@@ -154,8 +164,7 @@ def reference_arm(args):
         "ms_per_step": 1e3 * t / len(times), "higher_is_better": True, "scaling": SCALING[args.workload],
         "vs_baseline": None, "dtype": "int64+f64", "data": "synthetic",
         "eval_steps_per_sec": steps_tot / t,
-        "config": {"workload": "%s (configs[%d])" % (args.workload, int(args.workload[1]) - 1 if args.workload != "C0" else 0),
-                   "sample": desc},
+        "config": dict(bench_config(args.workload, args.gpus), sample=desc),
         "cpu_baseline": {"value": value, "unit": "forms/s", "cores": threads, "kind": "oracle",
                          "sample": desc},
         "e2e": {"value": value, "unit": "forms/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
@@ -369,14 +378,8 @@ def culi_arm(args):
         "scaling": SCALING[args.workload] if world > 1 else "weak", "vs_baseline": None,
         "dtype": "int64+f64", "data": "synthetic",
         "eval_steps_per_sec": steps_per_sec,
-        "config": {"workload": "%s (BASELINE configs[%d]): %s" % (
-                       args.workload, {"C1": 0, "C2": 1, "C3": 2, "C4": 3, "C5": 4}.get(args.workload, 0),
-                       {"C1": "1,024 integer arithmetic forms", "C2": "65,536 (fib n), n in 15..22",
-                        "C3": "(||| 1048576 f xs), closure+let+float", "C4": "262,144 macro forms",
-                        "C5": "16.8M mixed forms"}[args.workload]),
-                   "forms_per_gpu": len(shard_idx), "units_per_gpu": units_rank,
-                   "parallelism": "dp%d" % world, "l2": "flushed between timed steps (512 MB write)",
-                   "binning": not (args.flags & 1)},
+        "config": dict(bench_config(args.workload, world), forms_per_gpu=len(shard_idx),
+                       units_per_gpu=units_rank, binning=not (args.flags & 1)),
         "gpu_launches": kernels * args.steps,
         "phases_ms": {"dispatch": statistics.mean(disp_ms), "eval": statistics.mean(eval_ms),
                       "export": statistics.mean(exp_ms)},

@@ -1,0 +1,24 @@
+"""Small batches over every language feature, run under compute-sanitizer (tools/sanitize.sh)."""
+import os
+import sys
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+from paper_conf_cluster_subdbn18_b200 import culi, workloads as W  # noqa: E402
+
+culi.load()
+defs = "\n".join([W.FIB_DEF, W.FACT_DEF, W.SUM_DEF, W.SUM_LIST_DEF] + W.C4_MACROS + W.C3_DEFS_HEAD +
+                 ["(define xs '(0.5 1.5 -2.0 3.25))"])
+edge = [l.split("\t")[0] for l in open(os.path.join(ROOT, "tests/golden/edge_cases.tsv"))
+        if l.strip() and not l.startswith("#")]
+forms = "\n".join(edge + W.c1(64).form_lines() + W.c2(64, lo=3, hi=9).form_lines() +
+                  W.c4(256).form_lines() + W.c5(512).form_lines() + ["(||| 4 f xs)", "(||| 3 + '(1 2 3) '(4 5 6))"])
+ctx = culi.Context(slots=148 * 128, heap_nodes=1 << 22, vstack_entries=1024)
+ctx.define(defs)
+for flags in (0, culi.CULI_F_NO_BINNING | culi.CULI_F_NO_FANOUT):
+    c2 = culi.Context(slots=148 * 128, heap_nodes=1 << 22, vstack_entries=1024, flags=flags)
+    c2.define(defs)
+    r = c2.eval_batch(forms)
+    print(len(r), r.totals())
+    c2.close()
+print("done")
