@@ -125,6 +125,7 @@ void culi_shutdown(culi_ctx* c) {
   cudaFree(c->npend);
   cudaFree(c->nfallback);
   c->fallback.release();
+  c->wide.release();
   c->roots.release(); c->keys.release(); c->keys_alt.release(); c->perm.release();
   c->perm_alt.release(); c->rtag.release(); c->rerr.release(); c->dtemp.release();
   c->rsteps.release(); c->rword.release(); c->payload.release();
@@ -177,6 +178,7 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.maxdesc = c->maxdesc;
   A.fallback = c->fallback.p;
   A.nfallback = c->nfallback;
+  A.wide = (!define_mode && c->batch_has_wide) ? c->wide.p : nullptr;
   A.payload = c->payload.p;
   A.pcount = c->pcount;
   A.pcap = c->payload.n;
@@ -320,15 +322,30 @@ static int prepare_batch(culi_ctx* c, const Image& img) {
   c->batch_forms = nf;
   c->batch_strings = img.strings;
   CK(c->fallback.ensure(std::max<size_t>(c->maxdesc, 1)));
-  c->batch_has_par = false;                          // does any form start with the ||| symbol?
-  for (uint32_t r : img.roots) {
+  // does any form start with the ||| symbol (a6), or have >= WIDE_MIN arguments (wide forms, K12)?
+  c->batch_has_par = false;
+  c->batch_has_wide = false;
+  std::vector<uint32_t> wide;
+  for (uint32_t f = 0; f < nf; ++f) {
+    uint32_t r = img.roots[f];
     if (r < IMG_FIRST || (img.tag[r - IMG_FIRST] & KIND_MASK) != K_CONS) continue;
-    uint32_t h = (uint32_t)img.word[r - IMG_FIRST];
+    uint64_t rw = img.word[r - IMG_FIRST];
+    uint32_t h = (uint32_t)rw;
     if (h >= IMG_FIRST && (img.tag[h - IMG_FIRST] & KIND_MASK) == K_SYM &&
-        img.word[h - IMG_FIRST] == N_SPECIALS + BI_PAR) {
+        img.word[h - IMG_FIRST] == N_SPECIALS + BI_PAR)
       c->batch_has_par = true;
-      break;
+    uint32_t nargs = 0;
+    for (uint32_t q = (uint32_t)(rw >> 32); q >= IMG_FIRST; q = (uint32_t)(img.word[q - IMG_FIRST] >> 32)) ++nargs;
+    if (nargs >= WIDE_MIN) {
+      if (wide.empty()) wide.assign(nf, 0);
+      wide[f] = nargs;
+      c->batch_has_wide = true;
     }
+  }
+  if (c->batch_has_wide) {
+    CK(c->wide.ensure(nf));
+    CK(cudaMemcpyAsync(c->wide.p, wide.data(), nf * 4, cudaMemcpyHostToDevice, c->stream));
+    c->batch_has_par = true;                         // the fan-out kernels handle both
   }
   return CULI_OK;
 }

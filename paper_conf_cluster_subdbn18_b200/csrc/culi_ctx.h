@@ -80,6 +80,8 @@ struct culi_ctx {
   uint32_t* nfallback = nullptr;
   DevBuf<uint32_t> fallback;
   bool batch_has_par = false;
+  bool batch_has_wide = false;
+  DevBuf<uint32_t> wide;
   // uploaded batch (culi_upload)
   bool have_batch = false;
   uint64_t batch_nodes = 0;

@@ -65,6 +65,7 @@ struct EvalArgs {
   uint4* payload;              // export tokens (flat ||| results are written by the fan-out stage)
   unsigned long long* pcount;
   unsigned long long pcap;
+  const uint32_t* wide;        // per form: argument count of a wide top-level form, else 0 (host scan)
   uint32_t code_lo, code_n;    // node range staged in shared memory (persistent code segment)
   uint32_t gst;                // global-frame entries staged in shared memory
 };
@@ -72,8 +73,14 @@ struct EvalArgs {
 // One top-level (||| n f l1 .. lm) form whose arguments have been evaluated.
 constexpr uint32_t FANOUT_MAXM = 6;
 constexpr uint8_t E_PENDING = 0xfe;          // internal: record filled in by the fan-out finalizer
+// FAN_PAR: (||| n f l1..lm) elements.  Wide forms (>= WIDE_MIN arguments, K12 "per warp for wide forms"):
+// FAN_DATA (h a1..an) with h not applicable -> list (h v1..vn); FAN_LIST (list a1..an); FAN_FOLD (+ or *
+// a1..an, op in m).  For wide kinds element i evaluates argument i (depth 2); heads[0] = first arg cell.
+enum FanKind : uint32_t { FAN_PAR = 0, FAN_DATA = 1, FAN_LIST = 2, FAN_FOLD = 3 };
+constexpr uint32_t WIDE_MIN = 64;
 struct FanDesc {
-  uint32_t form, n, m, spine;                // spine: 2n nodes (n cells, then n box slots)
+  uint32_t form, n, m, spine;                // n: result cells; spine: 2n nodes (n cells, then n boxes)
+  uint32_t kind, nelem;                      // FanKind; elements to evaluate
   uint32_t ftag, depth;
   uint64_t fword;
   uint64_t steps0;                           // canonical steps before the first element

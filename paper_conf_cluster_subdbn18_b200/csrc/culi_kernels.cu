@@ -195,6 +195,29 @@ __global__ void __launch_bounds__(128, 4) culi_fanout_kernel(const __grid_consta
     uint64_t budget = A.fuel - D->steps0;
     unsigned long long my_steps = 0;
     uint32_t bad = 0, nonflat = 0;
+    if (D->kind != FAN_PAR) {                         // wide form: element i = argument i (depth 2)
+      uint32_t ne = D->nelem, first = D->kind == FAN_DATA ? 1u : 0u, c1 = D->heads[0];
+      for (uint32_t i = slot; i < ne; i += nthreads) {
+        uint32_t c = c1 + i;
+        if ((uint64_t)c >= top) { bad |= 1; continue; }
+        uint32_t tc = H.tag[c];
+        uint64_t wc = H.word[c];
+        if ((tc & KIND_MASK) != K_CONS || hi32(wc) != (i + 1 < ne ? c + 1 : 0u)) { bad |= 1; continue; }
+        FormOut o = eval_form<false, false>(C, lo32(wc), D->form, 0, 0, budget, D->depth + 1);
+        if (o.err) { bad |= 2; continue; }
+        my_steps += o.steps;
+        if (D->kind == FAN_FOLD) {                   // raw value record for the finalizer's fold
+          H.tag[spine + i] = (uint8_t)o.t;
+          H.word[spine + i] = o.w;
+          continue;
+        }
+        nonflat |= (o.t == K_CONS);
+        uint32_t j = first + i;
+        uint32_t ca = box_into(H, mkv(o.t, o.w), spine + n + j);
+        H.tag[spine + j] = K_CONS | TAG_PROPER;
+        H.word[spine + j] = pack2(ca, j + 1 < n ? spine + j + 1 : 0);
+      }
+    } else
     for (uint32_t i = slot; i < n; i += nthreads) {
       bool ok = true;
       *VS(C, 0) = vpack(f, 0);
@@ -242,6 +265,21 @@ __global__ void culi_fanout_finalize_kernel(const __grid_constant__ EvalArgs A) 
     }
     A.rerr[D->form] = 0;
     A.rsteps[D->form] = steps;
+    if (D->kind == FAN_FOLD) {                        // (+ / * a1 .. an): types, then left fold (c.6)
+      bool type_err = false;
+      for (uint32_t i = 0; i < D->nelem; ++i) type_err |= !is_num(A.H.tag[D->spine + i]);
+      if (type_err) {
+        A.rtag[D->form] = K_ERROR;
+        A.rerr[D->form] = E_TYPE;
+        A.rword[D->form] = 0;
+        continue;
+      }
+      V acc = mkv(A.H.tag[D->spine], A.H.word[D->spine]);
+      for (uint32_t i = 1; i < D->nelem; ++i) fold_step(D->m, acc, mkv(A.H.tag[D->spine + i], A.H.word[D->spine + i]));
+      A.rtag[D->form] = (uint8_t)acc.t;
+      A.rword[D->form] = acc.w;
+      continue;
+    }
     if (!D->nonflat && A.payload) {
       // a flat list (no element is a cons): 2n+1 tokens written in parallel by culi_flat_export_kernel
       unsigned long long ntok = 2ull * D->n + 1;

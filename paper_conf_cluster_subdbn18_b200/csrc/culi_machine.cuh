@@ -727,12 +727,12 @@ struct FormOut {
 //   (||| ...) form (depth 1) — one fan-out element (c.7); `budget` = fuel left after the ||| arguments.
 template <bool FANOUT, bool APPLY>
 __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32_t form, int apply_mode,
-                                             uint32_t apply_cnt, uint64_t fuel) {
+                                             uint32_t apply_cnt, uint64_t fuel, uint32_t d0 = 1) {
   const DevHeap& H = C.A->H;
   const uint32_t kcap = C.A->kcap, vcap = C.A->vcap, maxd = C.A->max_depth;
   const bool fanout = FANOUT && !APPLY && C.A->fanout;
   V v = mkv(K_NIL, 0), a0 = mkv(K_NIL, 0), a1 = mkv(K_NIL, 0);
-  uint32_t x = root, t = 0, env = 0, d = 1, cur = 0, base = 0, cnt = 0, sp = 0, vtop = 0;
+  uint32_t x = root, t = 0, env = 0, d = d0, cur = 0, base = 0, cnt = 0, sp = 0, vtop = 0;
   uint32_t a = 0, at = 0, nxt = 0, kd = 0, hop = 0;
   uint64_t w = 0, aw = 0, w0 = 0;
   uint64_t steps = 0;
@@ -796,6 +796,44 @@ EVAL_VALUE:
 
   // ======================================================== head value v, unevaluated args `cur`
 HEAD:
+  if (FANOUT && !APPLY && fanout && sp == 0 && d == 1 && C.A->wide && C.A->wide[form] >= WIDE_MIN) {
+    // a wide top-level form (K12): evaluate its arguments one per thread in the fan-out kernel
+    uint32_t kind = 0xffu, op = 0;
+    if (v.t == K_BUILTIN && v.w == BI_LIST) kind = FAN_LIST;
+    else if (v.t == K_BUILTIN && (v.w == BI_ADD || v.w == BI_MUL)) { kind = FAN_FOLD; op = (uint32_t)v.w; }
+    else if (v.t != K_BUILTIN && v.t != K_SPECIAL && v.t != K_CLOSURE && v.t != K_MACRO) kind = FAN_DATA;
+    if (kind != 0xffu) {
+      uint32_t slot = atomicAdd(C.A->npend, 1u);
+      if (slot < C.A->maxdesc) {
+        uint32_t nargs = C.A->wide[form];
+        uint32_t ncells = kind == FAN_DATA ? nargs + 1 : nargs, spine;
+        if (__builtin_expect(!!(!heap_alloc(H, kind == FAN_FOLD ? nargs : 2 * ncells, &spine)), 0)) FAIL(E_OOM);
+        if (kind == FAN_DATA) {                                   // cell 0 holds the head value
+          uint32_t ca = box_into(H, v, spine + ncells);
+          H.tag[spine] = K_CONS | TAG_PROPER;
+          H.word[spine] = pack2(ca, ncells > 1 ? spine + 1 : 0);
+        }
+        FanDesc* D = C.A->desc + slot;
+        D->form = form;
+        D->n = ncells;
+        D->m = op;
+        D->kind = kind;
+        D->nelem = nargs;
+        D->spine = spine;
+        D->ftag = v.t;
+        D->depth = d;
+        D->fword = v.w;
+        D->steps0 = steps;
+        D->top = atomicAdd(H.top, 0ull);
+        D->heads[0] = cur;
+        D->total = 0;
+        D->bad = 0;
+        D->nonflat = 0;
+        err = E_PENDING;
+        goto done;
+      }
+    }
+  }
   if (v.t == K_BUILTIN && ((FAST_OPS >> v.w) & 1)) {            // register fast path
     hop = (uint32_t)v.w;
     cnt = 0;
@@ -1028,6 +1066,8 @@ APPLY: {                                                        // apply vs[base
         D->form = form;
         D->n = n;
         D->m = cnt - 2;
+        D->kind = FAN_PAR;
+        D->nelem = n;
         D->spine = spine;
         D->ftag = f.t;
         D->depth = d;
@@ -1037,6 +1077,7 @@ APPLY: {                                                        // apply vs[base
         for (uint32_t j = 0; j < cnt - 2; ++j) D->heads[j] = (uint32_t)arg(C, base, 2 + j).w;
         D->total = 0;
         D->bad = 0;
+        D->nonflat = 0;
         err = E_PENDING;
         goto done;
       }

@@ -265,3 +265,28 @@ def test_upload_eval_fetch_repeatable(culi, oracle_mod):
     ms, kernels, high = ctx.last_timing()
     assert kernels >= 2 and all(m >= 0 for m in ms)
     ctx.release(h)
+
+
+def test_wide_forms(culi, oracle_mod):
+    """Top-level forms with >= 64 arguments take the wide path (arguments one per thread, K12)."""
+    rnd = random.Random(77)
+    forms = []
+    for n in (64, 65, 100, 257, 1000):
+        forms.append("(list %s)" % " ".join(str(rnd.randint(-9, 9)) for _ in range(n)))
+        forms.append("(+ %s)" % " ".join(str(rnd.randint(-2**62, 2**62)) for _ in range(n)))
+        forms.append("(* %s)" % " ".join(str(rnd.randint(-3, 3)) for _ in range(n)))
+        forms.append("(+ %s)" % " ".join(repr(rnd.uniform(-1e3, 1e3)) if rnd.random() < 0.5 else str(rnd.randint(-9, 9))
+                                         for _ in range(n)))       # mixed int/float: sequential left fold
+        forms.append("(%d %s)" % (n, " ".join("(fib %d)" % rnd.randint(0, 12) for _ in range(n))))
+        forms.append("(foo %s)" % " ".join(rnd.choice(["x", "'y", "(fact 5)", "nil", "T", "\"s\""]) for _ in range(n)))
+        forms.append("(list %s)" % " ".join("(list %d (+ %d 1))" % (i, i) for i in range(n)))
+    forms.append("(list %s (car 5) %s)" % (" ".join(["1"] * 40), " ".join(["(fib 10)"] * 40)))   # error mid-way
+    forms.append("(+ %s 'a %s)" % (" ".join(["1"] * 40), " ".join(["2"] * 40)))                    # TYPE after all args
+    forms.append("(list %s)" % " ".join(["(sum 400)"] * 70))                                       # DEPTH inside
+    assert_parity(culi, oracle_mod, DEFS, "\n".join(forms))
+
+
+def test_wide_forms_fuel(culi, oracle_mod):
+    forms = "(list %s)" % " ".join(["(fib 8)"] * 100)
+    for fuel in (500, 6000, 6800, 100000):
+        assert_parity(culi, oracle_mod, DEFS, forms, ctx_kw=dict(fuel=fuel), oracle_kw=dict(fuel=fuel))
