@@ -159,6 +159,10 @@ const char* culi_error_name(uint8_t err);
 /* Device time in ms of the phases of the last eval call: [0] dispatch, [1] eval, [2] export; and the
  * number of kernels launched by that call.  Heap high-water mark in nodes. */
 int culi_last_timing(const culi_ctx* ctx, float* ms3, uint32_t* kernels, uint64_t* heap_high);
+/* Path statistics of the last fetched batch: forms handled by the fan-out kernels (top-level ||| forms
+ * and wide forms) and, of those, forms re-evaluated sequentially (an element error,
+ * fuel overflow, or a short / non-contiguous list). */
+int culi_last_stats(const culi_ctx* ctx, uint32_t* fanout_forms, uint32_t* fallback_forms);
 
 #ifdef __cplusplus
 }

@@ -382,7 +382,8 @@ static int fetch(culi_ctx* c, culi_results** out) {
   for (int attempt = 0; attempt < 4; ++attempt) {
     int flags[8];
     unsigned long long pc = 0, top = 0;
-    uint32_t nfb = 0;
+    uint32_t nfb = 0, npend = 0;
+    CK(cudaMemcpyAsync(&npend, c->npend, 4, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(flags, c->flags, sizeof flags, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(&pc, c->pcount, 8, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(&top, c->H.top, 8, cudaMemcpyDeviceToHost, c->stream));
@@ -390,7 +391,12 @@ static int fetch(culi_ctx* c, culi_results** out) {
     CK(cudaStreamSynchronize(c->stream));
     c->heap_high = std::max<uint64_t>(c->heap_high, std::min<unsigned long long>(top, c->H.cap));
     if (flags[0] || flags[4]) return CULI_E_HEAP_FULL;
+    if (attempt == 0) {
+      c->last_fanout = (c->batch_has_par && !(c->opts.flags & CULI_F_NO_FANOUT)) ? std::min(npend, c->maxdesc) : 0;
+      c->last_fallback = 0;
+    }
     if (nfb && !flags[3]) {
+      c->last_fallback += nfb;
       int rc = rerun_fallback(c, nfb);
       if (rc) return rc;
       continue;
@@ -548,6 +554,13 @@ int culi_results_totals(const culi_results* r, uint64_t* total_steps, uint32_t* 
 }
 
 void culi_results_free(culi_results* r) { delete r; }
+
+int culi_last_stats(const culi_ctx* c, uint32_t* fanout_forms, uint32_t* fallback_forms) {
+  if (!c) return CULI_E_ARG;
+  if (fanout_forms) *fanout_forms = c->last_fanout;
+  if (fallback_forms) *fallback_forms = c->last_fallback;
+  return CULI_OK;
+}
 
 int culi_last_timing(const culi_ctx* c, float* ms3, uint32_t* kernels, uint64_t* heap_high) {
   if (!c) return CULI_E_ARG;

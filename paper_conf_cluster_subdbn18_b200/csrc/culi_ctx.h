@@ -81,6 +81,7 @@ struct culi_ctx {
   DevBuf<uint32_t> fallback;
   bool batch_has_par = false;
   bool batch_has_wide = false;
+  uint32_t last_fanout = 0, last_fallback = 0;
   DevBuf<uint32_t> wide;
   // uploaded batch (culi_upload)
   bool have_batch = false;

@@ -29,6 +29,7 @@ SYMBOLS = [
     "culi_result_int", "culi_result_float", "culi_print", "culi_results_totals", "culi_results_free",
     "culi_env_export", "culi_env_import", "culi_results_serialize", "culi_results_merge",
     "culi_status_string", "culi_error_name", "culi_last_timing", "culi_records_device",
+    "culi_last_stats",
 ]
 
 
@@ -86,6 +87,7 @@ def load(path: str = LIB_PATH) -> ctypes.CDLL:
         "culi_error_name": (ctypes.c_char_p, [ctypes.c_uint8]),
         "culi_last_timing": (I, [P, pp(ctypes.c_float), pp(U32), pp(U64)]),
         "culi_records_device": (I, [P, P, SZ, pp(SZ)]),
+        "culi_last_stats": (I, [P, pp(U32), pp(U32)]),
     }
     for name, (res, args) in sig.items():
         fn = getattr(L, name)
@@ -282,6 +284,12 @@ class Context:
         h = ctypes.c_uint64()
         _check(load().culi_last_timing(self._p, ms, ctypes.byref(k), ctypes.byref(h)), "culi_last_timing")
         return list(ms), k.value, h.value
+
+    def last_stats(self) -> tuple[int, int]:
+        """(forms handled by the fan-out kernels, of which re-evaluated sequentially) of the last batch."""
+        a, b = ctypes.c_uint32(), ctypes.c_uint32()
+        _check(load().culi_last_stats(self._p, ctypes.byref(a), ctypes.byref(b)), "culi_last_stats")
+        return a.value, b.value
 
     def records_device(self, dev_ptr: int | None, cap: int = 0) -> int:
         need = ctypes.c_size_t(0)

@@ -134,6 +134,10 @@ def test_c3_small(culi, oracle_mod):
 def test_c3_full(culi, oracle_mod):
     wl = W.c3()
     assert_parity(culi, oracle_mod, wl.defs, wl.forms, ctx_kw=dict(heap_nodes=1 << 26))
+    ctx = culi.Context(**{**SMALL, "heap_nodes": 1 << 26})
+    ctx.define(wl.defs)
+    ctx.eval_batch(wl.forms)
+    assert ctx.last_stats() == (1, 0)                 # the ||| form fanned out, no fallback
 
 
 def test_c4_full(culi, oracle_mod):
@@ -283,7 +287,14 @@ def test_wide_forms(culi, oracle_mod):
     forms.append("(list %s (car 5) %s)" % (" ".join(["1"] * 40), " ".join(["(fib 10)"] * 40)))   # error mid-way
     forms.append("(+ %s 'a %s)" % (" ".join(["1"] * 40), " ".join(["2"] * 40)))                    # TYPE after all args
     forms.append("(list %s)" % " ".join(["(sum 400)"] * 70))                                       # DEPTH inside
-    assert_parity(culi, oracle_mod, DEFS, "\n".join(forms))
+    text = "\n".join(forms)
+    assert_parity(culi, oracle_mod, DEFS, text)
+    ctx = culi.Context(**SMALL)
+    ctx.define(DEFS)
+    ctx.eval_batch(text)
+    fan, fb = ctx.last_stats()
+    assert fan == 5 * 7 + 3 and fb == 2, (fan, fb)    # every form above is wide (data/list/fold);
+    # (foo ...) wide forms too; the mid-way error and the DEPTH form fall back, the TYPE fold does not
 
 
 def test_wide_forms_fuel(culi, oracle_mod):
