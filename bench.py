@@ -308,7 +308,7 @@ def culi_arm(args):
     steps_per_sec = steps_all * args.steps / t_max
 
     # ---- e2e: the public C-ABI with host buffers (H2D of the image, D2H of records + payload)
-    h2d = img.nnodes * 9 + img.nforms * 4
+    h2d = img.pin()                      # inputs DMA'd from pinned host memory (bytes per step)
     e2e_ms, d2h = [], 0
     ctx.release(h)
     for k in range(args.e2e_steps):
@@ -317,7 +317,7 @@ def culi_arm(args):
             dist.barrier()
         a.record(stream)
         r = ctx.eval_batch(img)
-        d2h = len(r.serialize())
+        d2h = r.wire_bytes()
         if world > 1:
             from paper_conf_cluster_subdbn18_b200 import dist as D
             D.gather_results(r, wl.nforms)

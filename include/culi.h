@@ -93,6 +93,9 @@ void culi_shutdown(culi_ctx* ctx);
  * *err_offset (if non-NULL) receives the byte offset of the offending character / opening paren. */
 int culi_read(culi_ctx* ctx, const char* text, size_t len, culi_image** out, size_t* err_offset);
 uint32_t culi_image_nforms(const culi_image* img);
+/* Page-lock the image's host arrays (cudaHostRegister) so that uploads DMA them from pinned memory.
+ * Idempotent; undone by culi_image_free.  *h2d_bytes (if non-NULL) = bytes an upload of it copies. */
+int culi_image_pin(culi_image* img, uint64_t* h2d_bytes);
 uint64_t culi_image_nnodes(const culi_image* img);
 void culi_image_free(culi_image* img);
 
@@ -133,6 +136,8 @@ int culi_print(const culi_results* r, uint32_t i, char* buf, size_t cap, size_t*
 /* Sum of steps over all forms, and the number of forms with err != 0. */
 int culi_results_totals(const culi_results* r, uint64_t* total_steps, uint32_t* n_errors);
 void culi_results_free(culi_results* r);
+/* Bytes the fetch of these results copied device -> host (records + serialized value tokens). */
+int culi_results_wire_bytes(const culi_results* r, uint64_t* d2h_bytes);
 
 /* ---- distributed hooks ------------------------------------------------------------------
  * The collective itself is issued by the caller (torch.distributed NCCL broadcast / all_gather) on a

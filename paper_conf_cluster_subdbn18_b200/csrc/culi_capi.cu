@@ -148,6 +148,22 @@ uint32_t culi_image_nforms(const culi_image* im) { return im ? (uint32_t)im->img
 uint64_t culi_image_nnodes(const culi_image* im) { return im ? im->img.tag.size() : 0; }
 void culi_image_free(culi_image* im) { delete im; }
 
+int culi_image_pin(culi_image* im, uint64_t* h2d_bytes) {
+  if (!im) return CULI_E_ARG;
+  const Image& g = im->img;
+  if (h2d_bytes) *h2d_bytes = g.tag.size() * 9 + g.roots.size() * 4 + g.strings.size();
+  if (im->pinned) return CULI_OK;
+  bool ok = true;
+  if (!g.tag.empty())
+    ok &= cudaHostRegister((void*)g.tag.data(), g.tag.size(), cudaHostRegisterDefault) == cudaSuccess;
+  if (!g.word.empty())
+    ok &= cudaHostRegister((void*)g.word.data(), g.word.size() * 8, cudaHostRegisterDefault) == cudaSuccess;
+  if (!g.roots.empty())
+    ok &= cudaHostRegister((void*)g.roots.data(), g.roots.size() * 4, cudaHostRegisterDefault) == cudaSuccess;
+  im->pinned = true;                                 // partial registrations are undone by the destructor
+  return ok ? CULI_OK : CULI_E_CUDA;
+}
+
 }  // extern "C"
 
 // ---- internal helpers ------------------------------------------------------------------------------
@@ -414,22 +430,17 @@ static int fetch(culi_ctx* c, culi_results** out) {
     }
     culi_results* r = new (std::nothrow) culi_results;
     if (!r) return CULI_E_ARG;
-    r->r.rec.resize(nf);
-    std::vector<uint8_t> t(nf), e(nf);
-    std::vector<uint64_t> s(nf), w(nf);
-    if (nf) {
-      CK(cudaMemcpyAsync(t.data(), c->rtag.p, nf, cudaMemcpyDeviceToHost, c->stream));
-      CK(cudaMemcpyAsync(e.data(), c->rerr.p, nf, cudaMemcpyDeviceToHost, c->stream));
-      CK(cudaMemcpyAsync(s.data(), c->rsteps.p, nf * 8, cudaMemcpyDeviceToHost, c->stream));
-      CK(cudaMemcpyAsync(w.data(), c->rword.p, nf * 8, cudaMemcpyDeviceToHost, c->stream));
+    r->r.resize(nf);
+    if (nf) {                                        // straight into the result arrays
+      CK(cudaMemcpyAsync(r->r.tag.data(), c->rtag.p, nf, cudaMemcpyDeviceToHost, c->stream));
+      CK(cudaMemcpyAsync(r->r.err.data(), c->rerr.p, nf, cudaMemcpyDeviceToHost, c->stream));
+      CK(cudaMemcpyAsync(r->r.steps.data(), c->rsteps.p, nf * 8, cudaMemcpyDeviceToHost, c->stream));
+      CK(cudaMemcpyAsync(r->r.word.data(), c->rword.p, nf * 8, cudaMemcpyDeviceToHost, c->stream));
     }
-    std::vector<uint4> pay(pc);
-    if (pc) CK(cudaMemcpyAsync(pay.data(), c->payload.p, pc * sizeof(uint4), cudaMemcpyDeviceToHost, c->stream));
-    CK(cudaStreamSynchronize(c->stream));
-    for (uint32_t i = 0; i < nf; ++i) r->r.rec[i] = Record{t[i], e[i], s[i], w[i]};
+    static_assert(sizeof(Token) == sizeof(uint4), "token layout = device uint4 {word.lo, word.hi, tag, 0}");
     r->r.payload.resize(pc);
-    for (size_t k = 0; k < pc; ++k)
-      r->r.payload[k] = Token{((uint64_t)pay[k].y << 32) | pay[k].x, pay[k].z, 0};
+    if (pc) CK(cudaMemcpyAsync(r->r.payload.data(), c->payload.p, pc * sizeof(uint4), cudaMemcpyDeviceToHost, c->stream));
+    CK(cudaStreamSynchronize(c->stream));
     r->r.syms = c->syms;
     r->r.strings = c->strings + c->batch_strings;
     *out = r;
@@ -496,11 +507,11 @@ int culi_records_device(culi_ctx* c, void* dev_buf, size_t cap, size_t* bytes) {
   return CULI_OK;
 }
 
-uint32_t culi_results_count(const culi_results* r) { return r ? (uint32_t)r->r.rec.size() : 0; }
+uint32_t culi_results_count(const culi_results* r) { return r ? (uint32_t)r->r.size() : 0; }
 
 int culi_result_info(const culi_results* r, uint32_t i, uint8_t* tag, uint8_t* err, uint64_t* steps) {
-  if (!r || i >= r->r.rec.size()) return CULI_E_ARG;
-  const Record& x = r->r.rec[i];
+  if (!r || i >= r->r.size()) return CULI_E_ARG;
+  const Record x = r->r.at(i);
   if (tag) *tag = x.tag;
   if (err) *err = x.err;
   if (steps) *steps = x.steps;
@@ -508,23 +519,23 @@ int culi_result_info(const culi_results* r, uint32_t i, uint8_t* tag, uint8_t* e
 }
 
 int culi_result_int(const culi_results* r, uint32_t i, int64_t* v) {
-  if (!r || i >= r->r.rec.size() || !v) return CULI_E_ARG;
-  const Record& x = r->r.rec[i];
+  if (!r || i >= r->r.size() || !v) return CULI_E_ARG;
+  const Record x = r->r.at(i);
   if (x.err || x.tag != K_INT) return CULI_E_ARG;
   *v = (int64_t)x.word;
   return CULI_OK;
 }
 
 int culi_result_float(const culi_results* r, uint32_t i, double* v) {
-  if (!r || i >= r->r.rec.size() || !v) return CULI_E_ARG;
-  const Record& x = r->r.rec[i];
+  if (!r || i >= r->r.size() || !v) return CULI_E_ARG;
+  const Record x = r->r.at(i);
   if (x.err || x.tag != K_FLOAT) return CULI_E_ARG;
   std::memcpy(v, &x.word, 8);
   return CULI_OK;
 }
 
 int culi_print(const culi_results* r, uint32_t i, char* buf, size_t cap, size_t* needed) {
-  if (!r || i >= r->r.rec.size()) return CULI_E_ARG;
+  if (!r || i >= r->r.size()) return CULI_E_ARG;
   std::string s;
   r->r.print(i, s);
   if (needed) *needed = s.size();
@@ -544,9 +555,9 @@ int culi_results_totals(const culi_results* r, uint64_t* total_steps, uint32_t* 
   if (!r) return CULI_E_ARG;
   uint64_t t = 0;
   uint32_t ne = 0;
-  for (const Record& x : r->r.rec) {
-    t += x.steps;
-    ne += x.err != 0;
+  for (size_t q = 0; q < r->r.size(); ++q) {
+    t += r->r.steps[q];
+    ne += r->r.err[q] != 0;
   }
   if (total_steps) *total_steps = t;
   if (n_errors) *n_errors = ne;
@@ -554,6 +565,12 @@ int culi_results_totals(const culi_results* r, uint64_t* total_steps, uint32_t* 
 }
 
 void culi_results_free(culi_results* r) { delete r; }
+
+int culi_results_wire_bytes(const culi_results* r, uint64_t* d2h_bytes) {
+  if (!r || !d2h_bytes) return CULI_E_ARG;
+  *d2h_bytes = r->r.size() * 18 + r->r.payload.size() * sizeof(Token);
+  return CULI_OK;
+}
 
 int culi_last_stats(const culi_ctx* c, uint32_t* fanout_forms, uint32_t* fallback_forms) {
   if (!c) return CULI_E_ARG;

@@ -17,6 +17,13 @@ using namespace culi;
 
 struct culi_image {
   Image img;
+  bool pinned = false;
+  ~culi_image() {
+    if (!pinned) return;
+    if (!img.tag.empty()) cudaHostUnregister(img.tag.data());
+    if (!img.word.empty()) cudaHostUnregister(img.word.data());
+    if (!img.roots.empty()) cudaHostUnregister(img.roots.data());
+  }
 };
 
 struct culi_results {

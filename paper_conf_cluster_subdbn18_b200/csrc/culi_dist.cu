@@ -8,6 +8,7 @@
 // caller all-gathers the blobs; culi_results_merge re-interns symbols by name and reorders by form index.
 #include <cuda_runtime.h>
 
+#include <algorithm>
 #include <cstring>
 #include <memory>
 #include <new>
@@ -144,7 +145,7 @@ int culi_results_serialize(const culi_results* r, void* buf, size_t cap, size_t*
   std::string names = names_blob(*R.syms);
   ResHeader h{};
   h.magic = RES_MAGIC;
-  h.nforms = R.rec.size();
+  h.nforms = R.size();
   h.npayload = R.payload.size();
   h.names_bytes = names.size();
   h.nstr = R.strings.size();
@@ -156,7 +157,8 @@ int culi_results_serialize(const culi_results* r, void* buf, size_t cap, size_t*
   char* p = (char*)buf;
   std::memcpy(p, &h, sizeof h);
   p += sizeof h;
-  for (const Record& x : R.rec) {
+  for (size_t q = 0; q < R.size(); ++q) {
+    const Record x = R.at(q);
     RecWire w{};
     w.steps = x.steps;
     w.word = x.word;
@@ -189,7 +191,9 @@ int culi_results_merge(const void* const* blobs, const size_t* sizes, int nranks
     if (h.magic != RES_MAGIC) return CULI_E_ARG;
     total += h.nforms;
   }
-  M.rec.assign(total, Record{K_ERROR, E_OOM, 0, 0});
+  M.resize(total);
+  std::fill(M.tag.begin(), M.tag.end(), (uint8_t)K_ERROR);
+  std::fill(M.err.begin(), M.err.end(), (uint8_t)E_OOM);
   std::vector<char> seen(total, 0);
   for (int k = 0; k < nranks; ++k) {
     const char* p = (const char*)blobs[k];
@@ -234,7 +238,10 @@ int culi_results_merge(const void* const* blobs, const size_t* sizes, int nranks
         if (w.tag == K_CONS || w.tag == K_STR) word = pack2((uint32_t)(lo32h(word) + pay_base), (uint32_t)(word >> 32));
         else word = fix(w.tag, word);
       }
-      M.rec[gi] = Record{w.tag, w.err, w.steps, word};
+      M.tag[gi] = w.tag;
+      M.err[gi] = w.err;
+      M.steps[gi] = w.steps;
+      M.word[gi] = word;
     }
   }
   M.syms = st;

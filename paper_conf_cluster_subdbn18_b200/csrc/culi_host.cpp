@@ -289,7 +289,7 @@ void Results::print_token_range(size_t& pos, std::string& out) const {
 }
 
 void Results::print(uint32_t i, std::string& out) const {
-  const Record& r = rec[i];
+  const Record r = at(i);
   if (r.err) { out += "#<error "; out += kErrName[r.err < 10 ? r.err : 9]; out += '>'; return; }
   if (r.tag == K_CONS || r.tag == K_STR) {
     size_t pos = (uint32_t)r.word;

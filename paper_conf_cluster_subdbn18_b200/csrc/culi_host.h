@@ -53,7 +53,12 @@ struct Token {
 };
 
 struct Results {
-  std::vector<Record> rec;
+  // records as structure of arrays, so the device arrays are copied straight in (no per-record work)
+  std::vector<uint8_t> tag, err;
+  std::vector<uint64_t> steps, word;
+  size_t size() const { return tag.size(); }
+  Record at(size_t i) const { return Record{tag[i], err[i], steps[i], word[i]}; }
+  void resize(size_t n) { tag.resize(n); err.resize(n); steps.resize(n); word.resize(n); }
   std::vector<Token> payload;
   std::shared_ptr<const SymTable> syms;   // names for SYM tokens
   std::string strings;                    // bytes for STR tokens

@@ -29,7 +29,7 @@ SYMBOLS = [
     "culi_result_int", "culi_result_float", "culi_print", "culi_results_totals", "culi_results_free",
     "culi_env_export", "culi_env_import", "culi_results_serialize", "culi_results_merge",
     "culi_status_string", "culi_error_name", "culi_last_timing", "culi_records_device",
-    "culi_last_stats",
+    "culi_last_stats", "culi_image_pin", "culi_results_wire_bytes",
 ]
 
 
@@ -88,6 +88,8 @@ def load(path: str = LIB_PATH) -> ctypes.CDLL:
         "culi_last_timing": (I, [P, pp(ctypes.c_float), pp(U32), pp(U64)]),
         "culi_records_device": (I, [P, P, SZ, pp(SZ)]),
         "culi_last_stats": (I, [P, pp(U32), pp(U32)]),
+        "culi_image_pin": (I, [P, pp(U64)]),
+        "culi_results_wire_bytes": (I, [P, pp(U64)]),
     }
     for name, (res, args) in sig.items():
         fn = getattr(L, name)
@@ -128,6 +130,12 @@ class Image:
     @property
     def nnodes(self) -> int:
         return load().culi_image_nnodes(self._p)
+
+    def pin(self) -> int:
+        """Page-lock the host arrays (uploads then DMA from pinned memory); returns the H2D bytes."""
+        b = ctypes.c_uint64(0)
+        _check(load().culi_image_pin(self._p, ctypes.byref(b)), "culi_image_pin")
+        return b.value
 
     def __del__(self):
         if getattr(self, "_p", None) and self._p.value:
@@ -171,6 +179,12 @@ class Results:
         s, e = ctypes.c_uint64(), ctypes.c_uint32()
         _check(load().culi_results_totals(self._p, ctypes.byref(s), ctypes.byref(e)), "culi_results_totals")
         return s.value, e.value
+
+    def wire_bytes(self) -> int:
+        """Bytes the fetch copied device -> host (records + value tokens)."""
+        b = ctypes.c_uint64(0)
+        _check(load().culi_results_wire_bytes(self._p, ctypes.byref(b)), "culi_results_wire_bytes")
+        return b.value
 
     def serialize(self) -> bytes:
         L = load()
