@@ -130,8 +130,26 @@ struct V {
   uint64_t w;
 };
 
-__device__ __forceinline__ uint32_t lo32(uint64_t w) { return (uint32_t)w; }
-__device__ __forceinline__ uint32_t hi32(uint64_t w) { return (uint32_t)(w >> 32); }
+// The halves of a node word are 32-bit node indices.  The empty asm makes each half an opaque 32-bit
+// value, so `base + index` compiles to one IMAD.WIDE.U32 instead of 64-bit shift/mask arithmetic on the
+// whole word (measured: 6 instructions per node address otherwise).
+#ifndef CULI_OPAQUE_HALVES
+#define CULI_OPAQUE_HALVES 1
+#endif
+__device__ __forceinline__ uint32_t lo32(uint64_t w) {
+  uint32_t x = (uint32_t)w;
+#if CULI_OPAQUE_HALVES
+  asm("" : "+r"(x));
+#endif
+  return x;
+}
+__device__ __forceinline__ uint32_t hi32(uint64_t w) {
+  uint32_t x = (uint32_t)(w >> 32);
+#if CULI_OPAQUE_HALVES
+  asm("" : "+r"(x));
+#endif
+  return x;
+}
 __device__ __forceinline__ bool is_ref(uint32_t k) {
   return k == K_CONS || k == K_STR || k == K_CLOSURE || k == K_MACRO;
 }

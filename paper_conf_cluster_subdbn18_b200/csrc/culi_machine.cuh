@@ -30,6 +30,8 @@ namespace culi {
 
 extern __shared__ __align__(16) uint4 culi_smem[];   // [code nodes][global words][global tags]
 
+// Cold (out-of-line) helpers take Ctx by value: passing the hot path's Ctx by reference would make it
+// escape to memory, and every launch constant would then cost a local + a generic load (measured).
 struct Ctx {
   const EvalArgs* A;         // the launch's constants (a __grid_constant__ kernel parameter)
   uint4* kb;                 // &kst[slot]   (entry i at kb + i * nslots)
@@ -164,7 +166,7 @@ __device__ __forceinline__ V global_value(const Ctx& C, uint32_t sym) {
 }
 
 // full walk: innermost frame first, leftmost binding first, then the global frame; unbound -> itself
-__device__ CULI_COLD V lookup_slow(const Ctx& C, uint32_t sym, uint32_t env) {
+__device__ CULI_COLD V lookup_slow(Ctx C, uint32_t sym, uint32_t env) {
   while (env != 0) {
     if (env & STACK_ENV) {
       uint32_t h = env & ENV_IDX_MASK, n = (env >> 16) & 0x7fffu;
@@ -204,7 +206,7 @@ __device__ __forceinline__ V lookup(const Ctx& C, uint32_t sym, uint32_t env) {
 
 // Copy the stack frames a closure captures into the heap (frames are immutable, c.3, so a copy is
 // indistinguishable from the original).  Memoised in the stack header's .y field.
-__device__ CULI_COLD bool promote(const Ctx& C, uint32_t env, uint32_t* out) {
+__device__ CULI_COLD bool promote(Ctx C, uint32_t env, uint32_t* out) {
   const DevHeap& H = C.A->H;
   if (!(env & STACK_ENV)) { *out = env; return true; }
   for (;;) {
@@ -244,7 +246,7 @@ __device__ CULI_COLD bool promote(const Ctx& C, uint32_t env, uint32_t* out) {
 // A closure / macro is three nodes: {kind: code | env << 32}, {K_AUX: nparams | first param << 32} and
 // {K_AUX: body | params << 32}, so a call reads all it needs with three independent loads
 // (code = the cons (params . body); env = heap frame or 0).
-__device__ CULI_COLD bool make_closure(const Ctx& C, uint32_t kind, uint32_t code, uint32_t env,
+__device__ CULI_COLD bool make_closure(Ctx C, uint32_t kind, uint32_t code, uint32_t env,
                                           V* out) {
   uint32_t henv, a;
   if (!promote(C, env, &henv)) return false;
@@ -265,7 +267,7 @@ __device__ CULI_COLD bool make_closure(const Ctx& C, uint32_t kind, uint32_t cod
 }
 
 // c.5: a parameter list is a proper list of non-reserved symbols
-__device__ CULI_COLD bool valid_params(const Ctx& C, uint32_t ps) {
+__device__ CULI_COLD bool valid_params(Ctx C, uint32_t ps) {
   if (ps == 0) return true;
   uint32_t t = ntag(C, ps);
   if ((t & KIND_MASK) != K_CONS || !(t & TAG_PROPER)) return false;
@@ -411,7 +413,7 @@ __device__ __forceinline__ uint8_t fast2(const Ctx& C, uint32_t op, uint32_t arg
 }
 
 // equal: recursive on cons cells, with the V-stack above vtop as the explicit work stack
-__device__ CULI_COLD uint8_t equal_values(const Ctx& C, uint32_t vtop, V a, V b, bool* res) {
+__device__ CULI_COLD uint8_t equal_values(Ctx C, uint32_t vtop, V a, V b, bool* res) {
   uint32_t sp = vtop;
   for (;;) {
     bool same;
@@ -442,7 +444,7 @@ __device__ CULI_COLD uint8_t equal_values(const Ctx& C, uint32_t vtop, V a, V b,
 }
 
 // general builtin application over vs[base+1 .. base+cnt] (any arity)
-__device__ CULI_COLD uint8_t apply_builtin(const Ctx& C, uint32_t op, uint32_t base, uint32_t cnt,
+__device__ CULI_COLD uint8_t apply_builtin(Ctx C, uint32_t op, uint32_t base, uint32_t cnt,
                                               uint32_t vtop, V* out) {
   const DevHeap& H = C.A->H;
   if (((FAST_OPS >> op) & 1) && cnt <= 2) {
@@ -586,7 +588,7 @@ __device__ CULI_COLD uint8_t apply_builtin(const Ctx& C, uint32_t op, uint32_t b
 
 // (||| n f l1 .. lm) argument checks (c.7): arity, types left to right, then n >= 0 and every list
 // proper with >= n elements.  Returns 0 and fills n, or an error.
-__device__ CULI_COLD uint8_t par_check(const Ctx& C, uint32_t base, uint32_t cnt, uint32_t* n_out) {
+__device__ CULI_COLD uint8_t par_check(Ctx C, uint32_t base, uint32_t cnt, uint32_t* n_out) {
   if (cnt < 3) return E_ARITY;
   V nv = arg(C, base, 0), f = arg(C, base, 1);
   if (nv.t != K_INT) return E_TYPE;
@@ -607,7 +609,7 @@ __device__ CULI_COLD uint8_t par_check(const Ctx& C, uint32_t base, uint32_t cnt
 }
 
 // The O(1) part of par_check: arity, types, n >= 0, every list proper, and no empty list when n > 0.
-__device__ CULI_COLD uint8_t par_check_light(const Ctx& C, uint32_t base, uint32_t cnt, uint32_t* n_out) {
+__device__ CULI_COLD uint8_t par_check_light(Ctx C, uint32_t base, uint32_t cnt, uint32_t* n_out) {
   if (cnt < 3) return E_ARITY;
   V nv = arg(C, base, 0), f = arg(C, base, 1);
   if (nv.t != K_INT) return E_TYPE;
@@ -625,7 +627,7 @@ __device__ CULI_COLD uint8_t par_check_light(const Ctx& C, uint32_t base, uint32
 }
 
 // runtime syntax checks of special forms without TAG_VALID (c.5); cur = the argument list
-__device__ CULI_COLD bool special_syntax_ok(const Ctx& C, uint32_t op, uint32_t cur) {
+__device__ CULI_COLD bool special_syntax_ok(Ctx C, uint32_t op, uint32_t cur) {
   uint32_t n = 0;
   for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
   switch (op) {
