@@ -173,6 +173,7 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.kst = c->kst;
   A.vst = c->vst;
   A.nslots = c->nslots;
+  A.stride = c->nslots * (uint32_t)sizeof(uint4);
   A.kcap = c->kcap;
   A.vcap = c->vcap;
   A.roots = c->roots.p;

@@ -41,6 +41,7 @@ struct EvalArgs {
   uint4* kst;                  // K-stack, level-major: kst[level * nslots + slot]
   uint4* vst;                  // V-stack, level-major
   uint32_t nslots;
+  uint32_t stride;             // nslots * sizeof(uint4): byte distance between stack levels
   uint32_t kcap;               // K-stack entries per slot
   uint32_t vcap;               // V-stack entries per slot
   const uint32_t* roots;       // heap index of each form's datum

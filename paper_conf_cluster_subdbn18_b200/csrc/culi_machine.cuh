@@ -38,8 +38,13 @@ struct Ctx {
   uint4* vb;                 // &vst[slot]
 };
 
-__device__ __forceinline__ uint4* KS(const Ctx& C, uint32_t i) { return C.kb + (size_t)i * C.A->nslots; }
-__device__ __forceinline__ uint4* VS(const Ctx& C, uint32_t i) { return C.vb + (size_t)i * C.A->nslots; }
+// entry i of this thread's stacks: one IMAD.WIDE.U32 with the precomputed byte stride (nslots * 16)
+__device__ __forceinline__ uint4* KS(const Ctx& C, uint32_t i) {
+  return reinterpret_cast<uint4*>(reinterpret_cast<char*>(C.kb) + (size_t)i * C.A->stride);
+}
+__device__ __forceinline__ uint4* VS(const Ctx& C, uint32_t i) {
+  return reinterpret_cast<uint4*>(reinterpret_cast<char*>(C.vb) + (size_t)i * C.A->stride);
+}
 __device__ __forceinline__ uint4 vpack(V v, uint32_t sym) {
   return make_uint4(lo32(v.w), hi32(v.w), sym, v.t);
 }
@@ -699,13 +704,19 @@ __device__ __forceinline__ int try_leaf(const Ctx& C, uint32_t xt, uint64_t xw, 
       argc = 2;
     }
   }
-  for (uint32_t i = 0; i <= argc; ++i) {              // head step, then one step per argument
-    ++steps;
-    if (__builtin_expect(steps > fuel || dx + 1 > maxd, 0)) {
-      *err = steps > fuel ? E_FUEL : E_DEPTH;
-      return 2;
+  // head step, then one step per argument (argc + 1 steps at depth dx + 1), checked at once; on failure
+  // the first failing step decides: fuel before depth at each step (c.4 step 1)
+  if (__builtin_expect(steps + argc + 1 > fuel || dx + 1 > maxd, 0)) {
+    if (steps + 1 > fuel || dx + 1 <= maxd) {
+      *err = E_FUEL;
+      steps = fuel + 1;
+    } else {
+      *err = E_DEPTH;
+      steps = steps + 1;
     }
+    return 2;
   }
+  steps += argc + 1;
   V a0 = mkv(K_NIL, 0), a1 = mkv(K_NIL, 0);
   if (argc > 0) a0 = (t1 & KIND_MASK) == K_SYM ? lookup(C, (uint32_t)w1, env) : unbox_loaded(n1, t1, w1);
   if (argc > 1) a1 = (t2 & KIND_MASK) == K_SYM ? lookup(C, (uint32_t)w2, env) : unbox_loaded(n2, t2, w2);
