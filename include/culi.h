@@ -76,7 +76,8 @@ typedef struct {
 #define CULI_F_NO_BINNING 1u   /* evaluate forms in input order (no classify+sort dispatch, §8(a)5)     */
 #define CULI_F_NO_FANOUT  2u   /* evaluate top-level ||| forms in one thread (no fan-out, §8(a)6)        */
 #define CULI_F_NO_STAGING 4u   /* do not stage the global frame / hot code in shared memory (§8(a)4)     */
-#define CULI_F_NO_VOTING  8u   /* disable warp opcode voting in the eval loop                            */
+#define CULI_F_NO_VOTING  8u   /* reserved (no effect in this version)                                   */
+#define CULI_F_NO_NESTED 16u   /* run nested (non-top-level) ||| forms inside one thread (§8(f)1 off)     */
 
 /* Fill *opts with defaults (device 0, default stream, default sizes). */
 void culi_default_opts(culi_opts* opts);
@@ -165,9 +166,10 @@ const char* culi_error_name(uint8_t err);
  * number of kernels launched by that call.  Heap high-water mark in nodes. */
 int culi_last_timing(const culi_ctx* ctx, float* ms3, uint32_t* kernels, uint64_t* heap_high);
 /* Path statistics of the last fetched batch: forms handled by the fan-out kernels (top-level ||| forms
- * and wide forms) and, of those, forms re-evaluated sequentially (an element error,
- * fuel overflow, or a short / non-contiguous list). */
-int culi_last_stats(const culi_ctx* ctx, uint32_t* fanout_forms, uint32_t* fallback_forms);
+ * and wide forms), nested ||| evaluations that suspended and fanned out (§8(f)1),
+ * and forms re-evaluated sequentially (an element error, fuel overflow, a short / non-contiguous list). */
+int culi_last_stats(const culi_ctx* ctx, uint32_t* fanout_forms, uint32_t* fallback_forms,
+                    uint32_t* nested_forms);
 
 #ifdef __cplusplus
 }

@@ -90,6 +90,8 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   ok &= cudaMalloc(&c->desc, (size_t)c->maxdesc * sizeof(FanDesc)) == cudaSuccess;
   ok &= cudaMalloc(&c->npend, sizeof(uint32_t)) == cudaSuccess;
   ok &= cudaMalloc(&c->nfallback, sizeof(uint32_t)) == cudaSuccess;
+  ok &= cudaMalloc(&c->nnest, 2 * sizeof(uint32_t)) == cudaSuccess;
+  ok &= cudaMalloc(&c->ndesc, (size_t)c->maxnest * sizeof(NestDesc)) == cudaSuccess;
   for (int k = 0; k < 4 && ok; ++k) ok &= cudaEventCreate(&c->ev[k]) == cudaSuccess;
   if (!ok) { culi_shutdown(c); return CULI_E_CUDA; }
   c->H.cap = o.heap_nodes;
@@ -124,6 +126,10 @@ void culi_shutdown(culi_ctx* c) {
   cudaFree(c->desc);
   cudaFree(c->npend);
   cudaFree(c->nfallback);
+  cudaFree(c->nnest);
+  cudaFree(c->ndesc);
+  cudaFree(c->kst2);
+  cudaFree(c->vst2);
   c->fallback.release();
   c->wide.release();
   c->roots.release(); c->keys.release(); c->keys_alt.release(); c->perm.release();
@@ -167,6 +173,21 @@ int culi_image_pin(culi_image* im, uint64_t* h2d_bytes) {
 }  // extern "C"
 
 // ---- internal helpers ------------------------------------------------------------------------------
+// Does the ||| symbol occur in the image?  With skip_root_heads, occurrences that are the head of a
+// top-level form do not count: those forms go to the top-level fan-out (a6), never through nesting.
+// (Symbol nodes are shared within an image, so look at the cons cells that refer to it.)
+static bool image_mentions_par(const Image& img, bool skip_root_heads = false) {
+  uint32_t par = 0;
+  for (size_t k = 0; k < img.tag.size() && !par; ++k)
+    if ((img.tag[k] & KIND_MASK) == K_SYM && img.word[k] == N_SPECIALS + BI_PAR) par = IMG_FIRST + (uint32_t)k;
+  if (!par || !skip_root_heads) return par != 0;
+  std::vector<char> root(img.tag.size(), 0);
+  for (uint32_t r : img.roots)
+    if (r >= IMG_FIRST) root[r - IMG_FIRST] = 1;
+  for (size_t k = 0; k < img.tag.size(); ++k)
+    if ((img.tag[k] & KIND_MASK) == K_CONS && !root[k] && (uint32_t)img.word[k] == par) return true;
+  return false;
+}
 static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, int define_mode) {
   EvalArgs A{};
   A.H = c->H;
@@ -196,6 +217,13 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.fallback = c->fallback.p;
   A.nfallback = c->nfallback;
   A.wide = (!define_mode && c->batch_has_wide) ? c->wide.p : nullptr;
+  A.nest = (!define_mode && c->batch_may_nest && c->kst2 && !(c->opts.flags & CULI_F_NO_NESTED)) ? 1 : 0;
+  A.ndesc = c->ndesc;
+  A.nnest = c->nnest;
+  A.maxnest = c->maxnest;
+  A.kst2 = c->kst2;
+  A.vst2 = c->vst2;
+  A.finished = c->nnest + 1;
   A.payload = c->payload.p;
   A.pcount = c->pcount;
   A.pcap = c->payload.n;
@@ -245,10 +273,11 @@ extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed
   int rc = upload_image(c, img, str_base);
   if (rc) return rc;
   c->strings += img.strings;
+  c->persist_has_par = c->persist_has_par || image_mentions_par(img);
   rc = ensure_results(c, nf);
   if (rc) return rc;
   CK(launch_reset(c->stream, c->H.top, c->mark + img.tag.size(), c->next, c->pcount, c->flags, c->npend,
-                  c->nfallback));
+                  c->nfallback, c->nnest));
   EvalArgs A = make_args(c, nf, nullptr, 1);
   if (nf) CK(launch_define(c->stream, A));
   int flags[8];
@@ -275,7 +304,7 @@ static int run_batch_device(culi_ctx* c) {
   c->last_kernels = 0;
   CK(cudaEventRecord(c->ev[0], c->stream));
   CK(launch_reset(c->stream, c->H.top, c->mark + c->batch_nodes, c->next, c->pcount, c->flags, c->npend,
-                  c->nfallback));
+                  c->nfallback, c->nnest));
   ++c->last_kernels;
   uint32_t* perm = nullptr;
   if (!(c->opts.flags & CULI_F_NO_BINNING) && nf > 1) {
@@ -286,9 +315,11 @@ static int run_batch_device(culi_ctx* c) {
   CK(cudaEventRecord(c->ev[1], c->stream));
   EvalArgs A = make_args(c, nf, perm, 0);
   A.fanout = A.fanout && c->batch_has_par;
+  if (A.nest) { CK(launch_nest_clear(c->stream, c->ndesc, c->maxnest)); ++c->last_kernels; }
   uint32_t blocks = c->nslots / 128;
   uint32_t need = (nf + 127) / 128;
-  if (need < blocks) blocks = std::max<uint32_t>(need, 1);
+  // a batch that may suspend on nested ||| keeps the whole grid: idle threads apply the elements
+  if (need < blocks && !A.nest) blocks = std::max<uint32_t>(need, 1);
   if (nf) { CK(launch_eval(c->stream, A, blocks)); ++c->last_kernels; }
   if (nf && A.fanout && c->batch_has_par) {            // ||| fan-out (a6) + finalize (a8)
     CK(launch_fanout(c->stream, A, c->nslots / 128));
@@ -338,7 +369,14 @@ static int prepare_batch(culi_ctx* c, const Image& img) {
   c->batch_nodes = img.tag.size();
   c->batch_forms = nf;
   c->batch_strings = img.strings;
-  CK(c->fallback.ensure(std::max<size_t>(c->maxdesc, 1)));
+  CK(c->fallback.ensure((size_t)c->maxdesc + nf + 1));
+  // may ||| occur below the top level (nested fan-out, §8(f)1)?  any ||| symbol in the batch or in a definition
+  c->batch_may_nest = c->persist_has_par ||
+                      image_mentions_par(img, !(c->opts.flags & CULI_F_NO_FANOUT));
+  if (c->batch_may_nest && !c->kst2 && !(c->opts.flags & CULI_F_NO_NESTED)) {
+    CK(cudaMalloc(&c->kst2, (size_t)c->nslots * c->kcap * sizeof(uint4)));
+    CK(cudaMalloc(&c->vst2, (size_t)c->nslots * c->vcap * sizeof(uint4)));
+  }
   // does any form start with the ||| symbol (a6), or have >= WIDE_MIN arguments (wide forms, K12)?
   c->batch_has_par = false;
   c->batch_has_wide = false;
@@ -373,6 +411,7 @@ static int rerun_fallback(culi_ctx* c, uint32_t nfb) {
   CK(cudaMemsetAsync(c->next, 0, sizeof(uint32_t), c->stream));
   EvalArgs A = make_args(c, nfb, c->fallback.p, 0);
   A.fanout = 0;
+  A.nest = 0;
   CK(launch_eval(c->stream, A, std::max<uint32_t>(1, std::min<uint32_t>(c->nslots / 128, (nfb + 127) / 128))));
   ExportArgs X{};
   X.tag = c->H.tag;
@@ -399,8 +438,9 @@ static int fetch(culi_ctx* c, culi_results** out) {
   for (int attempt = 0; attempt < 4; ++attempt) {
     int flags[8];
     unsigned long long pc = 0, top = 0;
-    uint32_t nfb = 0, npend = 0;
+    uint32_t nfb = 0, npend = 0, nnest = 0;
     CK(cudaMemcpyAsync(&npend, c->npend, 4, cudaMemcpyDeviceToHost, c->stream));
+    CK(cudaMemcpyAsync(&nnest, c->nnest, 4, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(flags, c->flags, sizeof flags, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(&pc, c->pcount, 8, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(&top, c->H.top, 8, cudaMemcpyDeviceToHost, c->stream));
@@ -411,6 +451,7 @@ static int fetch(culi_ctx* c, culi_results** out) {
     if (attempt == 0) {
       c->last_fanout = (c->batch_has_par && !(c->opts.flags & CULI_F_NO_FANOUT)) ? std::min(npend, c->maxdesc) : 0;
       c->last_fallback = 0;
+      c->last_nested = c->batch_may_nest ? std::min(nnest, c->maxnest) : 0;
     }
     if (nfb && !flags[3]) {
       c->last_fallback += nfb;
@@ -573,8 +614,10 @@ int culi_results_wire_bytes(const culi_results* r, uint64_t* d2h_bytes) {
   return CULI_OK;
 }
 
-int culi_last_stats(const culi_ctx* c, uint32_t* fanout_forms, uint32_t* fallback_forms) {
+int culi_last_stats(const culi_ctx* c, uint32_t* fanout_forms, uint32_t* fallback_forms,
+                    uint32_t* nested_forms) {
   if (!c) return CULI_E_ARG;
+  if (nested_forms) *nested_forms = c->last_nested;
   if (fanout_forms) *fanout_forms = c->last_fanout;
   if (fallback_forms) *fallback_forms = c->last_fallback;
   return CULI_OK;

@@ -88,7 +88,15 @@ struct culi_ctx {
   DevBuf<uint32_t> fallback;
   bool batch_has_par = false;
   bool batch_has_wide = false;
-  uint32_t last_fanout = 0, last_fallback = 0;
+  // nested ||| (§8(f)1)
+  bool persist_has_par = false;      // some definition mentions |||
+  bool batch_may_nest = false;
+  NestDesc* ndesc = nullptr;
+  uint32_t maxnest = 4096;
+  uint32_t* nnest = nullptr;         // [0] descriptors written, [1] forms finished
+  uint4* kst2 = nullptr;             // secondary stacks, allocated on first use
+  uint4* vst2 = nullptr;
+  uint32_t last_fanout = 0, last_fallback = 0, last_nested = 0;
   DevBuf<uint32_t> wide;
   // uploaded batch (culi_upload)
   bool have_batch = false;

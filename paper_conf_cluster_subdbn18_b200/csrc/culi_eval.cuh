@@ -67,6 +67,13 @@ struct EvalArgs {
   unsigned long long* pcount;
   unsigned long long pcap;
   const uint32_t* wide;        // per form: argument count of a wide top-level form, else 0 (host scan)
+  uint32_t nest;               // nested ||| suspend + help, batch eval kernel only
+  struct NestDesc* ndesc;
+  uint32_t* nnest;
+  uint32_t maxnest;
+  uint4* kst2;                 // secondary stacks (elements run by a thread whose own form is suspended)
+  uint4* vst2;
+  uint32_t* finished;          // forms completed (threads without forms help until all are done)
   uint32_t code_lo, code_n;    // node range staged in shared memory (persistent code segment)
   uint32_t gst;                // global-frame entries staged in shared memory
 };
@@ -92,7 +99,24 @@ struct FanDesc {
   uint32_t nonflat;                          // some element value is a cons (export walks it)
   unsigned long long flat_off;               // payload offset of a flat result list
 };
-constexpr uint8_t K_FLATREC = 12;            // internal record tag: flat ||| result awaiting export
+constexpr uint8_t K_FLATREC = 12;
+
+// A nested (||| n f l1..lm) whose evaluation is suspended until its elements are applied (§8(f)1): the
+// owner thread saved {sp, vtop, steps}; any thread claims elements (next), applies f with the fuel left
+// and adds their steps; when done == n the owner resumes at RET with the result spine.
+constexpr uint32_t NEST_MIN = 32;
+constexpr uint8_t E_SUSPEND = 0xfc;
+struct NestDesc {
+  uint32_t form, n, m, spine;
+  uint32_t ftag, depth;
+  uint64_t fword;
+  uint64_t steps0;
+  uint64_t top;
+  uint32_t heads[FANOUT_MAXM];
+  uint32_t sp, vtop;
+  unsigned long long total;
+  uint32_t next, done, bad, ready;            // ready: fields published, elements claimable
+};            // internal record tag: flat ||| result awaiting export
 
 struct ExportArgs {
   const uint8_t* tag;
@@ -118,8 +142,9 @@ cudaError_t launch_define(cudaStream_t s, const EvalArgs& A);
 cudaError_t launch_export(cudaStream_t s, const ExportArgs& X, uint32_t blocks);
 cudaError_t launch_reset(cudaStream_t s, unsigned long long* top, unsigned long long top_value,
                          uint32_t* next, unsigned long long* pcount, int* flags, uint32_t* npend,
-                         uint32_t* nfallback);
+                         uint32_t* nfallback, uint32_t* nnest);
 cudaError_t launch_fanout(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
+cudaError_t launch_nest_clear(cudaStream_t s, struct NestDesc* d, uint32_t n);
 cudaError_t launch_flat_export(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
 cudaError_t launch_dispatch(cudaStream_t s, const DevHeap& H, const uint32_t* roots, uint32_t nforms,
                             uint32_t* keys, uint32_t* keys_alt, uint32_t* perm, uint32_t* perm_alt,

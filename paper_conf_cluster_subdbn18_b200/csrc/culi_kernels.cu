@@ -51,7 +51,57 @@ __device__ __forceinline__ Ctx make_ctx(const EvalArgs& A, uint32_t slot) {
 // Batch mode.  Shared memory per block: the persistent code segment [code_lo, code_lo + code_n) as
 // {w.lo, w.hi, tag, 0} and the global frame [0, gst) ("stage").  Each warp takes 32
 // consecutive forms of the (binned) order with one atomicAdd and runs them to completion.
-template <bool FANOUT>
+// ---- nested |||: claim and apply one element of descriptor D ---------------------------
+// Runs on the thread's secondary stacks (C2).  Element i: f applied to (l1[i] .. lm[i]) at the depth of the
+// ||| call, with the fuel left when the owner suspended.  A failed contiguity check or an element error
+// marks the descriptor bad (the owner's form is then re-evaluated sequentially, exactly).
+__device__ __forceinline__ bool nest_run_one(const EvalArgs& A, const Ctx& C2, NestDesc* D) {
+  if (*(volatile uint32_t*)&D->ready == 0) return false;
+  uint32_t n = D->n;
+  if (*(volatile uint32_t*)&D->next >= n) return false;
+  uint32_t i = atomicAdd(&D->next, 1u);
+  if (i >= n) return false;
+  const DevHeap& H = A.H;
+  uint32_t m = D->m, spine = D->spine;
+  bool ok = true;
+  *VS(C2, 0) = vpack(mkv(D->ftag, D->fword), 0);
+  for (uint32_t j = 0; j < m; ++j) {
+    uint32_t c = D->heads[j] + i;
+    if ((uint64_t)c >= D->top) { ok = false; break; }
+    uint32_t tc = H.tag[c];
+    uint64_t wc = H.word[c];
+    if ((tc & KIND_MASK) != K_CONS || (i + 1 < n && hi32(wc) != c + 1)) { ok = false; break; }
+    *VS(C2, 1 + j) = vpack(unbox(C2, lo32(wc)), 0);
+  }
+  if (!ok) {
+    atomicOr(&D->bad, 1u);
+  } else {
+    FormOut o = eval_form<false, true>(C2, 0, D->form, 1, m, A.fuel - D->steps0, D->depth);
+    if (o.err) {
+      atomicOr(&D->bad, 2u);
+    } else {
+      uint32_t ca = box_into(H, mkv(o.t, o.w), spine + n + i);
+      H.tag[spine + i] = K_CONS | TAG_PROPER;
+      H.word[spine + i] = pack2(ca, i + 1 < n ? spine + i + 1 : 0);
+      atomicAdd(&D->total, (unsigned long long)o.steps);
+    }
+  }
+  __threadfence();
+  atomicAdd(&D->done, 1u);
+  return true;
+}
+
+// Help any published descriptor with unclaimed elements; returns whether an element was applied.
+__device__ __forceinline__ bool nest_help_any(const EvalArgs& A, const Ctx& C2, NestDesc* prefer) {
+  if (prefer && nest_run_one(A, C2, prefer)) return true;
+  uint32_t nn = *(volatile uint32_t*)A.nnest;
+  if (nn > A.maxnest) nn = A.maxnest;
+  for (uint32_t k = 0; k < nn; ++k)
+    if (nest_run_one(A, C2, A.ndesc + k)) return true;
+  return false;
+}
+
+template <bool FANOUT, bool NEST>
 __global__ void __launch_bounds__(128, 4) culi_eval_kernel(const __grid_constant__ EvalArgs A) {
   uint4* scode = culi_smem;
   uint64_t* sgword = reinterpret_cast<uint64_t*>(culi_smem + A.code_n);
@@ -67,6 +117,12 @@ __global__ void __launch_bounds__(128, 4) culi_eval_kernel(const __grid_constant
   __syncthreads();
   uint32_t slot = blockIdx.x * blockDim.x + threadIdx.x;
   Ctx C = make_ctx(A, slot);
+  Ctx C2;
+  if (NEST) {
+    C2.A = &A;
+    C2.kb = A.kst2 + slot;
+    C2.vb = A.vst2 + slot;
+  }
   int lane = threadIdx.x & 31;
   for (;;) {
     uint32_t b = 0;
@@ -76,9 +132,35 @@ __global__ void __launch_bounds__(128, 4) culi_eval_kernel(const __grid_constant
     uint32_t i = b + lane;
     if (i < A.nforms) {
       uint32_t f = A.perm ? A.perm[i] : i;
-      FormOut o = eval_form<FANOUT, false>(C, A.roots[f], f, 0, 0, A.fuel);
+      FormOut o;
+      bool resume = false;
+      Resume R{};
+      for (;;) {
+        o = eval_form<FANOUT, false, NEST>(C, A.roots[f], f, 0, 0, A.fuel, 1, resume, R);
+        if (!NEST || o.err != E_SUSPEND) break;
+        NestDesc* D = A.ndesc + o.aux;                  // suspended on a nested |||: help until done
+        while (*(volatile uint32_t*)&D->done < D->n)
+          if (!nest_help_any(A, C2, D)) __nanosleep(128);
+        __threadfence();
+        uint64_t s = D->steps0 + *(volatile unsigned long long*)&D->total;
+        if (*(volatile uint32_t*)&D->bad || s > A.fuel) {   // decide exactly: sequential re-evaluation
+          A.fallback[atomicAdd(A.nfallback, 1u)] = f;
+          o.err = E_PENDING;
+          break;
+        }
+        R.sp = D->sp;
+        R.vtop = D->vtop;
+        R.steps = s;
+        R.v = mkv(K_CONS, D->spine);
+        resume = true;
+      }
       write_result(A, f, o);
+      if (NEST) atomicAdd(A.finished, 1u);
     }
+  }
+  if (NEST) {                                           // no forms left: help until every form is done
+    while (*(volatile uint32_t*)A.finished < A.nforms)
+      if (!nest_help_any(A, C2, nullptr)) __nanosleep(256);
   }
 }
 
@@ -152,13 +234,24 @@ __global__ void __launch_bounds__(128) culi_export_kernel(ExportArgs X) {
 
 __global__ void culi_reset_kernel(unsigned long long* top, unsigned long long top_value, uint32_t* next,
                                   unsigned long long* pcount, int* flags, uint32_t* npend,
-                                  uint32_t* nfallback) {
+                                  uint32_t* nfallback, uint32_t* nnest) {
   *top = top_value;
   *next = 0;
   *pcount = 0;
   *npend = 0;
   *nfallback = 0;
+  *nnest = 0;                                         // nnest[1] counts finished forms
+  nnest[1] = 0;
   for (int k = 0; k < 8; ++k) flags[k] = 0;
+}
+
+__global__ void culi_nest_clear_kernel(NestDesc* d, uint32_t n) {
+  for (uint32_t k = blockIdx.x * blockDim.x + threadIdx.x; k < n; k += gridDim.x * blockDim.x) d[k].ready = 0;
+}
+
+cudaError_t launch_nest_clear(cudaStream_t s, NestDesc* d, uint32_t n) {
+  culi_nest_clear_kernel<<<(n + 255) / 256, 256, 0, s>>>(d, n);
+  return cudaGetLastError();
 }
 
 // ---- ||| fan-out ------------------------------------------------
@@ -348,14 +441,17 @@ size_t eval_smem_bytes(const EvalArgs& A) {
 cudaError_t launch_eval(cudaStream_t s, const EvalArgs& A, uint32_t blocks) {
   size_t smem = eval_smem_bytes(A);
   if (smem > 48 * 1024) {
-    cudaError_t e = cudaFuncSetAttribute(A.fanout ? culi_eval_kernel<true> : culi_eval_kernel<false>,
-                                         cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    void (*k)(EvalArgs) = A.fanout ? (A.nest ? culi_eval_kernel<true, true> : culi_eval_kernel<true, false>)
+                                   : (A.nest ? culi_eval_kernel<false, true> : culi_eval_kernel<false, false>);
+    cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     if (e != cudaSuccess) return e;
   }
-  if (A.fanout)
-    culi_eval_kernel<true><<<blocks, 128, smem, s>>>(A);   // batches holding top-level ||| forms
-  else
-    culi_eval_kernel<false><<<blocks, 128, smem, s>>>(A);
+  // specialised on whether the batch holds top-level ||| / wide forms (FANOUT) and whether ||| can occur
+  // below the top level (NEST): batches without them run the lean kernel
+  if (A.fanout && A.nest) culi_eval_kernel<true, true><<<blocks, 128, smem, s>>>(A);
+  else if (A.fanout) culi_eval_kernel<true, false><<<blocks, 128, smem, s>>>(A);
+  else if (A.nest) culi_eval_kernel<false, true><<<blocks, 128, smem, s>>>(A);
+  else culi_eval_kernel<false, false><<<blocks, 128, smem, s>>>(A);
   return cudaGetLastError();
 }
 
@@ -371,8 +467,8 @@ cudaError_t launch_export(cudaStream_t s, const ExportArgs& X, uint32_t blocks) 
 
 cudaError_t launch_reset(cudaStream_t s, unsigned long long* top, unsigned long long top_value,
                          uint32_t* next, unsigned long long* pcount, int* flags, uint32_t* npend,
-                         uint32_t* nfallback) {
-  culi_reset_kernel<<<1, 1, 0, s>>>(top, top_value, next, pcount, flags, npend, nfallback);
+                         uint32_t* nfallback, uint32_t* nnest) {
+  culi_reset_kernel<<<1, 1, 0, s>>>(top, top_value, next, pcount, flags, npend, nfallback, nnest);
   return cudaGetLastError();
 }
 

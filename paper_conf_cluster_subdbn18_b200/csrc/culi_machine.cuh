@@ -733,14 +733,23 @@ struct FormOut {
   uint64_t w;
   uint64_t steps;
   uint8_t err;
+  uint32_t aux;        // E_SUSPEND: index of the nested-||| descriptor
+};
+
+// state to resume a suspended evaluation at RET with value v (the nested |||'s result)
+struct Resume {
+  uint32_t sp, vtop;
+  uint64_t steps;
+  V v;
 };
 
 // eval_form(C, root, form, 0, 0, fuel): evaluate the datum at node `root` at depth 1.
 // eval_form(C, 0, form, 1, m, budget): apply vs[0] to the m values vs[1..m] as the body of a top-level
 //   (||| ...) form (depth 1) — one fan-out element (c.7); `budget` = fuel left after the ||| arguments.
-template <bool FANOUT, bool APPLY>
+template <bool FANOUT, bool APPLY, bool NEST = false>
 __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32_t form, int apply_mode,
-                                             uint32_t apply_cnt, uint64_t fuel, uint32_t d0 = 1) {
+                                             uint32_t apply_cnt, uint64_t fuel, uint32_t d0 = 1,
+                                             bool resume = false, const Resume& R = Resume{}) {
   const DevHeap& H = C.A->H;
   const uint32_t kcap = C.A->kcap, vcap = C.A->vcap, maxd = C.A->max_depth;
   const bool fanout = FANOUT && !APPLY && C.A->fanout;
@@ -773,6 +782,15 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32
   } while (0)
 #define ATOMVAL(n, tt, ww) (((tt) & KIND_MASK) == K_SYM ? lookup(C, (uint32_t)(ww), env) : unbox_loaded((n), (tt), (ww)))
 
+  uint32_t aux = 0;
+  if (NEST && resume) {                                         // continue a suspended evaluation
+    sp = R.sp;
+    vtop = R.vtop;
+    steps = R.steps;
+    v = R.v;
+    if (sp > 0) ktop = *KS(C, sp - 1);
+    goto RET;
+  }
   if (APPLY && apply_mode) {
     base = 0;
     hv = *VS(C, 0);
@@ -1095,6 +1113,44 @@ APPLY: {                                                        // apply vs[base
         goto done;
       }
     }
+    if (NEST && !APPLY && C.A->nest && cnt >= 3 && cnt - 2 <= FANOUT_MAXM) {
+      // nested ||| (§8(f)1): suspend; the elements are applied by any threads, then we resume at RET
+      uint8_t e = par_check_light(C, base, cnt, &n);
+      if (__builtin_expect(!!(e), 0)) FAIL(e);
+      if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
+      if (n >= NEST_MIN) {
+        uint32_t slot = atomicAdd(C.A->nnest, 1u);
+        if (slot < C.A->maxnest) {
+          uint32_t spine;
+          if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
+          NestDesc* D = C.A->ndesc + slot;
+          V f = arg(C, base, 1);
+          D->form = form;
+          D->n = n;
+          D->m = cnt - 2;
+          D->spine = spine;
+          D->ftag = f.t;
+          D->depth = d;
+          D->fword = f.w;
+          D->steps0 = steps;
+          D->top = atomicAdd(H.top, 0ull);
+          for (uint32_t j = 0; j < cnt - 2; ++j) D->heads[j] = (uint32_t)arg(C, base, 2 + j).w;
+          D->sp = sp;
+          D->vtop = base;
+          D->total = 0;
+          D->bad = 0;
+          D->done = 0;
+          D->next = 0;
+          __threadfence();
+          atomicExch(&D->ready, 1u);                            // publish: elements may be claimed
+          if (kdirty) *KS(C, sp - 1) = ktop;                    // the resume reloads the top frame
+          v = mkv(K_CONS, spine);
+          aux = slot;
+          err = E_SUSPEND;
+          goto done;
+        }
+      }
+    }
     uint8_t e = par_check(C, base, cnt, &n);
     if (__builtin_expect(!!(e), 0)) FAIL(e);
     if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
@@ -1305,6 +1361,7 @@ done:
   o.w = v.w;
   o.steps = steps;
   o.err = err;
+  o.aux = aux;
   return o;
 }
 

@@ -21,6 +21,7 @@ CULI_F_NO_BINNING = 1
 CULI_F_NO_FANOUT = 2
 CULI_F_NO_STAGING = 4
 CULI_F_NO_VOTING = 8
+CULI_F_NO_NESTED = 16
 
 SYMBOLS = [
     "culi_default_opts", "culi_init", "culi_shutdown", "culi_read", "culi_image_nforms",
@@ -87,7 +88,7 @@ def load(path: str = LIB_PATH) -> ctypes.CDLL:
         "culi_error_name": (ctypes.c_char_p, [ctypes.c_uint8]),
         "culi_last_timing": (I, [P, pp(ctypes.c_float), pp(U32), pp(U64)]),
         "culi_records_device": (I, [P, P, SZ, pp(SZ)]),
-        "culi_last_stats": (I, [P, pp(U32), pp(U32)]),
+        "culi_last_stats": (I, [P, pp(U32), pp(U32), pp(U32)]),
         "culi_image_pin": (I, [P, pp(U64)]),
         "culi_results_wire_bytes": (I, [P, pp(U64)]),
     }
@@ -138,8 +139,8 @@ class Image:
         return b.value
 
     def __del__(self):
-        if getattr(self, "_p", None) and self._p.value:
-            load().culi_image_free(self._p)
+        if getattr(self, "_p", None) and self._p.value and _lib is not None:   # None at interpreter exit
+            _lib.culi_image_free(self._p)
             self._p = None
 
 
@@ -196,8 +197,8 @@ class Results:
         return buf.raw[: need.value]
 
     def __del__(self):
-        if getattr(self, "_p", None) and self._p.value:
-            load().culi_results_free(self._p)
+        if getattr(self, "_p", None) and self._p.value and _lib is not None:   # None at interpreter exit
+            _lib.culi_results_free(self._p)
             self._p = None
 
 
@@ -300,9 +301,11 @@ class Context:
         return list(ms), k.value, h.value
 
     def last_stats(self) -> tuple[int, int]:
-        """(forms handled by the fan-out kernels, of which re-evaluated sequentially) of the last batch."""
-        a, b = ctypes.c_uint32(), ctypes.c_uint32()
-        _check(load().culi_last_stats(self._p, ctypes.byref(a), ctypes.byref(b)), "culi_last_stats")
+        """(forms handled by the fan-out kernels, forms re-evaluated sequentially) of the last batch."""
+        a, b, c = ctypes.c_uint32(), ctypes.c_uint32(), ctypes.c_uint32()
+        _check(load().culi_last_stats(self._p, ctypes.byref(a), ctypes.byref(b), ctypes.byref(c)),
+               "culi_last_stats")
+        self.last_nested = c.value
         return a.value, b.value
 
     def records_device(self, dev_ptr: int | None, cap: int = 0) -> int:

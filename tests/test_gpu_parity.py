@@ -301,3 +301,43 @@ def test_wide_forms_fuel(culi, oracle_mod):
     forms = "(list %s)" % " ".join(["(fib 8)"] * 100)
     for fuel in (500, 6000, 6800, 100000):
         assert_parity(culi, oracle_mod, DEFS, forms, ctx_kw=dict(fuel=fuel), oracle_kw=dict(fuel=fuel))
+
+
+NESTED_DEFS = "\n".join([W.FIB_DEF, W.FACT_DEF,
+    "(define pfib (lambda (xs) (||| (length xs) fib xs)))",
+    "(define psq (lambda (xs) (||| (length xs) (lambda (x) (* x x)) xs)))",
+    "(define pscale (lambda (k xs) (||| (length xs) (lambda (x) (+ (* k x) 0.5)) xs)))",
+    "(define xs40 '(%s))" % " ".join(str(i % 13) for i in range(40)),
+    "(define xs100 '(%s))" % " ".join(str(i) for i in range(100)),
+    "(define xs3000 '(%s))" % " ".join(str(i % 17) for i in range(3000))])
+
+
+def test_nested_par(culi, oracle_mod):
+    """||| below the top level: suspended evaluations resume with the elements' results."""
+    forms = ["(pfib xs40)", "(car (pfib xs40))", "(+ 1 (length (psq xs100)))", "(psq xs3000)",
+             "(pscale 3 xs100)", "(pscale 2.5 xs3000)", "(list (pfib xs40) (psq xs100))",
+             "(let ((r (pfib xs40))) (equal r (pfib xs40)))",
+             "(||| 2 pfib (list xs40 xs40))",                               # nested inside a top-level fan-out
+             "(psq (list 1 2 3))",                                          # below NEST_MIN: sequential
+             "(psq (cons 'a xs40))",                                        # element TYPE error -> fallback
+             "(fact (length (psq xs100)))"] * 3
+    text = "\n".join(forms)
+    assert_parity(culi, oracle_mod, NESTED_DEFS, text)
+    ctx = culi.Context(**SMALL)
+    ctx.define(NESTED_DEFS)
+    r = ctx.eval_batch(text)
+    assert len(r) == len(forms)
+    fan, fb = ctx.last_stats()
+    # each call of pfib/psq/pscale on a >= 32-element list suspends once; the element-error form falls back
+    assert ctx.last_nested >= 3 * 9 and fb >= 3, (fan, fb, ctx.last_nested)
+    ctx2 = culi.Context(**SMALL, flags=culi.CULI_F_NO_NESTED)
+    ctx2.define(NESTED_DEFS)
+    r2 = ctx2.eval_batch(text)
+    assert r.printed() == r2.printed() and r.steps() == r2.steps()
+
+
+def test_nested_par_limits(culi, oracle_mod):
+    forms = "\n".join(["(pfib xs40)", "(psq xs3000)", "(pscale 2 xs40)"])      # (fib <= 12) elements
+    for fuel, depth in ((1 << 40, 1024), (5000, 1024), (200000, 1024), (1 << 40, 6), (1 << 40, 4)):
+        assert_parity(culi, oracle_mod, NESTED_DEFS, forms, ctx_kw=dict(fuel=fuel, max_depth=depth),
+                      oracle_kw=dict(fuel=fuel, max_depth=depth))
