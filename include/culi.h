@@ -78,6 +78,7 @@ typedef struct {
 #define CULI_F_NO_STAGING 4u   /* do not stage the global frame / hot code in shared memory (§8(a)4)     */
 #define CULI_F_NO_VOTING  8u   /* reserved (no effect in this version)                                   */
 #define CULI_F_NO_NESTED 16u   /* run nested (non-top-level) ||| forms inside one thread (§8(f)1 off)     */
+#define CULI_F_NO_SPLIT  32u   /* no argument splitting: each form is evaluated by one thread only        */
 
 /* Fill *opts with defaults (device 0, default stream, default sizes). */
 void culi_default_opts(culi_opts* opts);
@@ -170,6 +171,11 @@ int culi_last_timing(const culi_ctx* ctx, float* ms3, uint32_t* kernels, uint64_
  * and forms re-evaluated sequentially (an element error, fuel overflow, a short / non-contiguous list). */
 int culi_last_stats(const culi_ctx* ctx, uint32_t* fanout_forms, uint32_t* fallback_forms,
                     uint32_t* nested_forms);
+/* Argument splitting (an implementation choice, not a paper mechanism): the number of
+ * split groups the last fetched batch published — each group is up to 32 pending arguments of one warp
+ * that an idle warp offered to evaluate (evaluated by it, or taken back by the owners).  Results, steps
+ * and errors are identical with CULI_F_NO_SPLIT. */
+int culi_last_splits(const culi_ctx* ctx, uint32_t* groups);
 
 #ifdef __cplusplus
 }

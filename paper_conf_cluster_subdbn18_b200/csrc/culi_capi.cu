@@ -92,6 +92,8 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   ok &= cudaMalloc(&c->nfallback, sizeof(uint32_t)) == cudaSuccess;
   ok &= cudaMalloc(&c->nnest, 2 * sizeof(uint32_t)) == cudaSuccess;
   ok &= cudaMalloc(&c->ndesc, (size_t)c->maxnest * sizeof(NestDesc)) == cudaSuccess;
+  ok &= cudaMalloc(&c->groups, (size_t)c->maxgroups * sizeof(SplitGroup)) == cudaSuccess;
+  ok &= cudaMalloc(&c->gcount, 4 * sizeof(uint32_t)) == cudaSuccess;
   for (int k = 0; k < 4 && ok; ++k) ok &= cudaEventCreate(&c->ev[k]) == cudaSuccess;
   if (!ok) { culi_shutdown(c); return CULI_E_CUDA; }
   c->H.cap = o.heap_nodes;
@@ -103,6 +105,8 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
              cudaMemcpyAsync(c->H.word, w01, 16, cudaMemcpyHostToDevice, c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->H.gtag, K_UNBOUND, GCAP, c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->flags, 0, 8 * sizeof(int), c->stream) == cudaSuccess &&
+             cudaMemsetAsync(c->groups, 0, (size_t)c->maxgroups * sizeof(SplitGroup), c->stream) == cudaSuccess &&
+             cudaMemsetAsync(c->gcount, 0, 4 * sizeof(uint32_t), c->stream) == cudaSuccess &&
              cudaStreamSynchronize(c->stream) == cudaSuccess;
   if (!ok2) { culi_shutdown(c); return CULI_E_CUDA; }
   *out = c;
@@ -128,6 +132,8 @@ void culi_shutdown(culi_ctx* c) {
   cudaFree(c->nfallback);
   cudaFree(c->nnest);
   cudaFree(c->ndesc);
+  cudaFree(c->groups);
+  cudaFree(c->gcount);
   cudaFree(c->kst2);
   cudaFree(c->vst2);
   c->fallback.release();
@@ -224,6 +230,13 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.kst2 = c->kst2;
   A.vst2 = c->vst2;
   A.finished = c->nnest + 1;
+  A.split = (!define_mode && !(c->opts.flags & CULI_F_NO_SPLIT)) ? 1 : 0;
+  A.split_poll = 16;
+  A.groups = c->groups;
+  A.gcount = c->gcount;
+  A.hungry = reinterpret_cast<int*>(c->gcount + 2);
+  A.maxgroups = c->maxgroups;
+  A.epoch = c->epoch;
   A.payload = c->payload.p;
   A.pcount = c->pcount;
   A.pcap = c->payload.n;
@@ -277,7 +290,7 @@ extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed
   rc = ensure_results(c, nf);
   if (rc) return rc;
   CK(launch_reset(c->stream, c->H.top, c->mark + img.tag.size(), c->next, c->pcount, c->flags, c->npend,
-                  c->nfallback, c->nnest));
+                  c->nfallback, c->nnest, c->gcount));
   EvalArgs A = make_args(c, nf, nullptr, 1);
   if (nf) CK(launch_define(c->stream, A));
   int flags[8];
@@ -304,7 +317,8 @@ static int run_batch_device(culi_ctx* c) {
   c->last_kernels = 0;
   CK(cudaEventRecord(c->ev[0], c->stream));
   CK(launch_reset(c->stream, c->H.top, c->mark + c->batch_nodes, c->next, c->pcount, c->flags, c->npend,
-                  c->nfallback, c->nnest));
+                  c->nfallback, c->nnest, c->gcount));
+  ++c->epoch;
   ++c->last_kernels;
   uint32_t* perm = nullptr;
   if (!(c->opts.flags & CULI_F_NO_BINNING) && nf > 1) {
@@ -318,8 +332,9 @@ static int run_batch_device(culi_ctx* c) {
   if (A.nest) { CK(launch_nest_clear(c->stream, c->ndesc, c->maxnest)); ++c->last_kernels; }
   uint32_t blocks = c->nslots / 128;
   uint32_t need = (nf + 127) / 128;
-  // a batch that may suspend on nested ||| keeps the whole grid: idle threads apply the elements
-  if (need < blocks && !A.nest) blocks = std::max<uint32_t>(need, 1);
+  // a batch that may suspend on nested ||| or split arguments keeps the whole grid: idle warps apply the
+  // elements / evaluate split-off arguments
+  if (need < blocks && !A.nest && !A.split) blocks = std::max<uint32_t>(need, 1);
   if (nf) { CK(launch_eval(c->stream, A, blocks)); ++c->last_kernels; }
   if (nf && A.fanout && c->batch_has_par) {            // ||| fan-out (a6) + finalize (a8)
     CK(launch_fanout(c->stream, A, c->nslots / 128));
@@ -412,6 +427,7 @@ static int rerun_fallback(culi_ctx* c, uint32_t nfb) {
   EvalArgs A = make_args(c, nfb, c->fallback.p, 0);
   A.fanout = 0;
   A.nest = 0;
+  A.split = 0;
   CK(launch_eval(c->stream, A, std::max<uint32_t>(1, std::min<uint32_t>(c->nslots / 128, (nfb + 127) / 128))));
   ExportArgs X{};
   X.tag = c->H.tag;
@@ -438,8 +454,9 @@ static int fetch(culi_ctx* c, culi_results** out) {
   for (int attempt = 0; attempt < 4; ++attempt) {
     int flags[8];
     unsigned long long pc = 0, top = 0;
-    uint32_t nfb = 0, npend = 0, nnest = 0;
+    uint32_t nfb = 0, npend = 0, nnest = 0, ngroups = 0;
     CK(cudaMemcpyAsync(&npend, c->npend, 4, cudaMemcpyDeviceToHost, c->stream));
+    if (attempt == 0) CK(cudaMemcpyAsync(&ngroups, c->gcount, 4, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(&nnest, c->nnest, 4, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(flags, c->flags, sizeof flags, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(&pc, c->pcount, 8, cudaMemcpyDeviceToHost, c->stream));
@@ -452,6 +469,7 @@ static int fetch(culi_ctx* c, culi_results** out) {
       c->last_fanout = (c->batch_has_par && !(c->opts.flags & CULI_F_NO_FANOUT)) ? std::min(npend, c->maxdesc) : 0;
       c->last_fallback = 0;
       c->last_nested = c->batch_may_nest ? std::min(nnest, c->maxnest) : 0;
+      c->last_splits = std::min(ngroups, c->maxgroups);
     }
     if (nfb && !flags[3]) {
       c->last_fallback += nfb;
@@ -620,6 +638,12 @@ int culi_last_stats(const culi_ctx* c, uint32_t* fanout_forms, uint32_t* fallbac
   if (nested_forms) *nested_forms = c->last_nested;
   if (fanout_forms) *fanout_forms = c->last_fanout;
   if (fallback_forms) *fallback_forms = c->last_fallback;
+  return CULI_OK;
+}
+
+int culi_last_splits(const culi_ctx* c, uint32_t* groups) {
+  if (!c || !groups) return CULI_E_ARG;
+  *groups = c->last_splits;
   return CULI_OK;
 }
 

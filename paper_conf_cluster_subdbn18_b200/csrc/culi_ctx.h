@@ -96,7 +96,12 @@ struct culi_ctx {
   uint32_t* nnest = nullptr;         // [0] descriptors written, [1] forms finished
   uint4* kst2 = nullptr;             // secondary stacks, allocated on first use
   uint4* vst2 = nullptr;
-  uint32_t last_fanout = 0, last_fallback = 0, last_nested = 0;
+  uint32_t last_fanout = 0, last_fallback = 0, last_nested = 0, last_splits = 0;
+  // argument splitting
+  SplitGroup* groups = nullptr;
+  uint32_t maxgroups = 16384;
+  uint32_t* gcount = nullptr;        // [0] groups allocated, [1] queue head, [2] hungry (int)
+  uint32_t epoch = 0;                // batch counter: a group is ready when its ready word == epoch
   DevBuf<uint32_t> wide;
   // uploaded batch (culi_upload)
   bool have_batch = false;

@@ -76,6 +76,13 @@ struct EvalArgs {
   uint32_t* finished;          // forms completed (threads without forms help until all are done)
   uint32_t code_lo, code_n;    // node range staged in shared memory (persistent code segment)
   uint32_t gst;                // global-frame entries staged in shared memory
+  uint32_t split;              // argument splitting: idle warps evaluate pending arguments of busy ones
+  uint32_t split_poll;         // closure calls between two polls of the idle-warp counter
+  struct SplitGroup* groups;   // published split groups (one task per lane of the forking warp)
+  uint32_t* gcount;            // [0] groups allocated, [1] queue head (next group a thief looks at)
+  int* hungry;                 // idle thief warps minus open groups (owners fork while > 0)
+  uint32_t maxgroups;
+  uint32_t epoch;              // this launch's batch number (SplitGroup.ready == epoch: published)
 };
 
 // One top-level (||| n f l1 .. lm) form whose arguments have been evaluated.
@@ -116,7 +123,27 @@ struct NestDesc {
   uint32_t sp, vtop;
   unsigned long long total;
   uint32_t next, done, bad, ready;            // ready: fields published, elements claimable
-};            // internal record tag: flat ||| result awaiting export
+};
+
+// Argument splitting.  A busy warp that sees idle warps turns the lowest pending
+// argument of each lane's K-stack (the biggest unevaluated chunk: the next argument of the outermost
+// KF_ARGS frame) into a task; an idle warp claims the whole group and lane i evaluates task i.  Arguments
+// are pure (no mutation inside a batch, c.3/c.13 #25), so only steps, the first error and fuel need care:
+// the owner adds the task's steps at the join and decides errors/fuel exactly (c.4, c.10).
+struct SplitTask {
+  uint32_t expr, env, depth, pad;      // argument node, heap env, depth of its evaluation
+  unsigned long long budget;           // fuel left at the fork
+  unsigned long long rw, rsteps;       // result word, steps
+  uint32_t rt, rerr, done, pad2;
+};
+struct SplitGroup {
+  uint32_t state;                      // 0 open, 1 claimed by a thief warp, 2 taken back by the owners
+  uint32_t ready;                      // tasks published
+  uint32_t mask;                       // lanes with a task
+  uint32_t form;
+  SplitTask t[32];
+};
+constexpr uint32_t SPLIT_OPEN = 0, SPLIT_CLAIMED = 1, SPLIT_TAKEN = 2;
 
 struct ExportArgs {
   const uint8_t* tag;
@@ -142,7 +169,7 @@ cudaError_t launch_define(cudaStream_t s, const EvalArgs& A);
 cudaError_t launch_export(cudaStream_t s, const ExportArgs& X, uint32_t blocks);
 cudaError_t launch_reset(cudaStream_t s, unsigned long long* top, unsigned long long top_value,
                          uint32_t* next, unsigned long long* pcount, int* flags, uint32_t* npend,
-                         uint32_t* nfallback, uint32_t* nnest);
+                         uint32_t* nfallback, uint32_t* nnest, uint32_t* gcount);
 cudaError_t launch_fanout(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
 cudaError_t launch_nest_clear(cudaStream_t s, struct NestDesc* d, uint32_t n);
 cudaError_t launch_flat_export(cudaStream_t s, const EvalArgs& A, uint32_t blocks);

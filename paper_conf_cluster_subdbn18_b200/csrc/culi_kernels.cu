@@ -48,9 +48,6 @@ __device__ __forceinline__ Ctx make_ctx(const EvalArgs& A, uint32_t slot) {
   return C;
 }
 
-// Batch mode.  Shared memory per block: the persistent code segment [code_lo, code_lo + code_n) as
-// {w.lo, w.hi, tag, 0} and the global frame [0, gst) (SURVEY §8(a)4: "stage").  Each warp takes 32
-// consecutive forms of the (binned) order with one atomicAdd and runs them to completion.
 // ---- nested |||: claim and apply one element of descriptor D ---------------------------
 // Runs on the thread's secondary stacks (C2).  Element i: f applied to (l1[i] .. lm[i]) at the depth of the
 // ||| call, with the fuel left when the owner suspended.  A failed contiguity check or an element error
@@ -101,7 +98,33 @@ __device__ __forceinline__ bool nest_help_any(const EvalArgs& A, const Ctx& C2, 
   return false;
 }
 
-template <bool FANOUT, bool NEST>
+// ---- argument splitting: a warp with no form left is a thief -----------------------------
+// It has offered itself (A.hungry += 1); lane 0 claims published groups in order (queue head A.gcount[1]).
+// Returns the group, or 0xffffffff once every form of the batch is finished.
+__device__ __noinline__ uint32_t split_claim(const EvalArgs& A) {
+  for (;;) {
+    uint32_t h = *(volatile uint32_t*)&A.gcount[1];
+    uint32_t n = *(volatile uint32_t*)&A.gcount[0];
+    if (n > A.maxgroups) n = A.maxgroups;
+    if (h < n) {
+      if (atomicCAS(&A.gcount[1], h, h + 1) == h) {
+        SplitGroup* G = A.groups + h;
+        while (ld_acquire(&G->ready) != A.epoch) __nanosleep(32);
+        if (atomicCAS(&G->state, SPLIT_OPEN, SPLIT_CLAIMED) == SPLIT_OPEN) return h;
+      }
+      continue;
+    }
+    if (*(volatile uint32_t*)A.finished >= A.nforms) return 0xffffffffu;
+    __nanosleep(256);
+  }
+}
+
+// Batch mode.  Shared memory per block: the persistent code segment [code_lo, code_lo + code_n) as
+// {w.lo, w.hi, tag, 0} and the global frame [0, gst) (SURVEY §8(a)4: "stage").  Each warp takes 32
+// consecutive forms of the (binned) order with one atomicAdd and runs them to completion.  With SPLIT, a
+// warp that finds no form left becomes a thief: lane i of it evaluates task i of a claimed split group on
+// the warp's own stacks (one eval_form call site serves forms and tasks).
+template <bool FANOUT, bool NEST, bool SPLIT>
 __global__ void __launch_bounds__(128, 4) culi_eval_kernel(const __grid_constant__ EvalArgs A) {
   uint4* scode = culi_smem;
   uint64_t* sgword = reinterpret_cast<uint64_t*>(culi_smem + A.code_n);
@@ -124,19 +147,51 @@ __global__ void __launch_bounds__(128, 4) culi_eval_kernel(const __grid_constant
     C2.vb = A.vst2 + slot;
   }
   int lane = threadIdx.x & 31;
+  bool forms_left = true;
   for (;;) {
-    uint32_t b = 0;
-    if (lane == 0) b = atomicAdd(A.next, 32u);
-    b = __shfl_sync(0xffffffffu, b, 0);
-    if (b >= A.nforms) break;
-    uint32_t i = b + lane;
-    if (i < A.nforms) {
-      uint32_t f = A.perm ? A.perm[i] : i;
+    uint32_t f = 0, root = 0, env = 0, d = 1;
+    uint64_t fuel = A.fuel;
+    bool run;
+    SplitTask* T = nullptr;
+    if (!SPLIT || forms_left) {
+      uint32_t b = 0;
+      if (lane == 0) b = atomicAdd(A.next, 32u);
+      b = __shfl_sync(0xffffffffu, b, 0);
+      if (b >= A.nforms) {
+        if (!SPLIT) break;
+        forms_left = false;
+        if (lane == 0) atomicAdd(A.hungry, 1);                 // offer this warp to the busy ones
+        continue;
+      }
+      uint32_t i = b + lane;
+      run = i < A.nforms;
+      if (run) {
+        f = A.perm ? A.perm[i] : i;
+        root = A.roots[f];
+      }
+    } else {
+      uint32_t g = 0;
+      if (lane == 0) g = split_claim(A);
+      g = __shfl_sync(0xffffffffu, g, 0);
+      if (g == 0xffffffffu) break;
+      SplitGroup* G = A.groups + g;
+      ld_acquire(&G->ready);                                   // acquire the owners' task and env writes
+      run = (G->mask >> lane) & 1u;
+      if (run) {
+        T = &G->t[lane];
+        f = G->form;
+        root = T->expr;
+        env = T->env;
+        d = T->depth;
+        fuel = T->budget;
+      }
+    }
+    if (run) {
       FormOut o;
       bool resume = false;
       Resume R{};
       for (;;) {
-        o = eval_form<FANOUT, false, NEST>(C, A.roots[f], f, 0, 0, A.fuel, 1, resume, R);
+        o = eval_form<FANOUT, false, NEST, SPLIT>(C, root, f, 0, 0, fuel, d, resume, R, env);
         if (!NEST || o.err != E_SUSPEND) break;
         NestDesc* D = A.ndesc + o.aux;                  // suspended on a nested |||: help until done
         while (*(volatile uint32_t*)&D->done < D->n)
@@ -154,8 +209,21 @@ __global__ void __launch_bounds__(128, 4) culi_eval_kernel(const __grid_constant
         R.v = mkv(K_CONS, D->spine);
         resume = true;
       }
-      write_result(A, f, o);
-      if (NEST) atomicAdd(A.finished, 1u);
+      if (SPLIT && T) {                                 // a split-off argument: hand it to its owner
+        T->rt = o.t;
+        T->rw = o.w;
+        T->rsteps = o.steps;
+        T->rerr = o.err;
+        __threadfence();
+        st_release(&T->done, 1u);
+      } else {
+        write_result(A, f, o);
+        if (NEST || SPLIT) atomicAdd(A.finished, 1u);
+      }
+    }
+    if (SPLIT && !forms_left) {
+      __syncwarp();
+      if (lane == 0) atomicAdd(A.hungry, 1);                   // ready for the next group
     }
   }
   if (NEST) {                                           // no forms left: help until every form is done
@@ -234,8 +302,9 @@ __global__ void __launch_bounds__(128) culi_export_kernel(ExportArgs X) {
 
 __global__ void culi_reset_kernel(unsigned long long* top, unsigned long long top_value, uint32_t* next,
                                   unsigned long long* pcount, int* flags, uint32_t* npend,
-                                  uint32_t* nfallback, uint32_t* nnest) {
+                                  uint32_t* nfallback, uint32_t* nnest, uint32_t* gcount) {
   *top = top_value;
+  if (gcount) { gcount[0] = 0; gcount[1] = 0; gcount[2] = 0; }
   *next = 0;
   *pcount = 0;
   *npend = 0;
@@ -440,18 +509,18 @@ size_t eval_smem_bytes(const EvalArgs& A) {
 
 cudaError_t launch_eval(cudaStream_t s, const EvalArgs& A, uint32_t blocks) {
   size_t smem = eval_smem_bytes(A);
+  // specialised on whether the batch holds top-level ||| / wide forms (FANOUT), whether ||| can occur
+  // below the top level (NEST) and whether idle warps split arguments off busy ones (SPLIT; not combined
+  // with NEST, whose helpers use the idle warps)
+  void (*k)(EvalArgs);
+  if (A.nest) k = A.fanout ? culi_eval_kernel<true, true, false> : culi_eval_kernel<false, true, false>;
+  else if (A.split) k = A.fanout ? culi_eval_kernel<true, false, true> : culi_eval_kernel<false, false, true>;
+  else k = A.fanout ? culi_eval_kernel<true, false, false> : culi_eval_kernel<false, false, false>;
   if (smem > 48 * 1024) {
-    void (*k)(EvalArgs) = A.fanout ? (A.nest ? culi_eval_kernel<true, true> : culi_eval_kernel<true, false>)
-                                   : (A.nest ? culi_eval_kernel<false, true> : culi_eval_kernel<false, false>);
     cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     if (e != cudaSuccess) return e;
   }
-  // specialised on whether the batch holds top-level ||| / wide forms (FANOUT) and whether ||| can occur
-  // below the top level (NEST): batches without them run the lean kernel
-  if (A.fanout && A.nest) culi_eval_kernel<true, true><<<blocks, 128, smem, s>>>(A);
-  else if (A.fanout) culi_eval_kernel<true, false><<<blocks, 128, smem, s>>>(A);
-  else if (A.nest) culi_eval_kernel<false, true><<<blocks, 128, smem, s>>>(A);
-  else culi_eval_kernel<false, false><<<blocks, 128, smem, s>>>(A);
+  k<<<blocks, 128, smem, s>>>(A);
   return cudaGetLastError();
 }
 
@@ -467,8 +536,8 @@ cudaError_t launch_export(cudaStream_t s, const ExportArgs& X, uint32_t blocks) 
 
 cudaError_t launch_reset(cudaStream_t s, unsigned long long* top, unsigned long long top_value,
                          uint32_t* next, unsigned long long* pcount, int* flags, uint32_t* npend,
-                         uint32_t* nfallback, uint32_t* nnest) {
-  culi_reset_kernel<<<1, 1, 0, s>>>(top, top_value, next, pcount, flags, npend, nfallback, nnest);
+                         uint32_t* nfallback, uint32_t* nnest, uint32_t* gcount) {
+  culi_reset_kernel<<<1, 1, 0, s>>>(top, top_value, next, pcount, flags, npend, nfallback, nnest, gcount);
   return cudaGetLastError();
 }
 

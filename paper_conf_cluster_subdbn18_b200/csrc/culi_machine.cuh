@@ -726,7 +726,76 @@ __device__ __forceinline__ int try_leaf(const Ctx& C, uint32_t xt, uint64_t xw, 
 }
 
 // ---- the machine ---------------------------------------------------------------------------------------
-enum KKind : uint32_t { KF_HEAD = 1, KF_ARGS, KF_BODY, KF_IF, KF_LET, KF_DEFINE, KF_MACRO, KF_PAR, KF_DATA };
+enum KKind : uint32_t { KF_HEAD = 1, KF_ARGS, KF_BODY, KF_IF, KF_LET, KF_DEFINE, KF_MACRO, KF_PAR, KF_DATA,
+                       KF_JOIN };   // KF_JOIN: a KF_ARGS frame whose next argument was split off
+
+// ---- argument splitting ----------------------------------------------------------------
+__device__ __forceinline__ uint32_t ld_acquire(const uint32_t* p) {
+  uint32_t v;
+  asm volatile("ld.acquire.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ void st_release(uint32_t* p, uint32_t v) {
+  asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+
+// Called by the lanes of a warp at a poll point (their top continuation already flushed to memory).  If an
+// idle warp is waiting (a token in A.hungry), each lane looks for the outermost KF_ARGS frame whose next
+// argument is an unevaluated list, copies that frame's environment to the heap (promote) and publishes
+// the argument as task `lane` of one group; the frame becomes KF_JOIN and its V-stack header records the
+// group.  The owner later joins (RET KF_JOIN): it takes the group back if no thief claimed it.
+__device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t fuel, uint32_t form) {
+  const EvalArgs& A = *C.A;
+  unsigned mask = __activemask();
+  int lane = threadIdx.x & 31;
+  int leader = __ffs(mask) - 1;
+  int tok = 0;
+  if (lane == leader && *(volatile int*)A.hungry > 0) {
+    if (atomicSub(A.hungry, 1) > 0) tok = 1;
+    else atomicAdd(A.hungry, 1);
+  }
+  tok = __shfl_sync(mask, tok, leader);
+  if (!tok) return;
+  uint32_t lvl = 0xffffffffu, henv = 0;
+  uint4 fr = make_uint4(0, 0, 0, 0);
+  for (uint32_t i = 0; i < sp; ++i) {
+    uint4 f = *KS(C, i);
+    if (kkind(f.w) == KF_ARGS && f.x != 0 && (ntag(C, car_of(C, f.x)) & KIND_MASK) == K_CONS) {
+      lvl = i;
+      fr = f;
+      break;
+    }
+  }
+  bool have = lvl != 0xffffffffu && promote(C, fr.y, &henv);
+  unsigned part = __ballot_sync(mask, have);
+  uint32_t g = 0xffffffffu;
+  if (lane == leader && part) g = atomicAdd(A.gcount, 1u);
+  g = __shfl_sync(mask, g, leader);
+  if (!part || g >= A.maxgroups) {                              // nothing to split: return the token
+    if (lane == leader) atomicAdd(A.hungry, 1);
+    return;
+  }
+  SplitGroup* G = A.groups + g;
+  if (have) {
+    SplitTask* T = &G->t[lane];
+    T->expr = car_of(C, fr.x);
+    T->env = henv;
+    T->depth = kdepth(fr.w) + 1;                                // arguments run at depth d + 1
+    T->budget = fuel - steps;
+    T->done = 0;
+    KS(C, lvl)->w = (fr.w & ~(0xfu << 12)) | (KF_JOIN << 12);
+    VS(C, fr.z)->z = g + 1;                                     // the call's header: the group
+  }
+  __syncwarp(mask);
+  if (lane == leader) {
+    G->state = SPLIT_OPEN;
+    G->mask = part;
+    G->form = form;
+    __threadfence();
+    st_release(&G->ready, A.epoch);
+  }
+  __syncwarp(mask);
+}
 
 struct FormOut {
   uint32_t t;
@@ -746,15 +815,17 @@ struct Resume {
 // eval_form(C, root, form, 0, 0, fuel): evaluate the datum at node `root` at depth 1.
 // eval_form(C, 0, form, 1, m, budget): apply vs[0] to the m values vs[1..m] as the body of a top-level
 //   (||| ...) form (depth 1) — one fan-out element (c.7); `budget` = fuel left after the ||| arguments.
-template <bool FANOUT, bool APPLY, bool NEST = false>
+// eval_form<..., SPLIT>(C, root, form, 0, 0, budget, depth, false, {}, env): a split-off argument task.
+template <bool FANOUT, bool APPLY, bool NEST = false, bool SPLIT = false>
 __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32_t form, int apply_mode,
                                              uint32_t apply_cnt, uint64_t fuel, uint32_t d0 = 1,
-                                             bool resume = false, const Resume& R = Resume{}) {
+                                             bool resume = false, const Resume& R = Resume{},
+                                             uint32_t env0 = 0) {
   const DevHeap& H = C.A->H;
   const uint32_t kcap = C.A->kcap, vcap = C.A->vcap, maxd = C.A->max_depth;
   const bool fanout = FANOUT && !APPLY && C.A->fanout;
   V v = mkv(K_NIL, 0), a0 = mkv(K_NIL, 0), a1 = mkv(K_NIL, 0);
-  uint32_t x = root, t = 0, env = 0, d = d0, cur = 0, base = 0, cnt = 0, sp = 0, vtop = 0;
+  uint32_t x = root, t = 0, env = env0, d = d0, cur = 0, base = 0, cnt = 0, sp = 0, vtop = 0;
   uint32_t a = 0, at = 0, nxt = 0, kd = 0, hop = 0;
   uint64_t w = 0, aw = 0, w0 = 0;
   uint64_t steps = 0;
@@ -762,6 +833,7 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32
   uint4 k, ktop = make_uint4(0, 0, 0, 0);
   uint4 hv = make_uint4(0, 0, 0, 0);      // the value being applied (copy of vs[base])
   bool kdirty = false;                      // ktop holds frame sp-1 not yet written to memory
+  uint32_t pollc = SPLIT ? C.A->split_poll : 0;   // closure calls until the next split poll
 
 #define FAIL(e) do { err = (e); goto done; } while (0)
 #define STEP(depth)                                     \
@@ -1055,6 +1127,13 @@ ARGS:
 APPLY: {                                                        // apply vs[base] to cnt args
   V h = vunpack(hv);
   if (h.t == K_CLOSURE) {                                       // PAPER L456-460, c.4 CLOSURE
+    if (SPLIT && __builtin_expect(--pollc == 0, 0)) {
+      pollc = C.A->split_poll;
+      if (kdirty) *KS(C, sp - 1) = ktop;
+      kdirty = false;
+      try_split(C, sp, steps, fuel, form);
+      if (sp > 0) ktop = *KS(C, sp - 1);                        // the top frame may have become KF_JOIN
+    }
     uint64_t cwd = nword(C, (uint32_t)h.w);                     // three independent loads
     uint64_t aux = nword(C, (uint32_t)h.w + 1);
     uint64_t aux2 = nword(C, (uint32_t)h.w + 2);
@@ -1299,6 +1378,33 @@ RET:
     case KF_IF:
       vtop = k.z; cur = k.x; env = k.y; d = kd;
       goto IF_BRANCH;
+    case KF_JOIN: {                                             // argument `cnt + 1` was split off
+      base = k.z; cnt = kcount(k.w);
+      hv = *VS(C, base);
+      if (__builtin_expect(!!(base + 2 + cnt >= vcap), 0)) FAIL(E_OOM);
+      *VS(C, base + 1 + cnt) = vpack(v, 0);
+      ++cnt;
+      cur = k.x; env = k.y; d = kd;
+      SplitGroup* G = C.A->groups + (hv.z - 1);
+      uint32_t st = ld_acquire(&G->state);
+      if (st == SPLIT_OPEN) {                                   // unclaimed: take it back, evaluate here
+        st = atomicCAS(&G->state, SPLIT_OPEN, SPLIT_TAKEN);
+        if (st == SPLIT_OPEN) { atomicAdd(C.A->hungry, 1); st = SPLIT_TAKEN; }
+      }
+      if (st == SPLIT_TAKEN) goto ARGS;
+      SplitTask* T = &G->t[threadIdx.x & 31];
+      while (ld_acquire(&T->done) == 0) __nanosleep(200);
+      uint64_t ts = T->rsteps;
+      uint32_t te = T->rerr;
+      // c.10: the sequential count at the end of this argument is steps + ts; fuel is checked first
+      if (te == E_FUEL || steps + ts > fuel) { err = E_FUEL; steps = fuel + 1; goto done; }
+      steps += ts;
+      if (te) FAIL((uint8_t)te);
+      *VS(C, base + 1 + cnt) = vpack(mkv(T->rt, T->rw), 0);
+      ++cnt;
+      cur = cdr_of(C, cur);
+      goto ARGS;
+    }
     case KF_BODY:
       vtop = k.z; cur = k.x; env = k.y; d = kd;
       goto BODY;

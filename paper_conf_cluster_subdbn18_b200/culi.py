@@ -22,6 +22,7 @@ CULI_F_NO_FANOUT = 2
 CULI_F_NO_STAGING = 4
 CULI_F_NO_VOTING = 8
 CULI_F_NO_NESTED = 16
+CULI_F_NO_SPLIT = 32
 
 SYMBOLS = [
     "culi_default_opts", "culi_init", "culi_shutdown", "culi_read", "culi_image_nforms",
@@ -30,7 +31,7 @@ SYMBOLS = [
     "culi_result_int", "culi_result_float", "culi_print", "culi_results_totals", "culi_results_free",
     "culi_env_export", "culi_env_import", "culi_results_serialize", "culi_results_merge",
     "culi_status_string", "culi_error_name", "culi_last_timing", "culi_records_device",
-    "culi_last_stats", "culi_image_pin", "culi_results_wire_bytes",
+    "culi_last_stats", "culi_last_splits", "culi_image_pin", "culi_results_wire_bytes",
 ]
 
 
@@ -89,6 +90,7 @@ def load(path: str = LIB_PATH) -> ctypes.CDLL:
         "culi_last_timing": (I, [P, pp(ctypes.c_float), pp(U32), pp(U64)]),
         "culi_records_device": (I, [P, P, SZ, pp(SZ)]),
         "culi_last_stats": (I, [P, pp(U32), pp(U32), pp(U32)]),
+        "culi_last_splits": (I, [P, pp(U32)]),
         "culi_image_pin": (I, [P, pp(U64)]),
         "culi_results_wire_bytes": (I, [P, pp(U64)]),
     }
@@ -307,6 +309,12 @@ class Context:
                "culi_last_stats")
         self.last_nested = c.value
         return a.value, b.value
+
+    def last_splits(self) -> int:
+        """Split groups published by the last batch (argument splitting)."""
+        g = ctypes.c_uint32()
+        _check(load().culi_last_splits(self._p, ctypes.byref(g)), "culi_last_splits")
+        return g.value
 
     def records_device(self, dev_ptr: int | None, cap: int = 0) -> int:
         need = ctypes.c_size_t(0)
