@@ -4,6 +4,7 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <cstdlib>
 #include <cstring>
 #include <memory>
 #include <new>
@@ -75,6 +76,8 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   c->kcap = 2 * o.max_depth + 8;
   c->vcap = o.vstack_entries;
   c->stream = (cudaStream_t)o.stream;
+  if (const char* e = getenv("CULI_SPLIT_POLL")) c->split_poll = std::max(1, atoi(e));      // tuning knobs
+  if (const char* e = getenv("CULI_SPLIT_SLEEP")) c->split_sleep = std::max(32, atoi(e));
   bool ok = true;
   ok &= cudaMalloc(&c->H.tag, o.heap_nodes) == cudaSuccess;
   ok &= cudaMalloc(&c->H.word, o.heap_nodes * 8) == cudaSuccess;
@@ -92,7 +95,8 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   ok &= cudaMalloc(&c->nfallback, sizeof(uint32_t)) == cudaSuccess;
   ok &= cudaMalloc(&c->nnest, 2 * sizeof(uint32_t)) == cudaSuccess;
   ok &= cudaMalloc(&c->ndesc, (size_t)c->maxnest * sizeof(NestDesc)) == cudaSuccess;
-  ok &= cudaMalloc(&c->groups, (size_t)c->maxgroups * sizeof(SplitGroup)) == cudaSuccess;
+  ok &= cudaMalloc(&c->groups, (size_t)c->nslots / 32 * SPLIT_GPW * sizeof(SplitGroup)) == cudaSuccess;
+  ok &= cudaMalloc(&c->gqueue, (size_t)c->gqcap * sizeof(uint32_t)) == cudaSuccess;
   ok &= cudaMalloc(&c->gcount, 4 * sizeof(uint32_t)) == cudaSuccess;
   for (int k = 0; k < 4 && ok; ++k) ok &= cudaEventCreate(&c->ev[k]) == cudaSuccess;
   if (!ok) { culi_shutdown(c); return CULI_E_CUDA; }
@@ -105,7 +109,8 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
              cudaMemcpyAsync(c->H.word, w01, 16, cudaMemcpyHostToDevice, c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->H.gtag, K_UNBOUND, GCAP, c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->flags, 0, 8 * sizeof(int), c->stream) == cudaSuccess &&
-             cudaMemsetAsync(c->groups, 0, (size_t)c->maxgroups * sizeof(SplitGroup), c->stream) == cudaSuccess &&
+             cudaMemsetAsync(c->groups, 0xff, (size_t)c->nslots / 32 * SPLIT_GPW * sizeof(SplitGroup), c->stream) == cudaSuccess &&
+             cudaMemsetAsync(c->gqueue, 0, (size_t)c->gqcap * sizeof(uint32_t), c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->gcount, 0, 4 * sizeof(uint32_t), c->stream) == cudaSuccess &&
              cudaStreamSynchronize(c->stream) == cudaSuccess;
   if (!ok2) { culi_shutdown(c); return CULI_E_CUDA; }
@@ -133,6 +138,7 @@ void culi_shutdown(culi_ctx* c) {
   cudaFree(c->nnest);
   cudaFree(c->ndesc);
   cudaFree(c->groups);
+  cudaFree(c->gqueue);
   cudaFree(c->gcount);
   cudaFree(c->kst2);
   cudaFree(c->vst2);
@@ -231,12 +237,13 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.vst2 = c->vst2;
   A.finished = c->nnest + 1;
   A.split = (!define_mode && !(c->opts.flags & CULI_F_NO_SPLIT)) ? 1 : 0;
-  A.split_poll = 16;
+  A.split_poll = c->split_poll;
+  A.split_sleep = c->split_sleep;
   A.groups = c->groups;
+  A.gqueue = c->gqueue;
+  A.gqcap = c->gqcap;
   A.gcount = c->gcount;
   A.hungry = reinterpret_cast<int*>(c->gcount + 2);
-  A.maxgroups = c->maxgroups;
-  A.epoch = c->epoch;
   A.payload = c->payload.p;
   A.pcount = c->pcount;
   A.pcap = c->payload.n;
@@ -318,7 +325,6 @@ static int run_batch_device(culi_ctx* c) {
   CK(cudaEventRecord(c->ev[0], c->stream));
   CK(launch_reset(c->stream, c->H.top, c->mark + c->batch_nodes, c->next, c->pcount, c->flags, c->npend,
                   c->nfallback, c->nnest, c->gcount));
-  ++c->epoch;
   ++c->last_kernels;
   uint32_t* perm = nullptr;
   if (!(c->opts.flags & CULI_F_NO_BINNING) && nf > 1) {
@@ -469,7 +475,7 @@ static int fetch(culi_ctx* c, culi_results** out) {
       c->last_fanout = (c->batch_has_par && !(c->opts.flags & CULI_F_NO_FANOUT)) ? std::min(npend, c->maxdesc) : 0;
       c->last_fallback = 0;
       c->last_nested = c->batch_may_nest ? std::min(nnest, c->maxnest) : 0;
-      c->last_splits = std::min(ngroups, c->maxgroups);
+      c->last_splits = ngroups;
     }
     if (nfb && !flags[3]) {
       c->last_fallback += nfb;

@@ -98,10 +98,12 @@ struct culi_ctx {
   uint4* vst2 = nullptr;
   uint32_t last_fanout = 0, last_fallback = 0, last_nested = 0, last_splits = 0;
   // argument splitting
-  SplitGroup* groups = nullptr;
-  uint32_t maxgroups = 16384;
-  uint32_t* gcount = nullptr;        // [0] groups allocated, [1] queue head, [2] hungry (int)
-  uint32_t epoch = 0;                // batch counter: a group is ready when its ready word == epoch
+  SplitGroup* groups = nullptr;      // SPLIT_GPW per warp of the grid
+  uint32_t* gqueue = nullptr;
+  uint32_t gqcap = 1u << 18;
+  uint32_t* gcount = nullptr;        // [0] queue tail (groups published), [1] queue head, [2] hungry (int)
+  uint32_t split_poll = 64;          // closure calls between polls (env CULI_SPLIT_POLL)
+  uint32_t split_sleep = 4096;       // idle-warp back-off cap in ns (env CULI_SPLIT_SLEEP)
   DevBuf<uint32_t> wide;
   // uploaded batch (culi_upload)
   bool have_batch = false;

@@ -78,11 +78,12 @@ struct EvalArgs {
   uint32_t gst;                // global-frame entries staged in shared memory
   uint32_t split;              // argument splitting: idle warps evaluate pending arguments of busy ones
   uint32_t split_poll;         // closure calls between two polls of the idle-warp counter
-  struct SplitGroup* groups;   // published split groups (one task per lane of the forking warp)
-  uint32_t* gcount;            // [0] groups allocated, [1] queue head (next group a thief looks at)
-  int* hungry;                 // idle thief warps minus open groups (owners fork while > 0)
-  uint32_t maxgroups;
-  uint32_t epoch;              // this launch's batch number (SplitGroup.ready == epoch: published)
+  uint32_t split_sleep;        // longest back-off (ns) of an idle warp polling for split groups
+  struct SplitGroup* groups;   // SPLIT_GPW group slots per warp of the grid (slot reused after its join)
+  uint32_t* gqueue;            // ring of published group ids + 1 (0 = empty), gqcap entries
+  uint32_t gqcap;              // power of two
+  uint32_t* gcount;            // [0] queue tail (groups published), [1] queue head (next entry a thief takes)
+  int* hungry;                 // idle thief warps minus open groups (owners split while > 0)
 };
 
 // One top-level (||| n f l1 .. lm) form whose arguments have been evaluated.
@@ -138,11 +139,12 @@ struct SplitTask {
 };
 struct SplitGroup {
   uint32_t state;                      // 0 open, 1 claimed by a thief warp, 2 taken back by the owners
-  uint32_t ready;                      // tasks published
+  uint32_t remaining;                  // owner lanes that have not joined yet (0: the slot is free again)
   uint32_t mask;                       // lanes with a task
   uint32_t form;
   SplitTask t[32];
 };
+constexpr uint32_t SPLIT_GPW = 8;      // group slots per warp
 constexpr uint32_t SPLIT_OPEN = 0, SPLIT_CLAIMED = 1, SPLIT_TAKEN = 2;
 
 struct ExportArgs {

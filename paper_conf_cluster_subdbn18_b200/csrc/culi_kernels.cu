@@ -101,21 +101,28 @@ __device__ __forceinline__ bool nest_help_any(const EvalArgs& A, const Ctx& C2, 
 // ---- argument splitting: a warp with no form left is a thief -----------------------------
 // It has offered itself (A.hungry += 1); lane 0 claims published groups in order (queue head A.gcount[1]).
 // Returns the group, or 0xffffffff once every form of the batch is finished.
+// Idle warps back off exponentially (up to A.split_sleep ns) so that they do not hammer the L2 line of the
+// queue counters.  A queue entry whose group is no longer open (taken back, or reused and already
+// claimed) is skipped.
 __device__ __noinline__ uint32_t split_claim(const EvalArgs& A) {
+  uint32_t ns = 64;
   for (;;) {
     uint32_t h = *(volatile uint32_t*)&A.gcount[1];
     uint32_t n = *(volatile uint32_t*)&A.gcount[0];
-    if (n > A.maxgroups) n = A.maxgroups;
     if (h < n) {
       if (atomicCAS(&A.gcount[1], h, h + 1) == h) {
-        SplitGroup* G = A.groups + h;
-        while (ld_acquire(&G->ready) != A.epoch) __nanosleep(32);
-        if (atomicCAS(&G->state, SPLIT_OPEN, SPLIT_CLAIMED) == SPLIT_OPEN) return h;
+        uint32_t* qe = &A.gqueue[h & (A.gqcap - 1)];
+        uint32_t e;
+        while ((e = ld_acquire(qe)) == 0) __nanosleep(32);
+        *qe = 0;
+        if (atomicCAS(&A.groups[e - 1].state, SPLIT_OPEN, SPLIT_CLAIMED) == SPLIT_OPEN) return e - 1;
       }
+      ns = 64;
       continue;
     }
     if (*(volatile uint32_t*)A.finished >= A.nforms) return 0xffffffffu;
-    __nanosleep(256);
+    __nanosleep(ns);
+    ns = ns * 2 > A.split_sleep ? A.split_sleep : ns * 2;
   }
 }
 
@@ -137,6 +144,7 @@ __global__ void __launch_bounds__(128, 4) culi_eval_kernel(const __grid_constant
     sgword[i] = A.H.gword[i];
     sgtag[i] = A.H.gtag[i];
   }
+  if (SPLIT && threadIdx.x < 4) culi_split_busy[threadIdx.x] = 0;
   __syncthreads();
   uint32_t slot = blockIdx.x * blockDim.x + threadIdx.x;
   Ctx C = make_ctx(A, slot);
@@ -175,7 +183,7 @@ __global__ void __launch_bounds__(128, 4) culi_eval_kernel(const __grid_constant
       g = __shfl_sync(0xffffffffu, g, 0);
       if (g == 0xffffffffu) break;
       SplitGroup* G = A.groups + g;
-      ld_acquire(&G->ready);                                   // acquire the owners' task and env writes
+      ld_acquire(&G->state);                                   // acquire the owners' task and env writes
       run = (G->mask >> lane) & 1u;
       if (run) {
         T = &G->t[lane];

@@ -739,23 +739,36 @@ __device__ __forceinline__ void st_release(uint32_t* p, uint32_t v) {
   asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
 }
 
+// In-use bits of the SPLIT_GPW group slots of each warp of the block (the block has 4 warps); cleared by
+// the kernel prologue, set by try_split, cleared by the last owner lane that joins the group.
+__shared__ uint32_t culi_split_busy[4];
+
 // Called by the lanes of a warp at a poll point (their top continuation already flushed to memory).  If an
-// idle warp is waiting (a token in A.hungry), each lane looks for the outermost KF_ARGS frame whose next
-// argument is an unevaluated list, copies that frame's environment to the heap (promote) and publishes
-// the argument as task `lane` of one group; the frame becomes KF_JOIN and its V-stack header records the
-// group.  The owner later joins (RET KF_JOIN): it takes the group back if no thief claimed it.
+// idle warp is waiting (a token in A.hungry) and the warp has a free group slot, each lane looks for the
+// outermost KF_ARGS frame whose next argument is an unevaluated list, copies that frame's environment to
+// the heap (promote) and publishes the argument as task `lane` of the group; the frame becomes KF_JOIN and
+// its V-stack header records the group.  The owner later joins (RET KF_JOIN): it takes the group back if
+// no thief claimed it.
 __device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t fuel, uint32_t form) {
   const EvalArgs& A = *C.A;
   unsigned mask = __activemask();
   int lane = threadIdx.x & 31;
   int leader = __ffs(mask) - 1;
-  int tok = 0;
+  uint32_t* busy = &culi_split_busy[threadIdx.x >> 5];
+  int j = -1;
   if (lane == leader && *(volatile int*)A.hungry > 0) {
-    if (atomicSub(A.hungry, 1) > 0) tok = 1;
-    else atomicAdd(A.hungry, 1);
+    uint32_t freeb = ~*(volatile uint32_t*)busy & ((1u << SPLIT_GPW) - 1u);
+    if (freeb) {
+      if (atomicSub(A.hungry, 1) > 0) {
+        j = __ffs(freeb) - 1;
+        atomicOr(busy, 1u << j);
+      } else {
+        atomicAdd(A.hungry, 1);
+      }
+    }
   }
-  tok = __shfl_sync(mask, tok, leader);
-  if (!tok) return;
+  j = __shfl_sync(mask, j, leader);
+  if (j < 0) return;
   uint32_t lvl = 0xffffffffu, henv = 0;
   uint4 fr = make_uint4(0, 0, 0, 0);
   for (uint32_t i = 0; i < sp; ++i) {
@@ -768,14 +781,16 @@ __device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t
   }
   bool have = lvl != 0xffffffffu && promote(C, fr.y, &henv);
   unsigned part = __ballot_sync(mask, have);
-  uint32_t g = 0xffffffffu;
-  if (lane == leader && part) g = atomicAdd(A.gcount, 1u);
-  g = __shfl_sync(mask, g, leader);
-  if (!part || g >= A.maxgroups) {                              // nothing to split: return the token
-    if (lane == leader) atomicAdd(A.hungry, 1);
+  if (!part) {                                                  // nothing to split: return slot and token
+    if (lane == leader) {
+      atomicAnd(busy, ~(1u << j));
+      atomicAdd(A.hungry, 1);
+    }
     return;
   }
+  uint32_t g = (blockIdx.x * blockDim.x + threadIdx.x) / 32 * SPLIT_GPW + (uint32_t)j;
   SplitGroup* G = A.groups + g;
+  if (lane == leader) G->state = SPLIT_TAKEN;                   // not claimable while it is rewritten
   if (have) {
     SplitTask* T = &G->t[lane];
     T->expr = car_of(C, fr.x);
@@ -788,13 +803,21 @@ __device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t
   }
   __syncwarp(mask);
   if (lane == leader) {
-    G->state = SPLIT_OPEN;
     G->mask = part;
+    G->remaining = __popc(part);
     G->form = form;
     __threadfence();
-    st_release(&G->ready, A.epoch);
+    st_release(&G->state, SPLIT_OPEN);
+    uint32_t q = atomicAdd(&A.gcount[0], 1u);
+    st_release(&A.gqueue[q & (A.gqcap - 1)], g + 1);
   }
   __syncwarp(mask);
+}
+
+// the owner lane is done with group G (joined): the last one frees the warp's slot
+__device__ __forceinline__ void split_release(const EvalArgs& A, uint32_t g) {
+  if (atomicSub(&A.groups[g].remaining, 1u) == 1u)
+    atomicAnd(&culi_split_busy[threadIdx.x >> 5], ~(1u << (g % SPLIT_GPW)));
 }
 
 struct FormOut {
@@ -1385,22 +1408,25 @@ RET:
       *VS(C, base + 1 + cnt) = vpack(v, 0);
       ++cnt;
       cur = k.x; env = k.y; d = kd;
-      SplitGroup* G = C.A->groups + (hv.z - 1);
+      uint32_t g = hv.z - 1;
+      SplitGroup* G = C.A->groups + g;
       uint32_t st = ld_acquire(&G->state);
       if (st == SPLIT_OPEN) {                                   // unclaimed: take it back, evaluate here
         st = atomicCAS(&G->state, SPLIT_OPEN, SPLIT_TAKEN);
         if (st == SPLIT_OPEN) { atomicAdd(C.A->hungry, 1); st = SPLIT_TAKEN; }
       }
-      if (st == SPLIT_TAKEN) goto ARGS;
+      if (st == SPLIT_TAKEN) { split_release(*C.A, g); goto ARGS; }
       SplitTask* T = &G->t[threadIdx.x & 31];
       while (ld_acquire(&T->done) == 0) __nanosleep(200);
       uint64_t ts = T->rsteps;
       uint32_t te = T->rerr;
+      V tv = mkv(T->rt, T->rw);
+      split_release(*C.A, g);
       // c.10: the sequential count at the end of this argument is steps + ts; fuel is checked first
       if (te == E_FUEL || steps + ts > fuel) { err = E_FUEL; steps = fuel + 1; goto done; }
       steps += ts;
       if (te) FAIL((uint8_t)te);
-      *VS(C, base + 1 + cnt) = vpack(mkv(T->rt, T->rw), 0);
+      *VS(C, base + 1 + cnt) = vpack(tv, 0);
       ++cnt;
       cur = cdr_of(C, cur);
       goto ARGS;

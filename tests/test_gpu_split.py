@@ -65,7 +65,7 @@ def test_split_errors_first_in_order(culi, oracle_mod):
     assert splits > 0
 
 
-@pytest.mark.parametrize("fuel", [2, 60000, 112871, 112873, 130000, 182622, 182623, 182624, 1 << 40])
+@pytest.mark.parametrize("fuel", [10, 60000, 112871, 112873, 130000, 182622, 182623, 182624, 1 << 40])
 def test_split_fuel_limit(culi, oracle_mod, fuel):
     """fuel runs out before, inside or exactly at the end of a split-off argument (c.10)"""
     # (+ (fib 18) (fib 17)): 2 + S(18) + S(17) = 2 + 112,870 + 69,751 = 182,623 steps
