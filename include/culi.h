@@ -69,7 +69,7 @@ typedef struct {
   uint32_t max_depth;      /* canonical eval-nesting limit (c.10); 0 = default 1024; at most 4095         */
   uint64_t fuel;           /* canonical step limit per top-level form (c.10); 0 = default 2^40            */
   uint32_t vstack_entries; /* value-stack entries per resident thread; 0 = default 4096                   */
-  uint32_t slots;          /* resident eval threads (stack slots); 0 = default (SM count x 512)          */
+  uint32_t slots;          /* resident eval threads (stack slots); 0 = default (SM count x 1024)         */
   uint32_t flags;          /* CULI_F_* below                                                              */
 } culi_opts;
 

@@ -71,7 +71,7 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   }
   if (cudaSetDevice(o.device) != cudaSuccess) { delete c; return CULI_E_CUDA; }
   cudaDeviceGetAttribute(&c->sms, cudaDevAttrMultiProcessorCount, o.device);
-  if (o.slots == 0) o.slots = (uint32_t)c->sms * 512;
+  if (o.slots == 0) o.slots = (uint32_t)c->sms * 128 * CULI_BLOCKS_PER_SM;
   c->nslots = (o.slots + 127) / 128 * 128;
   c->kcap = 2 * o.max_depth + 8;
   c->vcap = o.vstack_entries;

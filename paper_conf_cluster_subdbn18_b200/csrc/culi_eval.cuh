@@ -20,6 +20,13 @@ namespace culi {
 
 constexpr uint32_t STACK_ENV = 0x80000000u;   // env reference into the thread's V-stack
 
+// Resident 128-thread eval blocks per SM (the register budget of __launch_bounds__) and so the default
+// number of stack slots (SM count x 128 x this).  The machine is latency-bound: more warps per scheduler
+// hide more of each warp's dependent-instruction latency.
+#ifndef CULI_BLOCKS_PER_SM
+#define CULI_BLOCKS_PER_SM 8
+#endif
+
 // Serve the persistent code segment from shared memory (see culi_machine.cuh ldnode); off by default.
 #ifndef CULI_STAGE_CODE
 #define CULI_STAGE_CODE 0

@@ -132,7 +132,7 @@ __device__ __noinline__ uint32_t split_claim(const EvalArgs& A) {
 // warp that finds no form left becomes a thief: lane i of it evaluates task i of a claimed split group on
 // the warp's own stacks (one eval_form call site serves forms and tasks).
 template <bool FANOUT, bool NEST, bool SPLIT>
-__global__ void __launch_bounds__(128, 4) culi_eval_kernel(const __grid_constant__ EvalArgs A) {
+__global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(const __grid_constant__ EvalArgs A) {
   uint4* scode = culi_smem;
   uint64_t* sgword = reinterpret_cast<uint64_t*>(culi_smem + A.code_n);
   uint8_t* sgtag = reinterpret_cast<uint8_t*>(sgword + A.gst);
@@ -338,7 +338,7 @@ cudaError_t launch_nest_clear(cudaStream_t s, NestDesc* d, uint32_t n) {
 // verifies (cons, inside the heap as it was when the descriptor was written, linked to cell i+1); a
 // failed check or an element error marks the form for exact sequential re-evaluation.  Results go to
 // the preallocated spine (cells [spine, spine+n), boxes [spine+n, spine+2n)): coalesced stores.
-__global__ void __launch_bounds__(128, 4) culi_fanout_kernel(const __grid_constant__ EvalArgs A) {
+__global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_fanout_kernel(const __grid_constant__ EvalArgs A) {
   uint4* scode = culi_smem;
   uint64_t* sgword = reinterpret_cast<uint64_t*>(culi_smem + A.code_n);
   uint8_t* sgtag = reinterpret_cast<uint8_t*>(sgword + A.gst);
