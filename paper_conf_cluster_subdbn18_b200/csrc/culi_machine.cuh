@@ -66,7 +66,11 @@ __device__ __forceinline__ bool is_ref_k(uint32_t k) { return (REF_MASK >> k) & 
 
 // ---- staged shared memory -----------------------------------------------------------------------------
 __device__ __forceinline__ const uint64_t* sm_gword(const Ctx& C) {
+#if CULI_STAGE_CODE
   return reinterpret_cast<const uint64_t*>(culi_smem + C.A->code_n);
+#else
+  return reinterpret_cast<const uint64_t*>(culi_smem);            // no code segment staged (code_n = 0)
+#endif
 }
 __device__ __forceinline__ const uint8_t* sm_gtag(const Ctx& C) {
   return reinterpret_cast<const uint8_t*>(sm_gword(C) + C.A->gst);
@@ -156,16 +160,16 @@ __device__ __forceinline__ bool proper_value(const Ctx& C, V v) {
 __device__ __forceinline__ V reserved_value(uint32_t sym) {
   return sym < N_SPECIALS ? mkv(K_SPECIAL, sym) : mkv(K_BUILTIN, sym - N_SPECIALS);
 }
+// symbols beyond the staged part of the global frame (and define mode, which stages nothing)
+__device__ CULI_COLD V global_value_hbm(Ctx C, uint32_t sym) {
+  uint32_t gt = C.A->H.gtag[sym];
+  if (gt == K_UNBOUND) return mkv(K_SYM, sym);
+  return mkv(gt, C.A->H.gword[sym]);
+}
 __device__ __forceinline__ V global_value(const Ctx& C, uint32_t sym) {
-  uint32_t gt;
-  uint64_t gw;
-  if (sym < C.A->gst) {
-    gt = sm_gtag(C)[sym];
-    gw = sm_gword(C)[sym];
-  } else {
-    gt = C.A->H.gtag[sym];
-    gw = C.A->H.gword[sym];
-  }
+  if (__builtin_expect(sym >= C.A->gst, 0)) return global_value_hbm(C, sym);
+  uint32_t gt = sm_gtag(C)[sym];
+  uint64_t gw = sm_gword(C)[sym];
   if (gt == K_UNBOUND) return mkv(K_SYM, sym);
   return mkv(gt, gw);
 }
@@ -353,8 +357,9 @@ constexpr uint64_t FAST_OPS =
     (1ull << BI_GE) | (1ull << BI_EQ) | (1ull << BI_NULL) | (1ull << BI_NOT) | (1ull << BI_ATOM) |
     (1ull << BI_CONSP) | (1ull << BI_NUMBERP) | (1ull << BI_SYMBOLP) | (1ull << BI_CAR) | (1ull << BI_CDR);
 
-// (op a0 [a1]) with argc <= 2 evaluated arguments in registers; same checks as the general path
-__device__ __forceinline__ uint8_t fast2(const Ctx& C, uint32_t op, uint32_t argc, V a0, V a1, V* out) {
+// (op a0 [a1]) with argc <= 2 evaluated arguments in registers; same checks as the general path.  Every
+// case; out of line (fast2 below inlines only the common ones, to keep the machine's hot code small).
+__device__ CULI_COLD uint8_t fast2_full(Ctx C, uint32_t op, uint32_t argc, V a0, V a1, V* out) {
   switch (op) {
     case BI_ADD: case BI_SUB: case BI_MUL: case BI_DIV: {
       if (argc == 0) {
@@ -417,6 +422,35 @@ __device__ __forceinline__ uint8_t fast2(const Ctx& C, uint32_t op, uint32_t arg
   }
 }
 
+// Inline front of fast2_full: int64 (+ - *) and comparisons of two INTs, null/not, car/cdr of a cons.
+// Instruction fetch is the machine's top stall: one compact copy per call site.
+__device__ __forceinline__ uint8_t fast2(const Ctx& C, uint32_t op, uint32_t argc, V a0, V a1, V* out) {
+  if (argc == 2 && a0.t == K_INT && a1.t == K_INT) {
+    uint64_t x = a0.w, y = a1.w;
+    if (op <= BI_MUL && op != BI_DIV) {
+      out->t = K_INT;
+      out->w = op == BI_ADD ? x + y : op == BI_SUB ? x - y : x * y;
+      return 0;
+    }
+    if (op >= BI_NUMEQ && op <= BI_GE) {
+      long long sx = (long long)x, sy = (long long)y;
+      bool lt = sx < sy, eq = sx == sy;
+      bool r = op == BI_NUMEQ ? eq : op == BI_LT ? lt : op == BI_GT ? !(lt || eq) : op == BI_LE ? (lt || eq) : !lt;
+      *out = mkb(r);
+      return 0;
+    }
+  }
+  if (argc == 1) {
+    if (op == BI_NULL || op == BI_NOT) { *out = mkb(a0.t == K_NIL); return 0; }
+    if ((op == BI_CAR || op == BI_CDR) && a0.t == K_CONS) {
+      uint64_t w = nword(C, (uint32_t)a0.w);
+      *out = unbox(C, op == BI_CAR ? lo32(w) : hi32(w));
+      return 0;
+    }
+  }
+  return fast2_full(C, op, argc, a0, a1, out);
+}
+
 // equal: recursive on cons cells, with the V-stack above vtop as the explicit work stack
 __device__ CULI_COLD uint8_t equal_values(Ctx C, uint32_t vtop, V a, V b, bool* res) {
   uint32_t sp = vtop;
@@ -454,7 +488,7 @@ __device__ CULI_COLD uint8_t apply_builtin(Ctx C, uint32_t op, uint32_t base, ui
   const DevHeap& H = C.A->H;
   if (((FAST_OPS >> op) & 1) && cnt <= 2) {
     V a0 = cnt > 0 ? arg(C, base, 0) : mkv(K_NIL, 0), a1 = cnt > 1 ? arg(C, base, 1) : mkv(K_NIL, 0);
-    return fast2(C, op, cnt, a0, a1, out);
+    return fast2_full(C, op, cnt, a0, a1, out);
   }
   switch (op) {
     case BI_ADD: case BI_SUB: case BI_MUL: case BI_DIV: {       // cnt >= 3: left fold (c.13 #29)
@@ -586,7 +620,7 @@ __device__ CULI_COLD uint8_t apply_builtin(Ctx C, uint32_t op, uint32_t base, ui
     }
     default: {                                       // fast ops with arity errors (cnt > 2)
       V a0 = arg(C, base, 0), a1 = arg(C, base, 1);
-      return fast2(C, op, cnt > 2 ? 3 : cnt, a0, a1, out);
+      return fast2_full(C, op, cnt > 2 ? 3 : cnt, a0, a1, out);
     }
   }
 }
