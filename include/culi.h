@@ -126,6 +126,32 @@ int culi_fetch_results(culi_ctx* ctx, uint32_t batch_handle, culi_results** out)
 /* Release an uploaded batch (resets the heap to the post-define mark). */
 int culi_release(culi_ctx* ctx, uint32_t batch_handle);
 
+/* ---- device reader -----------------------------------------------------------------
+ * The paper reads on the GPU (§III-B.b) and found parsing to be the dominant GPU
+ * phase (L785-788, L1081-1088); these calls read program text ON THE DEVICE, straight into the heap: a
+ * data-parallel lexer (scan of per-byte transition functions), a bracket-depth scan, token
+ * classification + int64 / correctly rounded binary64 parsing, device symbol interning (same dense ids as
+ * culi_read, so printing and the global environment are shared), a stable (depth, item) radix sort that
+ * groups list elements, and node emission with contiguous spines (c.14).  The image and every result are
+ * identical to culi_read + culi_define / culi_eval_batch on the same text (syntax: SURVEY §8(c).1).
+ *   text, len      : `len` bytes of program text (len < 2^32 - 1).  text_on_device != 0: a device pointer
+ *                    (any alignment; 16-byte aligned reads when aligned), else host memory (copied to the
+ *                    device first; page-locked memory copies fastest).  Borrowed for the call only.
+ *   err_offset     : on CULI_E_PARSE, the same byte offset culi_read reports (first offending character,
+ *                    else the innermost construct still open at the end of the text).
+ * culi_define_text: culi_define on the read forms (same failure reporting).
+ * culi_eval_text  : culi_eval_batch on the read forms (synchronous, results on the host).
+ * culi_upload_text: read + prepare a batch for culi_eval_uploaded / culi_fetch_results (*nforms = forms).
+ * culi_last_read  : device time in ms of the last device read (lex .. emit, text already in HBM), its
+ *                   item count (structural characters + datum starts) and the nodes it emitted. */
+int culi_define_text(culi_ctx* ctx, const char* text, size_t len, int text_on_device, uint32_t* failed_index,
+                     uint8_t* failed_err, size_t* err_offset);
+int culi_eval_text(culi_ctx* ctx, const char* text, size_t len, int text_on_device, culi_results** out,
+                   size_t* err_offset);
+int culi_upload_text(culi_ctx* ctx, const char* text, size_t len, int text_on_device, uint32_t* batch_handle,
+                     uint32_t* nforms, size_t* err_offset);
+int culi_last_read(const culi_ctx* ctx, float* ms, uint64_t* items, uint64_t* nodes);
+
 /* ---- results (host) --------------------------------------------------------------------------------- */
 uint32_t culi_results_count(const culi_results* r);
 /* tag: culi_tag (CULI_ERROR when err != 0); err: culi_err; steps: canonical eval steps (c.4). */

@@ -9,7 +9,7 @@ HERE = os.path.dirname(os.path.abspath(__file__))
 ROOT = os.path.dirname(HERE)
 CSRC = os.path.join(HERE, "csrc")
 LIB = os.path.join(HERE, "libculi.so")
-SOURCES = ["culi_host.cpp", "culi_kernels.cu", "culi_dispatch.cu", "culi_capi.cu", "culi_dist.cu"]
+SOURCES = ["culi_host.cpp", "culi_kernels.cu", "culi_dispatch.cu", "culi_capi.cu", "culi_dist.cu", "culi_reader.cu"]
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
 FLAGS = ["-O3", "-std=c++17", "-lineinfo", "--fmad=false", "-Xcompiler", "-fPIC,-O2,-ffp-contract=off",
@@ -24,6 +24,10 @@ def _stale(target: str, deps: list[str]) -> bool:
 
 
 def build(verbose: bool = False, force: bool = False, ptxas_v: bool = False) -> str:
+    if HERE not in sys.path:
+        sys.path.insert(0, HERE)
+    import gen_pow5
+    gen_pow5.write(os.path.join(CSRC, "culi_pow5.inc"))
     deps = [os.path.join(CSRC, f) for f in os.listdir(CSRC)] + [os.path.join(ROOT, "include", "culi.h")]
     if not force and not _stale(LIB, deps):
         return LIB

@@ -147,6 +147,7 @@ void culi_shutdown(culi_ctx* c) {
   c->roots.release(); c->keys.release(); c->keys_alt.release(); c->perm.release();
   c->perm_alt.release(); c->rtag.release(); c->rerr.release(); c->dtemp.release();
   c->rsteps.release(); c->rword.release(); c->payload.release();
+  c->rd.release();
   for (auto& e : c->ev) if (e) cudaEventDestroy(e);
   delete c;
 }
@@ -284,19 +285,11 @@ static int ensure_results(culi_ctx* c, uint32_t nforms) {
   return CULI_OK;
 }
 
-extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed_index,
-                           uint8_t* failed_err) {
-  if (!c || !defs) return CULI_E_ARG;
-  const Image& img = defs->img;
-  uint32_t nf = (uint32_t)img.roots.size();
-  uint32_t str_base = (uint32_t)c->strings.size();
-  int rc = upload_image(c, img, str_base);
+// Evaluate the nf definition forms already in the heap at c->mark (nnodes image nodes), in order.
+static int run_define(culi_ctx* c, uint32_t nf, uint64_t nnodes, uint32_t* failed_index, uint8_t* failed_err) {
+  int rc = ensure_results(c, nf);
   if (rc) return rc;
-  c->strings += img.strings;
-  c->persist_has_par = c->persist_has_par || image_mentions_par(img);
-  rc = ensure_results(c, nf);
-  if (rc) return rc;
-  CK(launch_reset(c->stream, c->H.top, c->mark + img.tag.size(), c->next, c->pcount, c->flags, c->npend,
+  CK(launch_reset(c->stream, c->H.top, c->mark + nnodes, c->next, c->pcount, c->flags, c->npend,
                   c->nfallback, c->nnest, c->gcount));
   EvalArgs A = make_args(c, nf, nullptr, 1);
   if (nf) CK(launch_define(c->stream, A));
@@ -316,6 +309,30 @@ extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed
     return CULI_E_DEFINE;
   }
   return CULI_OK;
+}
+
+extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed_index,
+                           uint8_t* failed_err) {
+  if (!c || !defs) return CULI_E_ARG;
+  const Image& img = defs->img;
+  uint32_t nf = (uint32_t)img.roots.size();
+  uint32_t str_base = (uint32_t)c->strings.size();
+  int rc = upload_image(c, img, str_base);
+  if (rc) return rc;
+  c->strings += img.strings;
+  c->persist_has_par = c->persist_has_par || image_mentions_par(img);
+  return run_define(c, nf, img.tag.size(), failed_index, failed_err);
+}
+
+extern "C" int culi_define_text(culi_ctx* c, const char* text, size_t len, int text_on_device,
+                                uint32_t* failed_index, uint8_t* failed_err, size_t* err_offset) {
+  if (!c || (!text && len)) return CULI_E_ARG;
+  ReadOut ro;
+  int rc = device_read(c, text, len, text_on_device != 0, &ro, err_offset);
+  if (rc) return rc;
+  c->strings += ro.strings;
+  c->persist_has_par = c->persist_has_par || ro.par_root_head || ro.par_nested;
+  return run_define(c, ro.nforms, ro.nodes, failed_index, failed_err);
 }
 
 // Run dispatch + eval + export for the uploaded batch (device only, stream-ordered, no host sync).
@@ -371,12 +388,12 @@ static int run_batch_device(culi_ctx* c) {
   return CULI_OK;
 }
 
-static int prepare_batch(culi_ctx* c, const Image& img) {
-  uint32_t nf = (uint32_t)img.roots.size();
-  uint32_t str_base = (uint32_t)c->strings.size();
-  int rc = upload_image(c, img, str_base);
-  if (rc) return rc;
-  rc = ensure_results(c, nf);
+// Buffers and launch decisions for a batch whose image is already in the heap at c->mark (uploaded from a
+// host image or written by the device reader).  par_any / par_nonroot: the ||| symbol is the car of some
+// cell / of some cell other than a top-level form's first cell; par_head: some form is (||| ...).
+static int finish_prepare(culi_ctx* c, uint32_t nf, uint64_t nnodes, std::string strings, bool par_any,
+                          bool par_nonroot, bool par_head, bool has_wide) {
+  int rc = ensure_results(c, nf);
   if (rc) return rc;
   size_t n = std::max<uint32_t>(nf, 1);
   CK(c->keys.ensure(n));
@@ -385,22 +402,31 @@ static int prepare_batch(culi_ctx* c, const Image& img) {
   CK(c->perm_alt.ensure(n));
   CK(c->dtemp.ensure(dispatch_temp_bytes(nf)));
   // tokens: ~4 per form; a ||| result list can be as long as the persistent segment (2 tokens per cell)
-  CK(c->payload.ensure(std::max<size_t>(4 * (size_t)nf + 2 * (size_t)(c->mark + img.tag.size()), 1 << 16)));
+  CK(c->payload.ensure(std::max<size_t>(4 * (size_t)nf + 2 * (size_t)(c->mark + nnodes), 1 << 16)));
   c->have_batch = true;
-  c->batch_nodes = img.tag.size();
+  c->batch_nodes = nnodes;
   c->batch_forms = nf;
-  c->batch_strings = img.strings;
+  c->batch_strings = std::move(strings);
   CK(c->fallback.ensure((size_t)c->maxdesc + nf + 1));
   // may ||| occur below the top level (nested fan-out, §8(f)1)?  any ||| symbol in the batch or in a definition
-  c->batch_may_nest = c->persist_has_par ||
-                      image_mentions_par(img, !(c->opts.flags & CULI_F_NO_FANOUT));
+  c->batch_may_nest = c->persist_has_par || ((c->opts.flags & CULI_F_NO_FANOUT) ? par_any : par_nonroot);
   if (c->batch_may_nest && !c->kst2 && !(c->opts.flags & CULI_F_NO_NESTED)) {
     CK(cudaMalloc(&c->kst2, (size_t)c->nslots * c->kcap * sizeof(uint4)));
     CK(cudaMalloc(&c->vst2, (size_t)c->nslots * c->vcap * sizeof(uint4)));
   }
+  c->batch_has_par = par_head;
+  c->batch_has_wide = has_wide;
+  if (has_wide) c->batch_has_par = true;             // the fan-out kernels handle both
+  return CULI_OK;
+}
+
+static int prepare_batch(culi_ctx* c, const Image& img) {
+  uint32_t nf = (uint32_t)img.roots.size();
+  uint32_t str_base = (uint32_t)c->strings.size();
+  int rc = upload_image(c, img, str_base);
+  if (rc) return rc;
   // does any form start with the ||| symbol (a6), or have >= WIDE_MIN arguments (wide forms, K12)?
-  c->batch_has_par = false;
-  c->batch_has_wide = false;
+  bool par_head = false, has_wide = false;
   std::vector<uint32_t> wide;
   for (uint32_t f = 0; f < nf; ++f) {
     uint32_t r = img.roots[f];
@@ -409,21 +435,30 @@ static int prepare_batch(culi_ctx* c, const Image& img) {
     uint32_t h = (uint32_t)rw;
     if (h >= IMG_FIRST && (img.tag[h - IMG_FIRST] & KIND_MASK) == K_SYM &&
         img.word[h - IMG_FIRST] == N_SPECIALS + BI_PAR)
-      c->batch_has_par = true;
+      par_head = true;
     uint32_t nargs = 0;
     for (uint32_t q = (uint32_t)(rw >> 32); q >= IMG_FIRST; q = (uint32_t)(img.word[q - IMG_FIRST] >> 32)) ++nargs;
     if (nargs >= WIDE_MIN) {
       if (wide.empty()) wide.assign(nf, 0);
       wide[f] = nargs;
-      c->batch_has_wide = true;
+      has_wide = true;
     }
   }
-  if (c->batch_has_wide) {
+  if (has_wide) {
     CK(c->wide.ensure(nf));
     CK(cudaMemcpyAsync(c->wide.p, wide.data(), nf * 4, cudaMemcpyHostToDevice, c->stream));
-    c->batch_has_par = true;                         // the fan-out kernels handle both
   }
-  return CULI_OK;
+  return finish_prepare(c, nf, img.tag.size(), img.strings, image_mentions_par(img, false),
+                        image_mentions_par(img, true), par_head, has_wide);
+}
+
+// Device reader (§8(f)2) -> the same prepared batch.
+static int prepare_text(culi_ctx* c, const char* text, size_t len, bool on_device, size_t* err_offset) {
+  ReadOut ro;
+  int rc = device_read(c, text, len, on_device, &ro, err_offset);
+  if (rc) return rc;
+  return finish_prepare(c, ro.nforms, ro.nodes, std::move(ro.strings), ro.par_root_head || ro.par_nested,
+                        ro.par_nested, ro.par_root_head, ro.wide);
 }
 
 // ||| forms the fan-out could not decide (an element error, fuel overflow, a short or non-contiguous
@@ -527,6 +562,37 @@ int culi_eval_batch(culi_ctx* c, const culi_image* forms, culi_results** out) {
   rc = fetch(c, out);
   c->have_batch = false;
   return rc;
+}
+
+int culi_eval_text(culi_ctx* c, const char* text, size_t len, int text_on_device, culi_results** out,
+                   size_t* err_offset) {
+  if (!c || !out || (!text && len)) return CULI_E_ARG;
+  *out = nullptr;
+  int rc = prepare_text(c, text, len, text_on_device != 0, err_offset);
+  if (rc) return rc;
+  rc = run_batch_device(c);
+  if (rc) return rc;
+  rc = fetch(c, out);
+  c->have_batch = false;
+  return rc;
+}
+
+int culi_upload_text(culi_ctx* c, const char* text, size_t len, int text_on_device, uint32_t* handle,
+                     uint32_t* nforms, size_t* err_offset) {
+  if (!c || (!text && len)) return CULI_E_ARG;
+  int rc = prepare_text(c, text, len, text_on_device != 0, err_offset);
+  if (rc) return rc;
+  if (handle) *handle = 1;
+  if (nforms) *nforms = c->batch_forms;
+  return CULI_OK;
+}
+
+int culi_last_read(const culi_ctx* c, float* ms, uint64_t* items, uint64_t* nodes) {
+  if (!c) return CULI_E_ARG;
+  if (ms) *ms = c->rd.last_ms;
+  if (items) *items = c->rd.last_items;
+  if (nodes) *nodes = c->rd.last_nodes;
+  return CULI_OK;
 }
 
 int culi_upload(culi_ctx* c, const culi_image* forms, uint32_t* handle) {

@@ -10,6 +10,7 @@
 #include "../../include/culi.h"
 #include "culi_eval.cuh"
 #include "culi_host.h"
+#include "culi_reader.h"
 
 inline uint32_t lo32h(uint64_t w) { return (uint32_t)w; }
 
@@ -55,6 +56,31 @@ struct DevBuf {
 
 constexpr uint32_t GCAP = 1u << 22;           // symbol ids supported (global table entries)
 constexpr uint64_t STR_CAP = 64ull << 20;      // string bytes
+
+// device reader working set (culi_reader.cu), allocated on first use
+struct ReaderState {
+  DevSyms S;
+  uint32_t synced = 0;               // host names already in the device table
+  uint64_t pool_top = 0;             // device name pool bytes mirrored on the host
+  ReadInfo* info = nullptr;
+  DevBuf<uint8_t> text, tiles, temp, ikind, ivt;
+  DevBuf<uint32_t> tstate, toff, small, ipos, b32, roff, keys, keys2, vals, vals2, iparent, ij, ik, slen, soff;
+  DevBuf<int> a32, depth, hmax;
+  DevBuf<uint64_t> ival;
+  float last_ms = 0;
+  uint64_t last_items = 0, last_nodes = 0, last_bytes = 0;
+  void release() {
+    cudaFree(S.key); cudaFree(S.id); cudaFree(S.noff); cudaFree(S.pool); cudaFree(S.count); cudaFree(info);
+    S = DevSyms{};
+    info = nullptr;
+    for (auto* b : {&text, &tiles, &temp, &ikind, &ivt}) b->release();
+    for (auto* b : {&tstate, &toff, &small, &ipos, &b32, &roff, &keys, &keys2, &vals, &vals2, &iparent, &ij, &ik,
+                    &slen, &soff})
+      b->release();
+    for (auto* b : {&a32, &depth, &hmax}) b->release();
+    ival.release();
+  }
+};
 
 }  // namespace culi_detail
 using namespace culi_detail;
@@ -111,6 +137,7 @@ struct culi_ctx {
   uint32_t batch_forms = 0;
   uint32_t* batch_perm = nullptr;
   std::string batch_strings;
+  ReaderState rd;
   // timing
   cudaEvent_t ev[4] = {nullptr, nullptr, nullptr, nullptr};
   uint32_t last_kernels = 0;

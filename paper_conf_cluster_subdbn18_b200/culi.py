@@ -32,6 +32,7 @@ SYMBOLS = [
     "culi_env_export", "culi_env_import", "culi_results_serialize", "culi_results_merge",
     "culi_status_string", "culi_error_name", "culi_last_timing", "culi_records_device",
     "culi_last_stats", "culi_last_splits", "culi_image_pin", "culi_results_wire_bytes",
+    "culi_define_text", "culi_eval_text", "culi_upload_text", "culi_last_read",
 ]
 
 
@@ -93,6 +94,10 @@ def load(path: str = LIB_PATH) -> ctypes.CDLL:
         "culi_last_splits": (I, [P, pp(U32)]),
         "culi_image_pin": (I, [P, pp(U64)]),
         "culi_results_wire_bytes": (I, [P, pp(U64)]),
+        "culi_define_text": (I, [P, P, SZ, I, pp(U32), pp(ctypes.c_uint8), pp(SZ)]),
+        "culi_eval_text": (I, [P, P, SZ, I, pp(P), pp(SZ)]),
+        "culi_upload_text": (I, [P, P, SZ, I, pp(U32), pp(U32), pp(SZ)]),
+        "culi_last_read": (I, [P, pp(ctypes.c_float), pp(U64), pp(U64)]),
     }
     for name, (res, args) in sig.items():
         fn = getattr(L, name)
@@ -171,6 +176,16 @@ class Results:
 
     def printed(self) -> list[str]:
         return [self.print(i) for i in range(len(self))]
+
+    def float_value(self, i: int) -> float:
+        v = ctypes.c_double()
+        _check(load().culi_result_float(self._p, i, ctypes.byref(v)), "culi_result_float")
+        return v.value
+
+    def int_value(self, i: int) -> int:
+        v = ctypes.c_int64()
+        _check(load().culi_result_int(self._p, i, ctypes.byref(v)), "culi_result_int")
+        return v.value
 
     def steps(self) -> list[int]:
         return [self.info(i)[2] for i in range(len(self))]
@@ -270,6 +285,56 @@ class Context:
             err.failed_err = fe.value
             raise err
         _check(rc, "culi_define")
+
+    # --- device reader: text -> heap on the GPU ----------------------------------------
+    @staticmethod
+    def _text(text):
+        """(pointer, length, on_device, keepalive) for str / bytes (host) or a uint8 tensor (host or cuda)."""
+        if isinstance(text, str):
+            text = text.encode()
+        if isinstance(text, (bytes, bytearray)):
+            buf = ctypes.create_string_buffer(bytes(text), len(text))
+            return ctypes.cast(buf, ctypes.c_void_p), len(text), 0, buf
+        return ctypes.c_void_p(text.data_ptr()), text.numel() * text.element_size(), int(text.is_cuda), text
+
+    def define_text(self, text) -> None:
+        ptr, n, dev, keep = self._text(text)
+        fi, fe, off = ctypes.c_uint32(0), ctypes.c_uint8(0), ctypes.c_size_t(0)
+        rc = load().culi_define_text(self._p, ptr, n, dev, ctypes.byref(fi), ctypes.byref(fe), ctypes.byref(off))
+        if rc == -2:
+            raise ParseError(rc, off.value)
+        if rc == -6:
+            err = CuliError(rc, "culi_define_text (form %d: %s)" % (fi.value, ERR_NAMES[fe.value]))
+            err.failed_index = fi.value
+            err.failed_err = fe.value
+            raise err
+        _check(rc, "culi_define_text")
+
+    def eval_text(self, text) -> Results:
+        ptr, n, dev, keep = self._text(text)
+        out, off = ctypes.c_void_p(), ctypes.c_size_t(0)
+        rc = load().culi_eval_text(self._p, ptr, n, dev, ctypes.byref(out), ctypes.byref(off))
+        if rc == -2:
+            raise ParseError(rc, off.value)
+        _check(rc, "culi_eval_text")
+        return Results(out.value)
+
+    def upload_text(self, text) -> tuple[int, int]:
+        """Read on the device and prepare the batch; returns (handle, number of forms)."""
+        ptr, n, dev, keep = self._text(text)
+        h, nf, off = ctypes.c_uint32(0), ctypes.c_uint32(0), ctypes.c_size_t(0)
+        rc = load().culi_upload_text(self._p, ptr, n, dev, ctypes.byref(h), ctypes.byref(nf), ctypes.byref(off))
+        if rc == -2:
+            raise ParseError(rc, off.value)
+        _check(rc, "culi_upload_text")
+        return h.value, nf.value
+
+    def last_read(self) -> tuple[float, int, int]:
+        """(device ms, items, nodes) of the last device read."""
+        ms, it, nd = ctypes.c_float(), ctypes.c_uint64(), ctypes.c_uint64()
+        _check(load().culi_last_read(self._p, ctypes.byref(ms), ctypes.byref(it), ctypes.byref(nd)),
+               "culi_last_read")
+        return ms.value, it.value, nd.value
 
     def eval_batch(self, forms: str | bytes | Image) -> Results:
         img = forms if isinstance(forms, Image) else self.read(forms)
