@@ -10,7 +10,11 @@ from paper_conf_cluster_subdbn18_b200 import workloads as W  # noqa: E402
 
 def main():
   culi.load()
-  for name, wl in [("C1", W.c1()), ("C3", W.c3()), ("C4", W.c4()), ("C5-1M", W.c5(1 << 20))]:
+  import os
+  sel = os.environ.get("PROBE", "C1,C3,C4,C5-1M").split(",")
+  mk = {"C1": lambda: W.c1(), "C3": lambda: W.c3(), "C4": lambda: W.c4(), "C5-1M": lambda: W.c5(1 << 20),
+        "C5-4M": lambda: W.c5(1 << 22)}
+  for name, wl in [(k, mk[k]()) for k in sel]:
       ctx = culi.Context(heap_nodes=1 << 28)
       text = wl.defs if name == "C3" else wl.forms
       if name != "C3" and wl.defs:
