@@ -79,6 +79,7 @@ typedef struct {
 #define CULI_F_NO_VOTING  8u   /* reserved (no effect in this version)                                   */
 #define CULI_F_NO_NESTED 16u   /* run nested (non-top-level) ||| forms inside one thread (§8(f)1 off)     */
 #define CULI_F_NO_SPLIT  32u   /* no argument splitting: each form is evaluated by one thread only        */
+#define CULI_F_NO_GC     64u   /* do not compact the persistent heap segment after culi_define (§8(f)3)  */
 
 /* Fill *opts with defaults (device 0, default stream, default sizes). */
 void culi_default_opts(culi_opts* opts);
@@ -151,6 +152,21 @@ int culi_eval_text(culi_ctx* ctx, const char* text, size_t len, int text_on_devi
 int culi_upload_text(culi_ctx* ctx, const char* text, size_t len, int text_on_device, uint32_t* batch_handle,
                      uint32_t* nforms, size_t* err_offset);
 int culi_last_read(const culi_ctx* ctx, float* ms, uint64_t* items, uint64_t* nodes);
+
+/* ---- heap reclamation ----------------------------------------------------------------
+ * The paper hands out "the sequentially next free node" of a fixed node array and marks nodes that are no
+ * longer needed as free (§III-A.c).  Batch allocations are released wholesale after every
+ * batch; the persistent segment (definitions and what their evaluation allocated) is compacted on the
+ * device after every culi_define / culi_define_text unless CULI_F_NO_GC: nodes reachable from the global
+ * environment are kept (mark from the global table, contiguous cons runs traced as one object) and slid
+ * down in address order, so contiguous list spines stay contiguous (c.14) and results are unchanged.
+ * culi_collect   : run the compaction now (not while a batch is uploaded: CULI_E_STATE).  *live_nodes =
+ *                  nodes kept, *freed_nodes = nodes reclaimed.  Without scratch room above the segment
+ *                  (2 x live > capacity) the segment is left as it is (freed = 0).
+ * culi_heap_usage: *persistent_nodes = heap nodes in use between batches (the post-define mark, including
+ *                  nodes 0/1), *capacity = heap nodes, *freed_total = nodes reclaimed so far. */
+int culi_collect(culi_ctx* ctx, uint64_t* live_nodes, uint64_t* freed_nodes);
+int culi_heap_usage(const culi_ctx* ctx, uint64_t* persistent_nodes, uint64_t* capacity, uint64_t* freed_total);
 
 /* ---- results (host) --------------------------------------------------------------------------------- */
 uint32_t culi_results_count(const culi_results* r);

@@ -9,7 +9,7 @@ HERE = os.path.dirname(os.path.abspath(__file__))
 ROOT = os.path.dirname(HERE)
 CSRC = os.path.join(HERE, "csrc")
 LIB = os.path.join(HERE, "libculi.so")
-SOURCES = ["culi_host.cpp", "culi_kernels.cu", "culi_dispatch.cu", "culi_capi.cu", "culi_dist.cu", "culi_reader.cu"]
+SOURCES = ["culi_host.cpp", "culi_kernels.cu", "culi_dispatch.cu", "culi_capi.cu", "culi_dist.cu", "culi_reader.cu", "culi_gc.cu"]
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
 FLAGS = ["-O3", "-std=c++17", "-lineinfo", "--fmad=false", "-Xcompiler", "-fPIC,-O2,-ffp-contract=off",

@@ -148,6 +148,7 @@ void culi_shutdown(culi_ctx* c) {
   c->perm_alt.release(); c->rtag.release(); c->rerr.release(); c->dtemp.release();
   c->rsteps.release(); c->rword.release(); c->payload.release();
   c->rd.release();
+  c->gc.release();
   for (auto& e : c->ev) if (e) cudaEventDestroy(e);
   delete c;
 }
@@ -285,6 +286,17 @@ static int ensure_results(culi_ctx* c, uint32_t nforms) {
   return CULI_OK;
 }
 
+static int run_collect(culi_ctx* c) {
+  uint64_t live = 0, freed = 0;
+  int rc = collect_persistent(c, &live, &freed);
+  if (rc) return rc;
+  c->gc.last_live = live;
+  c->gc.last_freed = freed;
+  c->gc.total_freed += freed;
+  ++c->gc.collections;
+  return CULI_OK;
+}
+
 // Evaluate the nf definition forms already in the heap at c->mark (nnodes image nodes), in order.
 static int run_define(culi_ctx* c, uint32_t nf, uint64_t nnodes, uint32_t* failed_index, uint8_t* failed_err) {
   int rc = ensure_results(c, nf);
@@ -301,6 +313,11 @@ static int run_define(culi_ctx* c, uint32_t nf, uint64_t nnodes, uint32_t* faile
   c->mark = std::min<unsigned long long>(top, c->H.cap);
   c->heap_high = std::max<uint64_t>(c->heap_high, top);
   c->defined = true;
+  // reclaim the persistent segment: keep what the global frame reaches (§8(f)3, culi_gc.cu)
+  if (!(c->opts.flags & CULI_F_NO_GC)) {
+    int g = run_collect(c);
+    if (g) return g;
+  }
   if (flags[0] && !flags[1]) return CULI_E_HEAP_FULL;
   if (flags[1]) {
     if (failed_index) *failed_index = (uint32_t)(flags[1] - 1);
@@ -584,6 +601,24 @@ int culi_upload_text(culi_ctx* c, const char* text, size_t len, int text_on_devi
   if (rc) return rc;
   if (handle) *handle = 1;
   if (nforms) *nforms = c->batch_forms;
+  return CULI_OK;
+}
+
+int culi_collect(culi_ctx* c, uint64_t* live_nodes, uint64_t* freed_nodes) {
+  if (!c) return CULI_E_ARG;
+  if (c->have_batch) return CULI_E_STATE;
+  int rc = run_collect(c);
+  if (rc) return rc;
+  if (live_nodes) *live_nodes = c->gc.last_live;
+  if (freed_nodes) *freed_nodes = c->gc.last_freed;
+  return CULI_OK;
+}
+
+int culi_heap_usage(const culi_ctx* c, uint64_t* persistent_nodes, uint64_t* capacity, uint64_t* freed_total) {
+  if (!c) return CULI_E_ARG;
+  if (persistent_nodes) *persistent_nodes = c->mark;
+  if (capacity) *capacity = c->H.cap;
+  if (freed_total) *freed_total = c->gc.total_freed;
   return CULI_OK;
 }
 

@@ -82,8 +82,24 @@ struct ReaderState {
   }
 };
 
+// heap reclamation working set (culi_gc.cu)
+struct GcState {
+  DevBuf<uint32_t> role, pos, q0, q1, cnt;
+  DevBuf<uint8_t> temp;
+  uint32_t last_rounds = 0;
+  uint64_t last_live = 0, last_freed = 0, total_freed = 0, collections = 0;
+  void release() {
+    for (auto* b : {&role, &pos, &q0, &q1, &cnt}) b->release();
+    temp.release();
+  }
+};
+
 }  // namespace culi_detail
 using namespace culi_detail;
+
+namespace culi {
+int collect_persistent(culi_ctx* c, uint64_t* live, uint64_t* freed);
+}
 
 struct culi_ctx {
   culi_opts opts;
@@ -138,6 +154,7 @@ struct culi_ctx {
   uint32_t* batch_perm = nullptr;
   std::string batch_strings;
   ReaderState rd;
+  GcState gc;
   // timing
   cudaEvent_t ev[4] = {nullptr, nullptr, nullptr, nullptr};
   uint32_t last_kernels = 0;

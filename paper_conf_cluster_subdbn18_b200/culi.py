@@ -23,6 +23,7 @@ CULI_F_NO_STAGING = 4
 CULI_F_NO_VOTING = 8
 CULI_F_NO_NESTED = 16
 CULI_F_NO_SPLIT = 32
+CULI_F_NO_GC = 64
 
 SYMBOLS = [
     "culi_default_opts", "culi_init", "culi_shutdown", "culi_read", "culi_image_nforms",
@@ -32,7 +33,8 @@ SYMBOLS = [
     "culi_env_export", "culi_env_import", "culi_results_serialize", "culi_results_merge",
     "culi_status_string", "culi_error_name", "culi_last_timing", "culi_records_device",
     "culi_last_stats", "culi_last_splits", "culi_image_pin", "culi_results_wire_bytes",
-    "culi_define_text", "culi_eval_text", "culi_upload_text", "culi_last_read",
+    "culi_define_text", "culi_eval_text", "culi_upload_text", "culi_last_read", "culi_collect",
+    "culi_heap_usage",
 ]
 
 
@@ -98,6 +100,8 @@ def load(path: str = LIB_PATH) -> ctypes.CDLL:
         "culi_eval_text": (I, [P, P, SZ, I, pp(P), pp(SZ)]),
         "culi_upload_text": (I, [P, P, SZ, I, pp(U32), pp(U32), pp(SZ)]),
         "culi_last_read": (I, [P, pp(ctypes.c_float), pp(U64), pp(U64)]),
+        "culi_collect": (I, [P, pp(U64), pp(U64)]),
+        "culi_heap_usage": (I, [P, pp(U64), pp(U64), pp(U64)]),
     }
     for name, (res, args) in sig.items():
         fn = getattr(L, name)
@@ -328,6 +332,18 @@ class Context:
             raise ParseError(rc, off.value)
         _check(rc, "culi_upload_text")
         return h.value, nf.value
+
+    def collect(self) -> tuple[int, int]:
+        """culi_collect: compact the persistent heap segment now; (live nodes, freed nodes)."""
+        a, b = ctypes.c_uint64(), ctypes.c_uint64()
+        _check(load().culi_collect(self._p, ctypes.byref(a), ctypes.byref(b)), "culi_collect")
+        return a.value, b.value
+
+    def heap_usage(self) -> tuple[int, int, int]:
+        """(persistent nodes in use, heap capacity, nodes reclaimed so far)."""
+        a, b, c = ctypes.c_uint64(), ctypes.c_uint64(), ctypes.c_uint64()
+        _check(load().culi_heap_usage(self._p, ctypes.byref(a), ctypes.byref(b), ctypes.byref(c)), "culi_heap_usage")
+        return a.value, b.value, c.value
 
     def last_read(self) -> tuple[float, int, int]:
         """(device ms, items, nodes) of the last device read."""
