@@ -70,7 +70,7 @@ struct ReaderState {
   float last_ms = 0;
   uint64_t last_items = 0, last_nodes = 0, last_bytes = 0;
   void release() {
-    cudaFree(S.key); cudaFree(S.id); cudaFree(S.noff); cudaFree(S.pool); cudaFree(S.count); cudaFree(info);
+    cudaFree(S.key); cudaFree(S.id); cudaFree(S.tag); cudaFree(S.noff); cudaFree(S.pool); cudaFree(S.count); cudaFree(info);
     S = DevSyms{};
     info = nullptr;
     for (auto* b : {&text, &tiles, &temp, &ikind, &ivt}) b->release();

@@ -14,6 +14,7 @@ constexpr uint32_t ROOT = 0xffffffffu;           // parent of a top-level datum
 struct DevSyms {
   uint64_t* key = nullptr;       // slot -> name hash (0 = empty)
   uint32_t* id = nullptr;        // slot -> symbol id (0xffffffff = being published)
+  uint64_t* tag = nullptr;       // slot -> first 7 name bytes | min(length, 255) << 56
   uint64_t* noff = nullptr;      // id -> pool offset | length << 32
   uint8_t* pool = nullptr;       // name bytes
   uint32_t* count = nullptr;     // [0] next id, [2..3] pool top (u64), [4] overflow
