@@ -64,7 +64,7 @@ struct ReaderState {
   uint64_t pool_top = 0;             // device name pool bytes mirrored on the host
   ReadInfo* info = nullptr;
   DevBuf<uint8_t> text, tiles, temp, ikind, ivt;
-  DevBuf<uint32_t> tstate, toff, small, ipos, b32, roff, keys, keys2, vals, vals2, iparent, ij, ik, slen, soff;
+  DevBuf<uint32_t> tstate, toff, small, ipos, b32, roff, keys, keys2, vals, vals2, iparent, ij, ik, slen, soff, vlist;
   DevBuf<int> a32, depth, hmax;
   DevBuf<uint64_t> ival;
   float last_ms = 0;
@@ -75,7 +75,7 @@ struct ReaderState {
     info = nullptr;
     for (auto* b : {&text, &tiles, &temp, &ikind, &ivt}) b->release();
     for (auto* b : {&tstate, &toff, &small, &ipos, &b32, &roff, &keys, &keys2, &vals, &vals2, &iparent, &ij, &ik,
-                    &slen, &soff})
+                    &slen, &soff, &vlist})
       b->release();
     for (auto* b : {&a32, &depth, &hmax}) b->release();
     ival.release();

@@ -35,7 +35,7 @@ struct ReadInfo {
   uint32_t last_pos;
   uint32_t nforms;
   uint32_t flags;                // RF_*
-  uint32_t pad;
+  uint32_t nvalid;               // lists queued for special-form syntax validation
 };
 constexpr uint32_t RF_PAR_ROOT_HEAD = 1;         // some top-level form is (||| ...)
 constexpr uint32_t RF_PAR_NESTED = 2;            // ||| is the car of some other cell

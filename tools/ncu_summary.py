@@ -73,10 +73,54 @@ def num(s):
     return float(str(s).replace(",", ""))
 
 
+UNIT = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9, "ns": 1e-9, "nsecond": 1e-9, "us": 1e-6,
+        "usecond": 1e-6, "ms": 1e-3, "msecond": 1e-3, "s": 1.0, "second": 1.0}
+
+
+def sweep(paths, peak_gbs=6547.5):
+    """Per workload and kernel (first launch of each kernel in the capture): the SURVEY §8(d) metrics."""
+    out = ["| config | kernel | time ms | DRAM GB | DRAM GB/s | %% of %.0f GB/s | warp eff. | L2 hit | issue active "
+           "| warps active | local B |" % peak_gbs, "|---|---|---|---|---|---|---|---|---|---|---|"]
+    for path in paths:
+        wl = path.rsplit("_", 1)[-1].split(".")[0]
+        rows = list(csv.reader(open(path, errors="replace")))
+        try:
+            hi = next(i for i, r in enumerate(rows) if "Metric Name" in r)
+        except StopIteration:
+            out.append("| %s | (no data) |" % wl)
+            continue
+        h = rows[hi]
+        ii, ki, mi, ui, vi = (h.index(x) for x in ("ID", "Kernel Name", "Metric Name", "Metric Unit", "Metric Value"))
+        per = {}
+        for r in rows[hi + 1:]:
+            if len(r) <= vi:
+                continue
+            per.setdefault((r[ki].split("(")[0], r[ii]), {})[r[mi]] = num(r[vi]) * UNIT.get(r[ui], 1.0)
+        seen = set()
+        for (k, lid), m in sorted(per.items(), key=lambda kv: int(kv[0][1])):
+            if k in seen:
+                continue
+            seen.add(k)
+            t = m.get("gpu__time_duration.sum", 0)
+            b = m.get("dram__bytes_read.sum", 0) + m.get("dram__bytes_write.sum", 0)
+            gbs = b / t / 1e9 if t else 0
+            loc = m.get("l1tex__t_bytes_pipe_lsu_mem_local_op_ld.sum", 0) + \
+                m.get("l1tex__t_bytes_pipe_lsu_mem_local_op_st.sum", 0)
+            out.append("| %s | %s | %.3f | %.3f | %.1f | %.2f%% | %.1f%% | %.1f%% | %.1f%% | %.1f%% | %.3g |" % (
+                wl, k.replace("void ", "")[:44], t * 1e3, b / 1e9, gbs, 100 * gbs / peak_gbs,
+                100 * m.get("smsp__thread_inst_executed_per_inst_executed.ratio", 0) / 32,
+                m.get("lts__t_sector_hit_rate.pct", 0), m.get("smsp__issue_active.avg.pct_of_peak_sustained_active", 0),
+                m.get("sm__warps_active.avg.pct_of_peak_sustained_active", 0), loc))
+    return "\n".join(out)
+
+
 def main():
     mode, path = sys.argv[1], sys.argv[2]
     if mode == "launches":
         print(launches(path))
+        return
+    if mode == "sweep":
+        print(sweep(sys.argv[2:]))
         return
     res = full(path)
     for d in res:
