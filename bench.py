@@ -215,8 +215,10 @@ def culi_arm(args):
     cdev = torch.device("cuda", local) if backend == "nccl" else torch.device("cpu")   # collective buffers
     B.build()
     culi.load()
-    stream = torch.cuda.current_stream()
     dev = torch.device("cuda", local)
+    # a dedicated (capturable) stream for the whole run: culi_eval_uploaded replays a CUDA graph on it
+    stream = torch.cuda.Stream(device=dev)
+    torch.cuda.set_stream(stream)
 
     # ---- workload + shard (rank r takes forms i mod k == r)
     wl = WORKLOADS[args.workload](world if SCALING[args.workload] == "weak" else 1, rank)

@@ -80,6 +80,7 @@ typedef struct {
 #define CULI_F_NO_NESTED 16u   /* run nested (non-top-level) ||| forms inside one thread (§8(f)1 off)     */
 #define CULI_F_NO_SPLIT  32u   /* no argument splitting: each form is evaluated by one thread only        */
 #define CULI_F_NO_GC     64u   /* do not compact the persistent heap segment after culi_define (§8(f)3)  */
+#define CULI_F_NO_GRAPH 128u   /* culi_eval_uploaded issues its launches directly (no CUDA-graph replay)  */
 
 /* Fill *opts with defaults (device 0, default stream, default sizes). */
 void culi_default_opts(culi_opts* opts);
@@ -119,7 +120,8 @@ int culi_eval_batch(culi_ctx* ctx, const culi_image* forms, culi_results** out);
 
 /* Device-resident variant for timing (bench.py "value"): the image must already be uploaded with
  * culi_upload (done once); each call runs relocate-free dispatch + eval + export on the device and
- * leaves records on the device.  No host copies, no host synchronisation. */
+ * leaves records on the device.  No host copies, no host synchronisation.  On a non-default stream the
+ * first call captures the step into a CUDA graph and later calls replay it (CULI_F_NO_GRAPH: no graph). */
 int culi_upload(culi_ctx* ctx, const culi_image* forms, uint32_t* batch_handle);
 int culi_eval_uploaded(culi_ctx* ctx, uint32_t batch_handle);
 /* Copy the device-resident results of the last culi_eval_uploaded call to the host (synchronises). */

@@ -26,6 +26,11 @@ using namespace culi;
     if (_e != cudaSuccess) return CULI_E_CUDA;  \
   } while (0)
 
+static void drop_graph(culi_ctx* c) {
+  if (c->graph_exec) cudaGraphExecDestroy(c->graph_exec);
+  c->graph_exec = nullptr;
+}
+
 extern "C" {
 
 void culi_default_opts(culi_opts* o) {
@@ -147,6 +152,7 @@ void culi_shutdown(culi_ctx* c) {
   c->roots.release(); c->keys.release(); c->keys_alt.release(); c->perm.release();
   c->perm_alt.release(); c->rtag.release(); c->rerr.release(); c->dtemp.release();
   c->rsteps.release(); c->rword.release(); c->payload.release();
+  drop_graph(c);
   c->rd.release();
   c->gc.release();
   for (auto& e : c->ev) if (e) cudaEventDestroy(e);
@@ -352,11 +358,20 @@ extern "C" int culi_define_text(culi_ctx* c, const char* text, size_t len, int t
   return run_define(c, ro.nforms, ro.nodes, failed_index, failed_err);
 }
 
+// Phase timing events; while the step is being captured into a graph they become external event-record
+// nodes, so culi_last_timing also works after a replay.
+static cudaError_t record_event(culi_ctx* c, int k) {
+  cudaStreamCaptureStatus st = cudaStreamCaptureStatusNone;
+  if (c->stream) cudaStreamIsCapturing(c->stream, &st);
+  if (st == cudaStreamCaptureStatusActive) return cudaEventRecordWithFlags(c->ev[k], c->stream, cudaEventRecordExternal);
+  return cudaEventRecord(c->ev[k], c->stream);
+}
+
 // Run dispatch + eval + export for the uploaded batch (device only, stream-ordered, no host sync).
 static int run_batch_device(culi_ctx* c) {
   uint32_t nf = c->batch_forms;
   c->last_kernels = 0;
-  CK(cudaEventRecord(c->ev[0], c->stream));
+  CK(record_event(c, 0));
   CK(launch_reset(c->stream, c->H.top, c->mark + c->batch_nodes, c->next, c->pcount, c->flags, c->npend,
                   c->nfallback, c->nnest, c->gcount));
   ++c->last_kernels;
@@ -366,7 +381,7 @@ static int run_batch_device(culi_ctx* c) {
                        c->perm_alt.p, c->dtemp.p, c->dtemp.n, &perm, c->sms));
     c->last_kernels += 3;
   }
-  CK(cudaEventRecord(c->ev[1], c->stream));
+  CK(record_event(c, 1));
   EvalArgs A = make_args(c, nf, perm, 0);
   A.fanout = A.fanout && c->batch_has_par;
   if (A.nest) { CK(launch_nest_clear(c->stream, c->ndesc, c->maxnest)); ++c->last_kernels; }
@@ -380,7 +395,7 @@ static int run_batch_device(culi_ctx* c) {
     CK(launch_fanout(c->stream, A, c->nslots / 128));
     c->last_kernels += 2;
   }
-  CK(cudaEventRecord(c->ev[2], c->stream));
+  CK(record_event(c, 2));
   ExportArgs X{};
   X.tag = c->H.tag;
   X.word = c->H.word;
@@ -401,7 +416,7 @@ static int run_batch_device(culi_ctx* c) {
     CK(launch_flat_export(c->stream, A, c->sms * 8));
     c->last_kernels += 2;
   }
-  CK(cudaEventRecord(c->ev[3], c->stream));
+  CK(record_event(c, 3));
   return CULI_OK;
 }
 
@@ -410,6 +425,7 @@ static int run_batch_device(culi_ctx* c) {
 // cell / of some cell other than a top-level form's first cell; par_head: some form is (||| ...).
 static int finish_prepare(culi_ctx* c, uint32_t nf, uint64_t nnodes, std::string strings, bool par_any,
                           bool par_nonroot, bool par_head, bool has_wide) {
+  drop_graph(c);
   int rc = ensure_results(c, nf);
   if (rc) return rc;
   size_t n = std::max<uint32_t>(nf, 1);
@@ -639,9 +655,32 @@ int culi_upload(culi_ctx* c, const culi_image* forms, uint32_t* handle) {
   return CULI_OK;
 }
 
+// Repeated evaluation of one uploaded batch replays a CUDA graph of the whole device step (reset, dispatch,
+// eval, fan-out, export: ~10 launches), captured on the first call; small batches are launch-bound.
+// The legacy default stream cannot be captured: there the launches are issued directly.
 int culi_eval_uploaded(culi_ctx* c, uint32_t handle) {
   if (!c || handle != 1 || !c->have_batch) return CULI_E_STATE;
-  return run_batch_device(c);
+  if (!c->stream || (c->opts.flags & CULI_F_NO_GRAPH)) return run_batch_device(c);
+  if (!c->graph_exec) {
+    CK(cudaStreamBeginCapture(c->stream, cudaStreamCaptureModeThreadLocal));
+    int rc = run_batch_device(c);
+    cudaGraph_t g = nullptr;
+    cudaError_t e = cudaStreamEndCapture(c->stream, &g);
+    if (rc || e != cudaSuccess || !g) {
+      if (g) cudaGraphDestroy(g);
+      return rc ? rc : CULI_E_CUDA;
+    }
+    e = cudaGraphInstantiate(&c->graph_exec, g, 0);
+    cudaGraphDestroy(g);
+    if (e != cudaSuccess) {
+      c->graph_exec = nullptr;
+      return CULI_E_CUDA;
+    }
+    c->graph_kernels = c->last_kernels;
+  }
+  CK(cudaGraphLaunch(c->graph_exec, c->stream));
+  c->last_kernels = c->graph_kernels;
+  return CULI_OK;
 }
 
 int culi_fetch_results(culi_ctx* c, uint32_t handle, culi_results** out) {
@@ -652,6 +691,7 @@ int culi_fetch_results(culi_ctx* c, uint32_t handle, culi_results** out) {
 
 int culi_release(culi_ctx* c, uint32_t handle) {
   if (!c || handle != 1) return CULI_E_STATE;
+  drop_graph(c);
   c->have_batch = false;
   return CULI_OK;
 }

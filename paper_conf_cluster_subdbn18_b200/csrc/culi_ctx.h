@@ -155,6 +155,8 @@ struct culi_ctx {
   std::string batch_strings;
   ReaderState rd;
   GcState gc;
+  cudaGraphExec_t graph_exec = nullptr;  // culi_eval_uploaded replay of the uploaded batch
+  uint32_t graph_kernels = 0;
   // timing
   cudaEvent_t ev[4] = {nullptr, nullptr, nullptr, nullptr};
   uint32_t last_kernels = 0;

@@ -271,6 +271,35 @@ def test_upload_eval_fetch_repeatable(culi, oracle_mod):
     ctx.release(h)
 
 
+@pytest.mark.parametrize("cfg", ["c1", "c3", "c5"])
+def test_graph_replay_on_a_stream(culi, oracle_mod, cfg):
+    """culi_eval_uploaded on a non-default stream captures the device step into a CUDA graph and replays
+    it: same results as direct launches (CULI_F_NO_GRAPH) and the oracle."""
+    import torch
+    wl = {"c1": lambda: W.c1(), "c3": lambda: W.c3(3000), "c5": lambda: W.c5(4000)}[cfg]()
+    s = torch.cuda.Stream()
+    out = []
+    for flags in (0, culi.CULI_F_NO_GRAPH):
+        ctx = culi.Context(**SMALL, stream=s.cuda_stream, flags=flags)
+        if wl.defs:
+            ctx.define(wl.defs)
+        h = ctx.upload(wl.forms)
+        for _ in range(4):
+            ctx.eval_uploaded(h)
+        r = ctx.fetch_results(h)
+        out.append((r.printed(), r.steps()))
+        ctx.eval_uploaded(h)                    # a replay after a fetch is still valid
+        r2 = ctx.fetch_results(h)
+        assert (r2.printed(), r2.steps()) == out[-1]
+        ctx.release(h)
+        ctx.close()
+    assert out[0] == out[1]
+    o = oracle_mod.Session()
+    if wl.defs:
+        o.define(wl.defs)
+    assert not compare(out[0][0], out[0][1], o.eval(wl.forms))
+
+
 def test_wide_forms(culi, oracle_mod):
     """Top-level forms with >= 64 arguments take the wide path (arguments one per thread, K12)."""
     rnd = random.Random(77)
