@@ -21,4 +21,16 @@ for flags in (0, culi.CULI_F_NO_BINNING | culi.CULI_F_NO_FANOUT):
     r = c2.eval_batch(forms)
     print(len(r), r.totals())
     c2.close()
+# device reader (§8(f)2) incl. strings, quotes, comments, floats needing the big-integer path, and heap
+# reclamation (§8(f)3) after the definitions
+text = forms + "\n" + "\n".join(['"a (b) ; c"', "'(x . y)", "; comment\n(list 1 2.5 \"s\")",
+                                   "1.00000000000000000000000000000000000001e-300", "(quote (1 (2 (3))))"])
+for flags in (0, culi.CULI_F_NO_GC):
+    c3 = culi.Context(slots=148 * 128, heap_nodes=1 << 22, vstack_entries=1024, flags=flags)
+    c3.define_text(defs)
+    c3.define_text("(define tmp (list 1 2 3))\n(define tmp (reverse tmp))")
+    c3.collect()
+    r = c3.eval_text(text)
+    print(len(r), r.totals(), c3.heap_usage())
+    c3.close()
 print("done")
