@@ -71,8 +71,9 @@ struct Val {
 struct Cell { Val car, cdr; };                       // PAPER L326-333 Fig.2 (a cons cell)
 struct Closure { Val params; Val body; const Frame* env; };   // c.5 lambda / defmacro (lexical env)
 struct Frame {                                       // PAPER L383-398 §III-B.a Fig.6-7: (symbol,value)
-  const Frame* parent;                               // pairs plus a parent link; immutable (c.3)
-  std::vector<std::pair<uint32_t, Val>> binds;
+  const Frame* parent;                               // pairs plus a parent link; only setq changes a
+  std::vector<std::pair<uint32_t, Val>> binds;       // value (L408-413, R7)
+  bool persistent;                                   // created while defining (culi_define)
 };
 
 struct LispError { int code; };
@@ -87,9 +88,9 @@ struct Arena {
 };
 
 // ---- reserved names: special forms (c.5) then builtins (c.6) -------------------------------------
-enum Special { S_QUOTE, S_IF, S_DEFINE, S_DEFUN, S_DEFMACRO, S_LAMBDA, S_LET, S_PROGN, N_SPECIAL };
+enum Special { S_QUOTE, S_IF, S_DEFINE, S_DEFUN, S_DEFMACRO, S_LAMBDA, S_LET, S_PROGN, S_SETQ, N_SPECIAL };
 static const char* kSpecialNames[N_SPECIAL] = {"quote", "if", "define", "defun", "defmacro",
-                                               "lambda", "let", "progn"};
+                                               "lambda", "let", "progn", "setq"};
 enum Builtin {
   B_ADD, B_SUB, B_MUL, B_DIV, B_REM, B_MOD, B_SQRT, B_FLOAT, B_TRUNC,
   B_NUM_EQ, B_LT, B_GT, B_LE, B_GE, B_EQ, B_EQUAL, B_NULL, B_NOT,
@@ -389,7 +390,7 @@ struct Interp {
     }
   }
   Frame* new_frame(const Frame* parent) {
-    A.frames.push_back(Frame{parent, {}});
+    A.frames.push_back(Frame{parent, {}, define_mode});
     return &A.frames.back();
   }
 
@@ -465,6 +466,26 @@ struct Interp {
         Val r = mk_nil();
         for (Val x : a) r = eval(x, env, depth + 1);
         return r;
+      }
+      case S_SETQ: {
+        // "setq updates the nearest existing symbol that matches" — a local variable or,
+        // failing that, the global one.  DESIGN.md R7: the value is evaluated first; during a batch the
+        // global frame and frames made while defining are read-only (DEFINE_IN_BATCH), so independent
+        // forms share no mutable state; with no binding anywhere, a define-time setq creates the global.
+        if (n != 2 || !bindable(a[0])) fail(E_SYNTAX);
+        Val v = eval(a[1], env, depth + 1);
+        uint32_t sym = a[0].sym;
+        for (const Frame* f = env; f; f = f->parent)
+          for (auto& b : f->binds)
+            if (b.first == sym) {
+              if (!define_mode && f->persistent) fail(E_DEFINE_IN_BATCH);
+              const_cast<std::pair<uint32_t, Val>&>(b).second = v;
+              return v;
+            }
+        if (!define_mode) fail(E_DEFINE_IN_BATCH);
+        S.global_val[sym] = v;
+        S.global_bound[sym] = 1;
+        return v;
       }
     }
     fail(E_SYNTAX);

@@ -365,3 +365,50 @@ def test_generated_batches_run_clean(oracle_mod):
         res = s.eval(wl.forms)
         assert len(res) == wl.nforms
         assert all(r.err == 0 for r in res), [r for r in res if r.err][:3]
+
+
+SETQ_DEFS = "\n".join([
+    "(define make-counter (lambda () (let ((n 0)) (lambda () (setq n (+ n 1))))))",
+    "(define counter (let ((n 0)) (lambda () (setq n (+ n 1)))))",
+    "(define g 7)",
+    "(define k1 (counter))",
+    "(define k2 (counter))",
+])
+
+
+@pytest.fixture(scope="module")
+def setq_sess(oracle_mod):
+    s = oracle_mod.Session()
+    s.define(SETQ_DEFS)
+    return s
+
+
+@pytest.mark.parametrize("row", load_tsv("setq_pins.tsv"), ids=lambda r: r[0][:40])
+def test_setq_pins(setq_sess, row):
+    """setq under reading R7: hand-derived values and step counts."""
+    r = setq_sess.eval1(row[0])
+    assert (r.printed, r.steps) == (row[1], int(row[2])), row
+
+
+def test_setq_define_time_globals(oracle_mod):
+    """At define time setq updates (or creates) the global binding; batches see the result (L408-413)."""
+    s = oracle_mod.Session()
+    s.define("(define a 1)\n(setq a (+ a 41))\n(setq fresh 'made)\n(define f (lambda () a))")
+    assert [r.printed for r in s.eval("a\nfresh\n(f)")] == ["42", "made", "42"]
+
+
+def test_setq_counter_closed_form(oracle_mod):
+    """A counter closure called k times in one form returns k; steps = 9 + 8k (let 2 + make-counter 7 + k calls)."""
+    s = oracle_mod.Session()
+    s.define(SETQ_DEFS)
+    for k in (1, 2, 5, 17):
+        r = s.eval1("(let ((c (make-counter))) %s)" % " ".join(["(c)"] * k))
+        assert (r.printed, r.steps) == (str(k), 9 + 8 * k)
+
+
+def test_setq_forms_are_independent(oracle_mod):
+    """Two forms of one batch each get their own counter: no state leaks between independent forms."""
+    s = oracle_mod.Session()
+    s.define(SETQ_DEFS)
+    out = [r.printed for r in s.eval("(let ((c (make-counter))) (c) (c))\n(let ((c (make-counter))) (c))")]
+    assert out == ["2", "1"]
