@@ -208,6 +208,11 @@ static bool image_mentions_par(const Image& img, bool skip_root_heads = false) {
     if ((img.tag[k] & KIND_MASK) == K_CONS && !root[k] && (uint32_t)img.word[k] == par) return true;
   return false;
 }
+static bool image_mentions_setq(const Image& img) {
+  for (size_t k = 0; k < img.tag.size(); ++k)
+    if ((img.tag[k] & KIND_MASK) == K_SYM && img.word[k] == SP_SETQ) return true;
+  return false;
+}
 static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, int define_mode) {
   EvalArgs A{};
   A.H = c->H;
@@ -245,6 +250,16 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.vst2 = c->vst2;
   A.finished = c->nnest + 1;
   A.split = (!define_mode && !(c->opts.flags & CULI_F_NO_SPLIT)) ? 1 : 0;
+  // setq (R7): frames go to the heap when made, and a form runs in one thread only (no fan-out, nested
+  // fan-out or argument splitting: those evaluate parts of a form elsewhere, on copies of its frames)
+  A.mut = define_mode ? c->define_mut : c->batch_mut;
+  A.pmark = (uint32_t)c->mark;
+  if (A.mut && !define_mode) {
+    A.fanout = 0;
+    A.nest = 0;
+    A.split = 0;
+    A.wide = nullptr;
+  }
   A.split_poll = c->split_poll;
   A.split_sleep = c->split_sleep;
   A.groups = c->groups;
@@ -344,6 +359,8 @@ extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed
   if (rc) return rc;
   c->strings += img.strings;
   c->persist_has_par = c->persist_has_par || image_mentions_par(img);
+  c->define_mut = c->persist_has_setq || image_mentions_setq(img);
+  c->persist_has_setq = c->define_mut;
   return run_define(c, nf, img.tag.size(), failed_index, failed_err);
 }
 
@@ -355,6 +372,8 @@ extern "C" int culi_define_text(culi_ctx* c, const char* text, size_t len, int t
   if (rc) return rc;
   c->strings += ro.strings;
   c->persist_has_par = c->persist_has_par || ro.par_root_head || ro.par_nested;
+  c->define_mut = c->persist_has_setq || ro.setq;
+  c->persist_has_setq = c->define_mut;
   return run_define(c, ro.nforms, ro.nodes, failed_index, failed_err);
 }
 
@@ -424,7 +443,8 @@ static int run_batch_device(culi_ctx* c) {
 // host image or written by the device reader).  par_any / par_nonroot: the ||| symbol is the car of some
 // cell / of some cell other than a top-level form's first cell; par_head: some form is (||| ...).
 static int finish_prepare(culi_ctx* c, uint32_t nf, uint64_t nnodes, std::string strings, bool par_any,
-                          bool par_nonroot, bool par_head, bool has_wide) {
+                          bool par_nonroot, bool par_head, bool has_wide, bool setq) {
+  c->batch_mut = c->persist_has_setq || setq;
   drop_graph(c);
   int rc = ensure_results(c, nf);
   if (rc) return rc;
@@ -482,7 +502,7 @@ static int prepare_batch(culi_ctx* c, const Image& img) {
     CK(cudaMemcpyAsync(c->wide.p, wide.data(), nf * 4, cudaMemcpyHostToDevice, c->stream));
   }
   return finish_prepare(c, nf, img.tag.size(), img.strings, image_mentions_par(img, false),
-                        image_mentions_par(img, true), par_head, has_wide);
+                        image_mentions_par(img, true), par_head, has_wide, image_mentions_setq(img));
 }
 
 // Device reader (§8(f)2) -> the same prepared batch.
@@ -491,7 +511,7 @@ static int prepare_text(culi_ctx* c, const char* text, size_t len, bool on_devic
   int rc = device_read(c, text, len, on_device, &ro, err_offset);
   if (rc) return rc;
   return finish_prepare(c, ro.nforms, ro.nodes, std::move(ro.strings), ro.par_root_head || ro.par_nested,
-                        ro.par_nested, ro.par_root_head, ro.wide);
+                        ro.par_nested, ro.par_root_head, ro.wide, ro.setq);
 }
 
 // ||| forms the fan-out could not decide (an element error, fuel overflow, a short or non-contiguous

@@ -132,6 +132,8 @@ struct culi_ctx {
   bool batch_has_wide = false;
   // nested ||| (§8(f)1)
   bool persist_has_par = false;      // some definition mentions |||
+  bool persist_has_setq = false;     // some definition mentions setq (R7: batches run with heap frames)
+  bool batch_mut = false, define_mut = false;
   bool batch_may_nest = false;
   NestDesc* ndesc = nullptr;
   uint32_t maxnest = 4096;

@@ -62,6 +62,8 @@ struct EvalArgs {
   uint32_t max_depth;
   uint64_t fuel;
   int define_mode;
+  uint32_t mut;                // setq may run: every frame lives in the heap from creation
+  uint32_t pmark;              // heap nodes below this index are persistent (read-only for a batch's setq)
   int* flags;                  // [0] heap/stack exhausted, [1] define: index of failing form + 1, [2] its err
   uint32_t voting;             // warp opcode voting on/off
   uint32_t fanout;             // top-level ||| forms fan out over threads (batch eval kernel only)

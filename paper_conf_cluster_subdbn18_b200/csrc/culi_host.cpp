@@ -17,7 +17,7 @@
 namespace culi {
 
 const char* const kSpecialName[N_SPECIALS] = {"quote", "if", "define", "defun", "defmacro", "lambda",
-                                              "let", "progn"};
+                                              "let", "progn", "setq"};
 const char* const kBuiltinName[N_BUILTINS] = {
     "+", "-", "*", "/", "rem", "mod", "sqrt", "float", "trunc",
     "=", "<", ">", "<=", ">=", "eq", "equal", "null", "not",
@@ -140,7 +140,8 @@ struct Builder {
       case SP_IF: return n == 2 || n == 3;
       case SP_PROGN: return true;
       case SP_LAMBDA: return n >= 1 && params_ok(xs[1]);
-      case SP_DEFINE: return n == 2 && bindable(xs[1]);
+      case SP_DEFINE:
+      case SP_SETQ: return n == 2 && bindable(xs[1]);
       case SP_DEFUN:
       case SP_DEFMACRO: return n >= 2 && bindable(xs[1]) && params_ok(xs[2]);
       case SP_LET: {

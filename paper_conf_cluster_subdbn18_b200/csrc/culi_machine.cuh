@@ -275,6 +275,38 @@ __device__ CULI_COLD bool make_closure(Ctx C, uint32_t kind, uint32_t code, uint
   return true;
 }
 
+// (setq s v) after v was evaluated (R7): the innermost, leftmost binding of s in env; else the global.
+// In a batch, globals and frames made while defining (heap index < pmark) are read-only.
+__device__ CULI_COLD uint8_t setq_store(Ctx C, uint32_t sym, uint32_t env, V v) {
+  const DevHeap& H = C.A->H;
+  while (env != 0) {
+    if (env & STACK_ENV) {                                      // (frames are in the heap when mut is set)
+      uint32_t h = env & ENV_IDX_MASK, n = (env >> 16) & 0x7fffu;
+      for (uint32_t i = 1; i <= n; ++i) {
+        uint4* e = VS(C, h + i);
+        if (e->z == sym) { *e = vpack(v, sym); return 0; }
+      }
+      env = VS(C, h)->x;
+    } else {
+      uint64_t hw = nword(C, env);
+      uint32_t n = hi32(hw);
+      for (uint32_t i = 1; i <= n; ++i) {
+        uint64_t bw = nword(C, env + i);
+        if (lo32(bw) != sym) continue;
+        if (!C.A->define_mode && env < C.A->pmark) return E_DEFINE_IN_BATCH;
+        uint32_t vn = box_into(H, v, env + n + i);              // the binding's own value slot
+        H.word[env + i] = pack2(sym, vn);
+        return 0;
+      }
+      env = lo32(hw);
+    }
+  }
+  if (!C.A->define_mode) return E_DEFINE_IN_BATCH;
+  H.gtag[sym] = (uint8_t)v.t;
+  H.gword[sym] = v.w;
+  return 0;
+}
+
 // c.5: a parameter list is a proper list of non-reserved symbols
 __device__ CULI_COLD bool valid_params(Ctx C, uint32_t ps) {
   if (ps == 0) return true;
@@ -674,7 +706,8 @@ __device__ CULI_COLD bool special_syntax_ok(Ctx C, uint32_t op, uint32_t cur) {
     case SP_IF: return n == 2 || n == 3;
     case SP_PROGN: return true;
     case SP_LAMBDA: return n >= 1 && valid_params(C, car_of(C, cur));
-    case SP_DEFINE: return n == 2 && bindable_node(C, car_of(C, cur));
+    case SP_DEFINE:
+    case SP_SETQ: return n == 2 && bindable_node(C, car_of(C, cur));
     case SP_DEFUN: case SP_DEFMACRO:
       return n >= 2 && bindable_node(C, car_of(C, cur)) && valid_params(C, car_of(C, cdr_of(C, cur)));
     case SP_LET: {
@@ -761,7 +794,7 @@ __device__ __forceinline__ int try_leaf(const Ctx& C, uint32_t xt, uint64_t xw, 
 
 // ---- the machine ---------------------------------------------------------------------------------------
 enum KKind : uint32_t { KF_HEAD = 1, KF_ARGS, KF_BODY, KF_IF, KF_LET, KF_DEFINE, KF_MACRO, KF_PAR, KF_DATA,
-                       KF_JOIN };   // KF_JOIN: a KF_ARGS frame whose next argument was split off
+                       KF_JOIN, KF_SETQ };   // KF_JOIN: a KF_ARGS frame whose next argument was split off
 
 // ---- argument splitting ----------------------------------------------------------------
 __device__ __forceinline__ uint32_t ld_acquire(const uint32_t* p) {
@@ -893,6 +926,8 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32
   uint32_t pollc = SPLIT ? C.A->split_poll : 0;   // closure calls until the next split poll
 
 #define FAIL(e) do { err = (e); goto done; } while (0)
+// setq batches (R7): a frame moves to the heap as soon as it is made, so that no copy of it can go stale
+#define MUT_FRAME() do { uint32_t h_; if (__builtin_expect(!!(!promote(C, env, &h_)), 0)) FAIL(E_OOM); env = h_; } while (0)
 #define STEP(depth)                                     \
   do {                                                  \
     ++steps;                                            \
@@ -1085,6 +1120,13 @@ HEAD:
         cur = bl;
         goto LET_LOOP;
       }
+      case SP_SETQ: {                                           // R7: the value first, then the binding
+        w0 = nword(C, cur);
+        KPUSH(KF_SETQ, (uint32_t)nword(C, lo32(w0)), env, vtop, d, 0);
+        x = car_of(C, hi32(w0));
+        d = d + 1;
+        goto EVAL_NODE;
+      }
       case SP_DEFINE: {
         w0 = nword(C, cur);
         KPUSH(KF_DEFINE, (uint32_t)nword(C, lo32(w0)), env, vtop, d, 0);
@@ -1124,6 +1166,7 @@ HEAD:
     *VS(C, hdr) = make_uint4(menv, 0, n, K_FRAME);
     KPUSH(KF_MACRO, 0, env, hdr, d, 0);
     env = stack_env(hdr, n);
+    if (C.A->mut) MUT_FRAME();
     vtop = hdr + 1 + n;
     cur = body;
     goto BODY;
@@ -1210,6 +1253,7 @@ APPLY: {                                                        // apply vs[base
     if (__builtin_expect(!!(cnt >= 0x8000u), 0)) FAIL(E_OOM);
     *VS(C, base) = make_uint4(hi32(cwd), 0, cnt, K_FRAME);
     env = stack_env(base, cnt);
+    if (C.A->mut) MUT_FRAME();
     vtop = base + 1 + cnt;
     cur = body;
     goto BODY;
@@ -1363,6 +1407,7 @@ LET_LOOP:
   cur = VS(C, base)->x;                                         // body list stored in the header
   *VS(C, base) = make_uint4(env, 0, cnt, K_FRAME);
   env = stack_env(base, cnt);
+  if (C.A->mut) MUT_FRAME();
   vtop = base + 1 + cnt;
   goto BODY;
 
@@ -1481,6 +1526,12 @@ RET:
       ++cnt;
       cur = hi32(w0); env = k.y; d = kd;
       goto LET_LOOP;
+    }
+    case KF_SETQ: {
+      uint8_t e = setq_store(C, k.x, k.y, v);
+      if (__builtin_expect(!!(e), 0)) FAIL(e);
+      vtop = k.z;
+      goto RET;
     }
     case KF_DEFINE:
       H.gtag[k.x] = (uint8_t)v.t;
