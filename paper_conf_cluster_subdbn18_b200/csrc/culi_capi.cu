@@ -449,8 +449,8 @@ static int finish_prepare(culi_ctx* c, uint32_t nf, uint64_t nnodes, std::string
   int rc = ensure_results(c, nf);
   if (rc) return rc;
   size_t n = std::max<uint32_t>(nf, 1);
-  CK(c->keys.ensure(n));
-  CK(c->keys_alt.ensure(n));
+  CK(c->keys.ensure(2 * n));                         // 64-bit dispatch keys
+  CK(c->keys_alt.ensure(2 * n));
   CK(c->perm.ensure(n));
   CK(c->perm_alt.ensure(n));
   CK(c->dtemp.ensure(dispatch_temp_bytes(nf)));

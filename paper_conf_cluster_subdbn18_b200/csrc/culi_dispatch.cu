@@ -1,11 +1,12 @@
 // culi_dispatch.cu — classify + bin the forms of a batch before evaluation.
 //
 // The paper notes that divergent branches of a warp are serialised (§III-D.d).  Forms are
-// independent, so their evaluation order is free: we give each form a 32-bit key
-//   (head class << 16) | (0xffff - cost hint)
+// independent, so their evaluation order is free: we give each form a 64-bit key
+//   (head class << 48) | (shape hash << 16) | (0xffff - cost hint)
 // where the head class is the form's head symbol (user functions first, then reserved builtins, then
-// atoms / data), and the cost hint is the first argument when it is an integer literal (e.g. n of
-// (fib n)), so forms whose control flow is identical land in the same warp, heaviest first.  A radix
+// atoms / data), the shape hash covers the form's tree (kinds, symbols, structure; not number values),
+// and the cost hint is the first argument when it is an integer literal (e.g. n of (fib n)), so forms
+// whose control flow is identical land in the same warp, heaviest first.  A radix
 // sort (CUB, a plain library sort) of (key, form) gives the evaluation permutation; each warp of the
 // eval kernel then takes 32 consecutive forms of it.
 #include <cub/device/device_radix_sort.cuh>
@@ -15,13 +16,41 @@
 
 namespace culi {
 
+// Shape of a form: FNV-1a over a pre-order walk of its first 48 nodes — node kinds, symbol ids, list
+// structure; numbers contribute only their kind (their values are in the hint).  Forms with equal shape
+// expand macros and take calls in the same order, so a warp of them stays converged longer (C4).
+__device__ uint32_t shape_hash(const uint8_t* __restrict__ tag, const uint64_t* __restrict__ word, uint32_t x) {
+  uint32_t st[12];
+  int sp = 0;
+  uint32_t h = 2166136261u;
+  for (int visited = 0; visited < 48; ++visited) {
+    uint32_t t = tag[x] & KIND_MASK;
+    h = (h ^ t) * 16777619u;
+    if (t == K_SYM) h = (h ^ (uint32_t)word[x]) * 16777619u;
+    if (t == K_CONS) {
+      uint64_t w = word[x];
+      uint32_t cdr = (uint32_t)(w >> 32);
+      if (cdr) {
+        if (sp < 12) st[sp++] = cdr;
+        else h = (h ^ 0x9e3779b9u) * 16777619u;
+      }
+      x = (uint32_t)w;
+      continue;
+    }
+    if (sp == 0) break;
+    x = st[--sp];
+    h = (h ^ 0x55u) * 16777619u;                      // a subtree ended: keeps (a (b) c) != (a (b c))
+  }
+  return h;
+}
+
 __global__ void culi_classify_kernel(const uint8_t* __restrict__ tag, const uint64_t* __restrict__ word,
                                      const uint32_t* __restrict__ roots, uint32_t nforms,
-                                     uint32_t* __restrict__ keys, uint32_t* __restrict__ perm) {
+                                     unsigned long long* __restrict__ keys, uint32_t* __restrict__ perm) {
   uint32_t stride = gridDim.x * blockDim.x;
   for (uint32_t f = blockIdx.x * blockDim.x + threadIdx.x; f < nforms; f += stride) {
     uint32_t r = roots[f];
-    uint32_t cls = 0xffff, hint = 0;
+    uint32_t cls = 0xffff, hint = 0, shape = 0;
     if ((tag[r] & KIND_MASK) == K_CONS) {
       uint64_t w = word[r];
       uint32_t h = (uint32_t)w, rest = (uint32_t)(w >> 32);
@@ -42,30 +71,35 @@ __global__ void culi_classify_kernel(const uint8_t* __restrict__ tag, const uint
           if ((tag[ah] & KIND_MASK) == K_SYM) hint = 0xff00u | ((uint32_t)word[ah] & 0xff);
         }
       }
+      shape = shape_hash(tag, word, r);
     }
-    keys[f] = (cls << 16) | (0xffffu - hint);
+    keys[f] = ((unsigned long long)cls << 48) | ((unsigned long long)shape << 16) | (0xffffu - hint);
     perm[f] = f;
   }
 }
 
 size_t dispatch_temp_bytes(uint32_t nforms) {
   size_t bytes = 0;
-  cub::DeviceRadixSort::SortPairs((void*)nullptr, bytes, (const uint32_t*)nullptr, (uint32_t*)nullptr,
-                                  (const uint32_t*)nullptr, (uint32_t*)nullptr, (int)nforms);
+  cub::DeviceRadixSort::SortPairs((void*)nullptr, bytes, (const unsigned long long*)nullptr,
+                                  (unsigned long long*)nullptr, (const uint32_t*)nullptr, (uint32_t*)nullptr,
+                                  (int)nforms);
   return bytes + 256;
 }
 
 cudaError_t launch_dispatch(cudaStream_t s, const DevHeap& H, const uint32_t* roots, uint32_t nforms,
                             uint32_t* keys, uint32_t* keys_alt, uint32_t* perm, uint32_t* perm_alt,
                             void* temp, size_t temp_bytes, uint32_t** perm_out, int sms) {
+  // keys / keys_alt hold 2 x nforms words each (64-bit keys)
+  unsigned long long* k0 = reinterpret_cast<unsigned long long*>(keys);
+  unsigned long long* k1 = reinterpret_cast<unsigned long long*>(keys_alt);
   uint32_t blocks = (nforms + 255) / 256;
   if (blocks > (uint32_t)sms * 8) blocks = sms * 8;
   if (blocks == 0) blocks = 1;
-  culi_classify_kernel<<<blocks, 256, 0, s>>>(H.tag, H.word, roots, nforms, keys, perm);
+  culi_classify_kernel<<<blocks, 256, 0, s>>>(H.tag, H.word, roots, nforms, k0, perm);
   cudaError_t e = cudaGetLastError();
   if (e != cudaSuccess) return e;
   size_t tb = temp_bytes;
-  e = cub::DeviceRadixSort::SortPairs(temp, tb, keys, keys_alt, perm, perm_alt, (int)nforms, 0, 32, s);
+  e = cub::DeviceRadixSort::SortPairs(temp, tb, k0, k1, perm, perm_alt, (int)nforms, 0, 64, s);
   *perm_out = perm_alt;
   return e;
 }
