@@ -10,11 +10,72 @@
 #include <cmath>
 #include <cstdlib>
 #include <cstring>
+#include <map>
+#include <mutex>
+#include <unordered_map>
+
+#include <cuda_runtime.h>
 
 #include "../../include/culi.h"
 #include "culi_host.h"
 
 namespace culi {
+
+// ---- page-locked block cache for result arrays (culi_host.h ResultAlloc) --------------------------------
+namespace {
+constexpr size_t PIN_MIN = 1u << 20;             // smaller arrays: plain heap
+constexpr size_t PIN_CACHE_MAX = 8ull << 30;     // cached (free) pinned bytes kept at most
+struct PinCache {
+  std::mutex mu;
+  std::multimap<size_t, void*> free_blocks;      // capacity -> block
+  std::unordered_map<void*, size_t> cap;         // block -> capacity (pinned blocks only)
+  size_t cached = 0;
+};
+PinCache& pin_cache() {
+  static PinCache* c = new PinCache;             // never destroyed: frees may run at exit
+  return *c;
+}
+}  // namespace
+
+void* pinned_pool_alloc(size_t bytes) {
+  if (bytes < PIN_MIN) return ::operator new(bytes ? bytes : 1);
+  PinCache& C = pin_cache();
+  {
+    std::lock_guard<std::mutex> g(C.mu);
+    auto it = C.free_blocks.lower_bound(bytes);
+    if (it != C.free_blocks.end() && it->first <= 2 * bytes) {
+      void* p = it->second;
+      C.cached -= it->first;
+      C.free_blocks.erase(it);
+      return p;
+    }
+  }
+  size_t cap = size_t(1) << (64 - __builtin_clzll(bytes - 1));   // next power of two
+  void* p = nullptr;
+  if (cudaHostAlloc(&p, cap, cudaHostAllocDefault) != cudaSuccess) {
+    cudaGetLastError();
+    return ::operator new(bytes);                // no device / no pinned memory: plain heap
+  }
+  std::lock_guard<std::mutex> g(C.mu);
+  C.cap[p] = cap;
+  return p;
+}
+
+void pinned_pool_free(void* p, size_t bytes) {
+  if (!p) return;
+  if (bytes < PIN_MIN) { ::operator delete(p); return; }
+  PinCache& C = pin_cache();
+  std::lock_guard<std::mutex> g(C.mu);
+  auto it = C.cap.find(p);
+  if (it == C.cap.end()) { ::operator delete(p); return; }
+  if (C.cached + it->second > PIN_CACHE_MAX) {
+    C.cap.erase(it);
+    cudaFreeHost(p);
+    return;
+  }
+  C.cached += it->second;
+  C.free_blocks.emplace(it->second, p);
+}
 
 const char* const kSpecialName[N_SPECIALS] = {"quote", "if", "define", "defun", "defmacro", "lambda",
                                               "let", "progn", "setq"};

@@ -5,6 +5,7 @@
 #include <memory>
 #include <string>
 #include <unordered_map>
+#include <utility>
 #include <vector>
 
 #include "culi_internal.h"
@@ -52,14 +53,39 @@ struct Token {
   uint32_t pad;
 };
 
+// Host memory for result arrays: large blocks come from a process-wide cache of page-locked blocks (so the
+// device -> host copies of a fetch run at DMA speed and repeated fetches neither re-pin nor page-fault),
+// and elements are default-initialised (a fetch overwrites them; no zero fill).  culi_host.cpp.
+void* pinned_pool_alloc(size_t bytes);
+void pinned_pool_free(void* p, size_t bytes);
+template <typename T>
+struct ResultAlloc {
+  using value_type = T;
+  ResultAlloc() = default;
+  template <typename U>
+  ResultAlloc(const ResultAlloc<U>&) {}
+  T* allocate(size_t n) { return static_cast<T*>(pinned_pool_alloc(n * sizeof(T))); }
+  void deallocate(T* p, size_t n) { pinned_pool_free(p, n * sizeof(T)); }
+  template <typename U>
+  void construct(U* p) { ::new (static_cast<void*>(p)) U; }   // default-init: no zeroing
+  template <typename U, typename... A>
+  void construct(U* p, A&&... a) { ::new (static_cast<void*>(p)) U(std::forward<A>(a)...); }
+  template <typename U>
+  bool operator==(const ResultAlloc<U>&) const { return true; }
+  template <typename U>
+  bool operator!=(const ResultAlloc<U>&) const { return false; }
+};
+template <typename T>
+using rvec = std::vector<T, ResultAlloc<T>>;
+
 struct Results {
   // records as structure of arrays, so the device arrays are copied straight in (no per-record work)
-  std::vector<uint8_t> tag, err;
-  std::vector<uint64_t> steps, word;
+  rvec<uint8_t> tag, err;
+  rvec<uint64_t> steps, word;
   size_t size() const { return tag.size(); }
   Record at(size_t i) const { return Record{tag[i], err[i], steps[i], word[i]}; }
   void resize(size_t n) { tag.resize(n); err.resize(n); steps.resize(n); word.resize(n); }
-  std::vector<Token> payload;
+  rvec<Token> payload;
   std::shared_ptr<const SymTable> syms;   // names for SYM tokens
   std::string strings;                    // bytes for STR tokens
   void print(uint32_t i, std::string& out) const;
