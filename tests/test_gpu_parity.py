@@ -155,6 +155,36 @@ def test_c5_large(culi, oracle_mod):
     assert_parity(culi, oracle_mod, wl.defs, wl.forms, ctx_kw=dict(heap_nodes=1 << 27))
 
 
+def test_c5_full_size(culi, oracle_mod):
+    """configs[4] at full size (16,777,216 forms) in the bench's launch configuration, read on the device
+    (the e2e path): every (fib n) / (fact n) form against its closed form (value and step count, pinned in
+    test_oracle_pins), and a sample of every kind against the oracle."""
+    import math
+    wl = W.c5()
+    ctx = culi.Context(heap_nodes=1 << 30)
+    ctx.define(wl.defs)
+    res = ctx.eval_text(wl.forms)
+    lines = wl.form_lines()
+    assert len(res) == len(lines) == 16777216
+    _, nerr = res.totals()
+    idx_closed = [i for i in range(0, len(lines), 997) if lines[i].startswith(("(fib ", "(fact "))]
+    for i in idx_closed:
+        t, e, st = res.info(i)
+        n = int(lines[i].split()[1][:-1])
+        if lines[i].startswith("(fib "):
+            assert (res.int_value(i), st) == (fib_py(n), 27 * fib_py(n + 1) - 17), lines[i]
+        else:
+            w = (math.factorial(n) + 2 ** 63) % 2 ** 64 - 2 ** 63
+            assert (res.int_value(i), st) == (w, 15 * n - 5 if n >= 2 else 10), lines[i]
+    s = oracle_mod.Session()
+    s.define(wl.defs)
+    rnd = random.Random(7)
+    idx = sorted(rnd.sample(range(len(lines)), 3000))
+    o = s.eval("\n".join(lines[i] for i in idx))
+    bad = compare([res.print(i) for i in idx], [res.info(i)[2] for i in idx], o)
+    assert not bad, bad
+
+
 def test_c0(culi, oracle_mod):
     for n in (1, 31, 32, 33, 1000, 4096):
         wl = W.c0(n)
