@@ -1,8 +1,8 @@
 // culi_dispatch.cu — classify + bin the forms of a batch before evaluation.
 //
 // The paper notes that divergent branches of a warp are serialised (§III-D.d).  Forms are
-// independent, so their evaluation order is free: we give each form a 64-bit key
-//   (head class << 48) | (shape hash << 16) | (0xffff - cost hint)
+// independent, so their evaluation order is free: we give each form a 48-bit key
+//   (head class << 32) | (16-bit shape hash << 16) | (0xffff - cost hint)
 // where the head class is the form's head symbol (user functions first, then reserved builtins, then
 // atoms / data), the shape hash covers the form's tree (kinds, symbols, structure; not number values),
 // and the cost hint is the first argument when it is an integer literal (e.g. n of (fib n)), so forms
@@ -73,7 +73,9 @@ __global__ void culi_classify_kernel(const uint8_t* __restrict__ tag, const uint
       }
       shape = shape_hash(tag, word, r);
     }
-    keys[f] = ((unsigned long long)cls << 48) | ((unsigned long long)shape << 16) | (0xffffu - hint);
+    // 48 significant bits (6 radix passes): class 16 | shape 16 | inverted hint 16
+    keys[f] = ((unsigned long long)cls << 32) | ((unsigned long long)((shape ^ (shape >> 16)) & 0xffffu) << 16) |
+              (0xffffu - hint);
     perm[f] = f;
   }
 }
@@ -99,7 +101,7 @@ cudaError_t launch_dispatch(cudaStream_t s, const DevHeap& H, const uint32_t* ro
   cudaError_t e = cudaGetLastError();
   if (e != cudaSuccess) return e;
   size_t tb = temp_bytes;
-  e = cub::DeviceRadixSort::SortPairs(temp, tb, k0, k1, perm, perm_alt, (int)nforms, 0, 64, s);
+  e = cub::DeviceRadixSort::SortPairs(temp, tb, k0, k1, perm, perm_alt, (int)nforms, 0, 48, s);
   *perm_out = perm_alt;
   return e;
 }
