@@ -31,17 +31,22 @@ from paper_conf_cluster_subdbn18_b200 import workloads as W  # noqa: E402
 L2_FLUSH_BYTES = 512 << 20          # > 126 MB L2: flushed between timed iterations
 PEAKS_PATH = os.path.join(ROOT, "MEASURED_PEAKS.json")
 WORKLOADS = {
+    "C0": lambda n_rank, rank: W.c0(4096),
     "C1": lambda n_rank, rank: W.c1(1024 * n_rank),
     "C2": lambda n_rank, rank: W.c2(65536 * n_rank),
     "C3": lambda n_rank, rank: W.c3(1 << 20),
     "C4": lambda n_rank, rank: W.c4(262144 * n_rank),
     "C5": lambda n_rank, rank: W.c5(16777216),
 }
-SCALING = {"C1": "weak", "C2": "weak", "C3": "replicas", "C4": "weak", "C5": "strong"}
+SCALING = {"C0": "replicas", "C1": "weak", "C2": "weak", "C3": "replicas", "C4": "weak", "C5": "strong"}
 
 
 def bench_config(workload: str, world: int) -> dict:
     """The `config` object shared by the culi arm and the reference (oracle) arm."""
+    if workload == "C0":
+        return {"workload": "C0 (paper-shaped context, PAPER L703 Fig.15): (||| 4096 fib (5 ... 5)), "
+                            "units = element applications", "parallelism": "dp%d" % world,
+                "l2": "flushed between timed steps (512 MB write)"}
     idx = {"C1": 0, "C2": 1, "C3": 2, "C4": 3, "C5": 4}[workload]
     what = {"C1": "1,024 integer arithmetic forms", "C2": "65,536 (fib n) forms, n in 15..22",
             "C3": "(||| 1048576 f xs), closure + let + float", "C4": "262,144 macro forms",
@@ -139,7 +144,7 @@ def run_oracle(wl: W.Workload, max_forms: int, threads: int):
     return sample, desc, r
 
 
-ORACLE_SAMPLE = {"C1": 1024, "C2": 4096, "C3": 1 << 20, "C4": 262144, "C5": 262144}
+ORACLE_SAMPLE = {"C0": 4096, "C1": 1024, "C2": 4096, "C3": 1 << 20, "C4": 262144, "C5": 262144}
 
 
 def reference_arm(args):
@@ -381,7 +386,7 @@ def culi_arm(args):
     peak_inst = 148 * 4 * sm_mhz * 1e6 / 1e9          # G warp-instructions / s
     inst = prof.get("warp_inst_per_launch") if prof else None
     ach = inst / eval_s / 1e9 if inst else None
-    alg_bytes = {"C3": 36.0 * wl.units,                # per element: read cons + float, write cons + box
+    alg_bytes = {"C3": 36.0 * wl.units, "C0": 36.0 * wl.units,                # per element: read cons + float, write cons + box
                  "C2": 52.0 * len(shard_idx), "C1": 190.0 * len(shard_idx),
                  "C4": 120.0 * len(shard_idx), "C5": 120.0 * len(shard_idx)}.get(args.workload, 0.0)
     hbm_ach = alg_bytes / eval_s / 1e9
