@@ -33,4 +33,17 @@ for flags in (0, culi.CULI_F_NO_GC):
     r = c3.eval_text(text)
     print(len(r), r.totals(), c3.heap_usage())
     c3.close()
+# setq (mutable mode, R7) and CUDA-graph replay on a non-default stream
+import torch  # noqa: E402
+st = torch.cuda.Stream()
+c4 = culi.Context(slots=148 * 128, heap_nodes=1 << 22, vstack_entries=1024, stream=st.cuda_stream)
+c4.define("(define make-counter (lambda () (let ((n 0)) (lambda () (setq n (+ n 1))))))\n(define g 1)\n(setq g 2)")
+r = c4.eval_batch("(let ((c (make-counter))) (c) (c))\n(let ((acc 0)) (||| 3 (lambda (x) (setq acc (+ acc x))) '(1 2 3)) acc)\n(setq g 5)")
+print(r.printed())
+h = c4.upload(forms)
+for _ in range(3):
+    c4.eval_uploaded(h)
+print(c4.fetch_results(h).totals())
+c4.release(h)
+c4.close()
 print("done")
