@@ -1146,50 +1146,9 @@ HEAD:
       }
     }
   }
-  if (__builtin_expect(v.t == K_MACRO, 0)) {                    // c.4 MACRO branch (c.13 #13)
-    uint64_t mw = nword(C, (uint32_t)v.w);
-    uint32_t menv = hi32(mw);
-    uint64_t cw = nword(C, lo32(mw));
-    uint32_t ps = lo32(cw), body = hi32(cw);
-    uint32_t hdr = vtop, n = 0;
-    a = cur;
-    while (ps != 0 && a != 0) {                                 // bind params to UNevaluated forms
-      uint64_t pw = nword(C, ps), aw2 = nword(C, a);
-      if (__builtin_expect(!!(hdr + 1 + n >= vcap), 0)) FAIL(E_OOM);
-      *VS(C, hdr + 1 + n) = vpack(unbox(C, lo32(aw2)), (uint32_t)nword(C, lo32(pw)));
-      ++n;
-      ps = hi32(pw);
-      a = hi32(aw2);
-    }
-    if (__builtin_expect(!!(ps != 0 || a != 0), 0)) FAIL(E_ARITY);
-    if (__builtin_expect(!!(n >= 0x8000u), 0)) FAIL(E_OOM);
-    *VS(C, hdr) = make_uint4(menv, 0, n, K_FRAME);
-    KPUSH(KF_MACRO, 0, env, hdr, d, 0);
-    env = stack_env(hdr, n);
-    if (C.A->mut) MUT_FRAME();
-    vtop = hdr + 1 + n;
-    cur = body;
-    goto BODY;
-  }
+  if (__builtin_expect(v.t == K_MACRO, 0)) goto MACRO_CALL;    // c.4 MACRO branch (code below RET)
   // data list (L443-444) or (list ...): elements stream into a preallocated contiguous spine (c.14)
-  if ((v.t != K_BUILTIN && v.t != K_CLOSURE) || (v.t == K_BUILTIN && v.w == BI_LIST)) {
-    bool data = v.t != K_BUILTIN;
-    uint32_t n = data ? 1 : 0;
-    for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
-    if (n == 0) { v = mkv(K_NIL, 0); goto RET; }
-    uint32_t s;
-    if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &s)), 0)) FAIL(E_OOM);
-    if (data) {
-      uint32_t ca = box_into(H, v, s + n);
-      H.tag[s] = K_CONS | TAG_PROPER;
-      H.word[s] = pack2(ca, n > 1 ? s + 1 : 0);
-    }
-    if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
-    base = vtop;
-    *VS(C, base) = make_uint4(s, n, 0, 0);                      // {spine, n}
-    cnt = data ? 1 : 0;                                         // next element index
-    goto DATA_LOOP;
-  }
+  if ((v.t != K_BUILTIN && v.t != K_CLOSURE) || (v.t == K_BUILTIN && v.w == BI_LIST)) goto DATA_START;
   // BUILTIN or CLOSURE: evaluate the args left to right at depth d+1 onto the V-stack
   if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
   base = vtop;
@@ -1259,91 +1218,7 @@ APPLY: {                                                        // apply vs[base
     goto BODY;
   }
   if (__builtin_expect(!!(h.t != K_BUILTIN), 0)) FAIL(E_SYNTAX);
-  if ((uint32_t)h.w == BI_PAR) {                                // (||| n f l1 ... lm), c.7
-    uint32_t n;
-    if (fanout && sp == 0 && d == 1 && cnt >= 3 && cnt - 2 <= FANOUT_MAXM) {
-      // top-level ||| form: its arguments are evaluated; hand the elements to the fan-out kernel
-      // (SURVEY §8(a)6).  Errors decidable now are raised exactly; list lengths are verified by the
-      // element kernel (a short or non-contiguous list sends the form to sequential re-evaluation).
-      uint8_t e = par_check_light(C, base, cnt, &n);
-      if (__builtin_expect(!!(e), 0)) FAIL(e);
-      if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
-      uint32_t slot = atomicAdd(C.A->npend, 1u);
-      if (slot < C.A->maxdesc) {
-        uint32_t spine;
-        if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
-        FanDesc* D = C.A->desc + slot;
-        V f = arg(C, base, 1);
-        D->form = form;
-        D->n = n;
-        D->m = cnt - 2;
-        D->kind = FAN_PAR;
-        D->nelem = n;
-        D->spine = spine;
-        D->ftag = f.t;
-        D->depth = d;
-        D->fword = f.w;
-        D->steps0 = steps;
-        D->top = atomicAdd(H.top, 0ull);
-        for (uint32_t j = 0; j < cnt - 2; ++j) D->heads[j] = (uint32_t)arg(C, base, 2 + j).w;
-        D->total = 0;
-        D->bad = 0;
-        D->nonflat = 0;
-        err = E_PENDING;
-        goto done;
-      }
-    }
-    if (NEST && !APPLY && C.A->nest && cnt >= 3 && cnt - 2 <= FANOUT_MAXM) {
-      // nested ||| (§8(f)1): suspend; the elements are applied by any threads, then we resume at RET
-      uint8_t e = par_check_light(C, base, cnt, &n);
-      if (__builtin_expect(!!(e), 0)) FAIL(e);
-      if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
-      if (n >= NEST_MIN) {
-        uint32_t slot = atomicAdd(C.A->nnest, 1u);
-        if (slot < C.A->maxnest) {
-          uint32_t spine;
-          if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
-          NestDesc* D = C.A->ndesc + slot;
-          V f = arg(C, base, 1);
-          D->form = form;
-          D->n = n;
-          D->m = cnt - 2;
-          D->spine = spine;
-          D->ftag = f.t;
-          D->depth = d;
-          D->fword = f.w;
-          D->steps0 = steps;
-          D->top = atomicAdd(H.top, 0ull);
-          for (uint32_t j = 0; j < cnt - 2; ++j) D->heads[j] = (uint32_t)arg(C, base, 2 + j).w;
-          D->sp = sp;
-          D->vtop = base;
-          D->total = 0;
-          D->bad = 0;
-          D->done = 0;
-          D->next = 0;
-          __threadfence();
-          atomicExch(&D->ready, 1u);                            // publish: elements may be claimed
-          if (kdirty) *KS(C, sp - 1) = ktop;                    // the resume reloads the top frame
-          v = mkv(K_CONS, spine);
-          aux = slot;
-          err = E_SUSPEND;
-          goto done;
-        }
-      }
-    }
-    uint8_t e = par_check(C, base, cnt, &n);
-    if (__builtin_expect(!!(e), 0)) FAIL(e);
-    if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
-    uint32_t m = cnt - 2, spine;
-    if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
-    // state: vs[base] = {spine, n}, vs[base+1] = f, vs[base+2+j] = list cursor j
-    V f = arg(C, base, 1);
-    for (uint32_t j = 0; j < m; ++j) *VS(C, base + 2 + j) = *VS(C, base + 3 + j);
-    *VS(C, base + 1) = vpack(f, 0);
-    *VS(C, base) = make_uint4(spine, n, 0, 0);
-    KPUSH(KF_PAR, 0, 0, base, d, m);
-    goto PAR_NEXT;
-  }
+  if ((uint32_t)h.w == BI_PAR) goto PAR_APPLY;                 // (||| n f l1 ... lm), c.7 (below RET)
   {
     uint8_t e = apply_builtin(C, (uint32_t)h.w, base, cnt, vtop, &v);
     if (__builtin_expect(!!(e), 0)) FAIL(e);
@@ -1377,88 +1252,6 @@ IF_BRANCH:
   if (hi32(w0) != 0) { x = car_of(C, hi32(w0)); d = d + 1; goto EVAL_NODE; }
   v = mkv(K_NIL, 0);
   goto RET;
-
-  // ======================================================== let: binding `cur` next (parallel let)
-LET_LOOP:
-  while (cur != 0) {
-    w0 = nword(C, cur);
-    uint64_t bw = nword(C, lo32(w0));
-    uint32_t e = car_of(C, hi32(bw));
-    ldnode(C, e, at, aw);
-    STEP(d + 1);
-    V lv;
-    if ((at & KIND_MASK) == K_CONS) {
-      int leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &lv, &err);
-      if (__builtin_expect(leaf == 2, 0)) goto done;
-      if (leaf == 0) {
-        vtop = base + 1 + cnt;
-        KPUSH(KF_LET, cur, env, base, d, cnt);
-        x = e; t = at; w = aw; d = d + 1;
-        goto EVAL_CONS;
-      }
-    } else {
-      lv = ATOMVAL(e, at, aw);
-    }
-    if (__builtin_expect(!!(base + 1 + cnt >= vcap || cnt >= 0x7fffu), 0)) FAIL(E_OOM);
-    *VS(C, base + 1 + cnt) = vpack(lv, (uint32_t)nword(C, lo32(bw)));
-    ++cnt;
-    cur = hi32(w0);
-  }
-  cur = VS(C, base)->x;                                         // body list stored in the header
-  *VS(C, base) = make_uint4(env, 0, cnt, K_FRAME);
-  env = stack_env(base, cnt);
-  if (C.A->mut) MUT_FRAME();
-  vtop = base + 1 + cnt;
-  goto BODY;
-
-  // ======================================================== data list / list: element `cnt` next
-DATA_LOOP: {
-  uint4 st = *VS(C, base);
-  uint32_t s = st.x, n = st.y;
-  while (cur != 0) {
-    w0 = nword(C, cur);
-    a = lo32(w0);
-    nxt = hi32(w0);
-    ldnode(C, a, at, aw);
-    STEP(d + 1);
-    if ((at & KIND_MASK) == K_CONS) {
-      VS(C, base)->z = cnt;
-      vtop = base + 1;
-      KPUSH(KF_DATA, nxt, env, base, d, 0);
-      x = a; t = at; w = aw; d = d + 1;
-      goto EVAL_CONS;
-    }
-    v = ATOMVAL(a, at, aw);
-    uint32_t ca = box_into(H, v, s + n + cnt);
-    H.tag[s + cnt] = K_CONS | TAG_PROPER;
-    H.word[s + cnt] = pack2(ca, cnt + 1 < n ? s + cnt + 1 : 0);
-    ++cnt;
-    cur = nxt;
-  }
-  vtop = base;
-  v = mkv(K_CONS, s);
-  goto RET;
-}
-
-  // ======================================================== ||| : start element i (frame in ktop)
-PAR_NEXT: {
-  uint32_t m = kcount(ktop.w), pb = ktop.z;
-  V f = vunpack(*VS(C, pb + 1));
-  base = pb + 2 + m;
-  if (__builtin_expect(!!(base + 1 + m >= vcap), 0)) FAIL(E_OOM);
-  hv = vpack(f, 0);
-  *VS(C, base) = hv;
-  for (uint32_t j = 0; j < m; ++j) {
-    uint4* cj = VS(C, pb + 2 + j);
-    uint64_t wj = nword(C, cj->x);
-    *VS(C, base + 1 + j) = vpack(unbox(C, lo32(wj)), 0);
-    cj->x = hi32(wj);
-  }
-  cnt = m;
-  vtop = base + 1 + m;
-  d = kdepth(ktop.w);
-  goto APPLY;
-}
 
   // ======================================================== return v to the top continuation
 RET:
@@ -1567,6 +1360,224 @@ RET:
     default:
       FAIL(E_SYNTAX);
   }
+
+  // ---- cold sections, placed after the hot loop so that its instructions stay contiguous ----
+  // ======================================================== macro call (c.4 MACRO branch, c.13 #13)
+MACRO_CALL: {
+    uint64_t mw = nword(C, (uint32_t)v.w);
+    uint32_t menv = hi32(mw);
+    uint64_t cw = nword(C, lo32(mw));
+    uint32_t ps = lo32(cw), body = hi32(cw);
+    uint32_t hdr = vtop, n = 0;
+    a = cur;
+    while (ps != 0 && a != 0) {                                 // bind params to UNevaluated forms
+      uint64_t pw = nword(C, ps), aw2 = nword(C, a);
+      if (__builtin_expect(!!(hdr + 1 + n >= vcap), 0)) FAIL(E_OOM);
+      *VS(C, hdr + 1 + n) = vpack(unbox(C, lo32(aw2)), (uint32_t)nword(C, lo32(pw)));
+      ++n;
+      ps = hi32(pw);
+      a = hi32(aw2);
+    }
+    if (__builtin_expect(!!(ps != 0 || a != 0), 0)) FAIL(E_ARITY);
+    if (__builtin_expect(!!(n >= 0x8000u), 0)) FAIL(E_OOM);
+    *VS(C, hdr) = make_uint4(menv, 0, n, K_FRAME);
+    KPUSH(KF_MACRO, 0, env, hdr, d, 0);
+    env = stack_env(hdr, n);
+    if (C.A->mut) MUT_FRAME();
+    vtop = hdr + 1 + n;
+    cur = body;
+    goto BODY;
+}
+
+  // ======================================================== data list / (list ...): set up the spine
+DATA_START: {
+    bool data = v.t != K_BUILTIN;
+    uint32_t n = data ? 1 : 0;
+    for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
+    if (n == 0) { v = mkv(K_NIL, 0); goto RET; }
+    uint32_t s;
+    if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &s)), 0)) FAIL(E_OOM);
+    if (data) {
+      uint32_t ca = box_into(H, v, s + n);
+      H.tag[s] = K_CONS | TAG_PROPER;
+      H.word[s] = pack2(ca, n > 1 ? s + 1 : 0);
+    }
+    if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
+    base = vtop;
+    *VS(C, base) = make_uint4(s, n, 0, 0);                      // {spine, n}
+    cnt = data ? 1 : 0;                                         // next element index
+    goto DATA_LOOP;
+}
+
+  // ======================================================== (||| n f l1 ... lm), c.7
+PAR_APPLY: {
+    uint32_t n;
+    if (fanout && sp == 0 && d == 1 && cnt >= 3 && cnt - 2 <= FANOUT_MAXM) {
+      // top-level ||| form: its arguments are evaluated; hand the elements to the fan-out kernel
+      // (SURVEY §8(a)6).  Errors decidable now are raised exactly; list lengths are verified by the
+      // element kernel (a short or non-contiguous list sends the form to sequential re-evaluation).
+      uint8_t e = par_check_light(C, base, cnt, &n);
+      if (__builtin_expect(!!(e), 0)) FAIL(e);
+      if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
+      uint32_t slot = atomicAdd(C.A->npend, 1u);
+      if (slot < C.A->maxdesc) {
+        uint32_t spine;
+        if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
+        FanDesc* D = C.A->desc + slot;
+        V f = arg(C, base, 1);
+        D->form = form;
+        D->n = n;
+        D->m = cnt - 2;
+        D->kind = FAN_PAR;
+        D->nelem = n;
+        D->spine = spine;
+        D->ftag = f.t;
+        D->depth = d;
+        D->fword = f.w;
+        D->steps0 = steps;
+        D->top = atomicAdd(H.top, 0ull);
+        for (uint32_t j = 0; j < cnt - 2; ++j) D->heads[j] = (uint32_t)arg(C, base, 2 + j).w;
+        D->total = 0;
+        D->bad = 0;
+        D->nonflat = 0;
+        err = E_PENDING;
+        goto done;
+      }
+    }
+    if (NEST && !APPLY && C.A->nest && cnt >= 3 && cnt - 2 <= FANOUT_MAXM) {
+      // nested ||| (§8(f)1): suspend; the elements are applied by any threads, then we resume at RET
+      uint8_t e = par_check_light(C, base, cnt, &n);
+      if (__builtin_expect(!!(e), 0)) FAIL(e);
+      if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
+      if (n >= NEST_MIN) {
+        uint32_t slot = atomicAdd(C.A->nnest, 1u);
+        if (slot < C.A->maxnest) {
+          uint32_t spine;
+          if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
+          NestDesc* D = C.A->ndesc + slot;
+          V f = arg(C, base, 1);
+          D->form = form;
+          D->n = n;
+          D->m = cnt - 2;
+          D->spine = spine;
+          D->ftag = f.t;
+          D->depth = d;
+          D->fword = f.w;
+          D->steps0 = steps;
+          D->top = atomicAdd(H.top, 0ull);
+          for (uint32_t j = 0; j < cnt - 2; ++j) D->heads[j] = (uint32_t)arg(C, base, 2 + j).w;
+          D->sp = sp;
+          D->vtop = base;
+          D->total = 0;
+          D->bad = 0;
+          D->done = 0;
+          D->next = 0;
+          __threadfence();
+          atomicExch(&D->ready, 1u);                            // publish: elements may be claimed
+          if (kdirty) *KS(C, sp - 1) = ktop;                    // the resume reloads the top frame
+          v = mkv(K_CONS, spine);
+          aux = slot;
+          err = E_SUSPEND;
+          goto done;
+        }
+      }
+    }
+    uint8_t e = par_check(C, base, cnt, &n);
+    if (__builtin_expect(!!(e), 0)) FAIL(e);
+    if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
+    uint32_t m = cnt - 2, spine;
+    if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
+    // state: vs[base] = {spine, n}, vs[base+1] = f, vs[base+2+j] = list cursor j
+    V f = arg(C, base, 1);
+    for (uint32_t j = 0; j < m; ++j) *VS(C, base + 2 + j) = *VS(C, base + 3 + j);
+    *VS(C, base + 1) = vpack(f, 0);
+    *VS(C, base) = make_uint4(spine, n, 0, 0);
+    KPUSH(KF_PAR, 0, 0, base, d, m);
+    goto PAR_NEXT;
+}
+
+  // ======================================================== let: binding `cur` next (parallel let)
+LET_LOOP:
+  while (cur != 0) {
+    w0 = nword(C, cur);
+    uint64_t bw = nword(C, lo32(w0));
+    uint32_t e = car_of(C, hi32(bw));
+    ldnode(C, e, at, aw);
+    STEP(d + 1);
+    V lv;
+    if ((at & KIND_MASK) == K_CONS) {
+      int leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &lv, &err);
+      if (__builtin_expect(leaf == 2, 0)) goto done;
+      if (leaf == 0) {
+        vtop = base + 1 + cnt;
+        KPUSH(KF_LET, cur, env, base, d, cnt);
+        x = e; t = at; w = aw; d = d + 1;
+        goto EVAL_CONS;
+      }
+    } else {
+      lv = ATOMVAL(e, at, aw);
+    }
+    if (__builtin_expect(!!(base + 1 + cnt >= vcap || cnt >= 0x7fffu), 0)) FAIL(E_OOM);
+    *VS(C, base + 1 + cnt) = vpack(lv, (uint32_t)nword(C, lo32(bw)));
+    ++cnt;
+    cur = hi32(w0);
+  }
+  cur = VS(C, base)->x;                                         // body list stored in the header
+  *VS(C, base) = make_uint4(env, 0, cnt, K_FRAME);
+  env = stack_env(base, cnt);
+  if (C.A->mut) MUT_FRAME();
+  vtop = base + 1 + cnt;
+  goto BODY;
+
+  // ======================================================== data list / list: element `cnt` next
+DATA_LOOP: {
+  uint4 st = *VS(C, base);
+  uint32_t s = st.x, n = st.y;
+  while (cur != 0) {
+    w0 = nword(C, cur);
+    a = lo32(w0);
+    nxt = hi32(w0);
+    ldnode(C, a, at, aw);
+    STEP(d + 1);
+    if ((at & KIND_MASK) == K_CONS) {
+      VS(C, base)->z = cnt;
+      vtop = base + 1;
+      KPUSH(KF_DATA, nxt, env, base, d, 0);
+      x = a; t = at; w = aw; d = d + 1;
+      goto EVAL_CONS;
+    }
+    v = ATOMVAL(a, at, aw);
+    uint32_t ca = box_into(H, v, s + n + cnt);
+    H.tag[s + cnt] = K_CONS | TAG_PROPER;
+    H.word[s + cnt] = pack2(ca, cnt + 1 < n ? s + cnt + 1 : 0);
+    ++cnt;
+    cur = nxt;
+  }
+  vtop = base;
+  v = mkv(K_CONS, s);
+  goto RET;
+}
+
+  // ======================================================== ||| : start element i (frame in ktop)
+PAR_NEXT: {
+  uint32_t m = kcount(ktop.w), pb = ktop.z;
+  V f = vunpack(*VS(C, pb + 1));
+  base = pb + 2 + m;
+  if (__builtin_expect(!!(base + 1 + m >= vcap), 0)) FAIL(E_OOM);
+  hv = vpack(f, 0);
+  *VS(C, base) = hv;
+  for (uint32_t j = 0; j < m; ++j) {
+    uint4* cj = VS(C, pb + 2 + j);
+    uint64_t wj = nword(C, cj->x);
+    *VS(C, base + 1 + j) = vpack(unbox(C, lo32(wj)), 0);
+    cj->x = hi32(wj);
+  }
+  cnt = m;
+  vtop = base + 1 + m;
+  d = kdepth(ktop.w);
+  goto APPLY;
+}
+
 
 done:
 #undef FAIL
