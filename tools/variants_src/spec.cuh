@@ -1075,76 +1075,27 @@ HEAD:
     goto RET;
   }
   if (v.t == K_SPECIAL) {
-    uint32_t op = (uint32_t)v.w;
-    if (op == SP_DEFINE || op == SP_DEFUN || op == SP_DEFMACRO) {
-      if (__builtin_expect(!!(!C.A->define_mode), 0)) FAIL(E_DEFINE_IN_BATCH);
-    }
-    if (__builtin_expect(!!(!(t & TAG_VALID) && !special_syntax_ok(C, op, cur)), 0)) FAIL(E_SYNTAX);
-    switch (op) {
-      case SP_IF: {
-        w0 = nword(C, cur);
-        uint32_t c1 = hi32(w0);
-        a = lo32(w0);
-        ldnode(C, a, at, aw);
-        STEP(d + 1);
-        if ((at & KIND_MASK) == K_CONS) {
-          int leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &v, &err);
-          if (__builtin_expect(leaf == 2, 0)) goto done;
-          if (leaf == 0) {
-            KPUSH(KF_IF, c1, env, vtop, d, 0);
-            x = a; t = at; w = aw; d = d + 1;
-            goto EVAL_CONS;
-          }
-        } else {
-          v = ATOMVAL(a, at, aw);
+    if ((uint32_t)v.w == SP_IF && (t & TAG_VALID)) {
+      w0 = nword(C, cur);
+      uint32_t c1 = hi32(w0);
+      a = lo32(w0);
+      ldnode(C, a, at, aw);
+      STEP(d + 1);
+      if ((at & KIND_MASK) == K_CONS) {
+        int leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &v, &err);
+        if (__builtin_expect(leaf == 2, 0)) goto done;
+        if (leaf == 0) {
+          KPUSH(KF_IF, c1, env, vtop, d, 0);
+          x = a; t = at; w = aw; d = d + 1;
+          goto EVAL_CONS;
         }
-        cur = c1;
-        goto IF_BRANCH;
+      } else {
+        v = ATOMVAL(a, at, aw);
       }
-      case SP_QUOTE:
-        v = unbox(C, car_of(C, cur));
-        goto RET;
-      case SP_PROGN:
-        goto BODY;
-      case SP_LAMBDA:
-        if (__builtin_expect(!!(!make_closure(C, K_CLOSURE, cur, env, &v)), 0)) FAIL(E_OOM);
-        goto RET;
-      case SP_LET: {
-        w0 = nword(C, cur);
-        uint32_t bl = lo32(w0), body = hi32(w0);
-        if (bl == 0) { cur = body; goto BODY; }
-        if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
-        base = vtop;
-        *VS(C, base) = make_uint4(body, 0, 0, K_FRAME);         // header (holds the body for now)
-        cnt = 0;
-        cur = bl;
-        goto LET_LOOP;
-      }
-      case SP_SETQ: {                                           // R7: the value first, then the binding
-        w0 = nword(C, cur);
-        KPUSH(KF_SETQ, (uint32_t)nword(C, lo32(w0)), env, vtop, d, 0);
-        x = car_of(C, hi32(w0));
-        d = d + 1;
-        goto EVAL_NODE;
-      }
-      case SP_DEFINE: {
-        w0 = nword(C, cur);
-        KPUSH(KF_DEFINE, (uint32_t)nword(C, lo32(w0)), env, vtop, d, 0);
-        x = car_of(C, hi32(w0));
-        d = d + 1;
-        goto EVAL_NODE;
-      }
-      default: {                                                // defun / defmacro
-        w0 = nword(C, cur);
-        uint32_t s = (uint32_t)nword(C, lo32(w0));
-        V clo;
-        if (__builtin_expect(!!(!make_closure(C, op == SP_DEFUN ? K_CLOSURE : K_MACRO, hi32(w0), env, &clo)), 0)) FAIL(E_OOM);
-        H.gtag[s] = (uint8_t)clo.t;
-        H.gword[s] = clo.w;
-        v = mkv(K_SYM, s);
-        goto RET;
-      }
+      cur = c1;
+      goto IF_BRANCH;
     }
+    goto SPECIALS;
   }
   if (__builtin_expect(v.t == K_MACRO, 0)) goto MACRO_CALL;    // c.4 MACRO branch (code below RET)
   // data list (L443-444) or (list ...): elements stream into a preallocated contiguous spine (c.14)
@@ -1310,20 +1261,7 @@ RET:
       cur = k.x; env = k.y; vtop = k.z; d = kd;
       t = 0;                                                    // a computed head: no TAG_VALID
       goto HEAD;
-    case KF_LET: goto RET_LET;
-    case KF_SETQ: goto RET_SETQ;
-    case KF_DEFINE: goto RET_DEFINE;
-    case KF_MACRO: goto RET_MACRO;
-    case KF_PAR: goto RET_PAR;
-    case KF_DATA: goto RET_DATA;
-    default:
-      FAIL(E_SYNTAX);
-  }
-
-  // ---- cold sections, placed after the hot loop so that its instructions stay contiguous ----
-  // ======================================================== returns to the rarer continuations
-RET_LET: {
-
+    case KF_LET: {
       base = k.z; cnt = kcount(k.w);
       w0 = nword(C, k.x);
       uint32_t sym = (uint32_t)nword(C, car_of(C, lo32(w0)));
@@ -1332,27 +1270,23 @@ RET_LET: {
       ++cnt;
       cur = hi32(w0); env = k.y; d = kd;
       goto LET_LOOP;
-}
-RET_SETQ: {
-
+    }
+    case KF_SETQ: {
       uint8_t e = setq_store(C, k.x, k.y, v);
       if (__builtin_expect(!!(e), 0)) FAIL(e);
       vtop = k.z;
       goto RET;
-}
-RET_DEFINE: {
+    }
+    case KF_DEFINE:
       H.gtag[k.x] = (uint8_t)v.t;
       H.gword[k.x] = v.w;
       v = mkv(K_SYM, k.x);
       vtop = k.z;
       goto RET;
-}
-RET_MACRO: {
+    case KF_MACRO:                                              // evaluate the expansion
       vtop = k.z; env = k.y; d = kd + 1;
       goto EVAL_VALUE;
-}
-RET_PAR: {
-                                              // element i finished
+    case KF_PAR: {                                              // element i finished
       uint32_t m = kcount(k.w), i = k.x, pb = k.z;
       uint4 st = *VS(C, pb);
       uint32_t spine = st.x, n = st.y;
@@ -1362,9 +1296,8 @@ RET_PAR: {
       if (i + 1 == n) { v = mkv(K_CONS, spine); vtop = pb; goto RET; }
       KPUSH(KF_PAR, i + 1, 0, pb, kd, m);
       goto PAR_NEXT;
-}
-RET_DATA: {
-
+    }
+    case KF_DATA: {
       base = k.z;
       uint4 st = *VS(C, base);
       uint32_t s = st.x, n = st.y, i = st.z;
@@ -1374,6 +1307,83 @@ RET_DATA: {
       cnt = i + 1;
       cur = k.x; env = k.y; d = kd;
       goto DATA_LOOP;
+    }
+    default:
+      FAIL(E_SYNTAX);
+  }
+
+  // ---- cold sections, placed after the hot loop so that its instructions stay contiguous ----
+SPECIALS: {
+    uint32_t op = (uint32_t)v.w;
+    if (op == SP_DEFINE || op == SP_DEFUN || op == SP_DEFMACRO) {
+      if (__builtin_expect(!!(!C.A->define_mode), 0)) FAIL(E_DEFINE_IN_BATCH);
+    }
+    if (__builtin_expect(!!(!(t & TAG_VALID) && !special_syntax_ok(C, op, cur)), 0)) FAIL(E_SYNTAX);
+    switch (op) {
+      case SP_IF: {
+        w0 = nword(C, cur);
+        uint32_t c1 = hi32(w0);
+        a = lo32(w0);
+        ldnode(C, a, at, aw);
+        STEP(d + 1);
+        if ((at & KIND_MASK) == K_CONS) {
+          int leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &v, &err);
+          if (__builtin_expect(leaf == 2, 0)) goto done;
+          if (leaf == 0) {
+            KPUSH(KF_IF, c1, env, vtop, d, 0);
+            x = a; t = at; w = aw; d = d + 1;
+            goto EVAL_CONS;
+          }
+        } else {
+          v = ATOMVAL(a, at, aw);
+        }
+        cur = c1;
+        goto IF_BRANCH;
+      }
+      case SP_QUOTE:
+        v = unbox(C, car_of(C, cur));
+        goto RET;
+      case SP_PROGN:
+        goto BODY;
+      case SP_LAMBDA:
+        if (__builtin_expect(!!(!make_closure(C, K_CLOSURE, cur, env, &v)), 0)) FAIL(E_OOM);
+        goto RET;
+      case SP_LET: {
+        w0 = nword(C, cur);
+        uint32_t bl = lo32(w0), body = hi32(w0);
+        if (bl == 0) { cur = body; goto BODY; }
+        if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
+        base = vtop;
+        *VS(C, base) = make_uint4(body, 0, 0, K_FRAME);         // header (holds the body for now)
+        cnt = 0;
+        cur = bl;
+        goto LET_LOOP;
+      }
+      case SP_SETQ: {                                           // R7: the value first, then the binding
+        w0 = nword(C, cur);
+        KPUSH(KF_SETQ, (uint32_t)nword(C, lo32(w0)), env, vtop, d, 0);
+        x = car_of(C, hi32(w0));
+        d = d + 1;
+        goto EVAL_NODE;
+      }
+      case SP_DEFINE: {
+        w0 = nword(C, cur);
+        KPUSH(KF_DEFINE, (uint32_t)nword(C, lo32(w0)), env, vtop, d, 0);
+        x = car_of(C, hi32(w0));
+        d = d + 1;
+        goto EVAL_NODE;
+      }
+      default: {                                                // defun / defmacro
+        w0 = nword(C, cur);
+        uint32_t s = (uint32_t)nword(C, lo32(w0));
+        V clo;
+        if (__builtin_expect(!!(!make_closure(C, op == SP_DEFUN ? K_CLOSURE : K_MACRO, hi32(w0), env, &clo)), 0)) FAIL(E_OOM);
+        H.gtag[s] = (uint8_t)clo.t;
+        H.gword[s] = clo.w;
+        v = mkv(K_SYM, s);
+        goto RET;
+      }
+    }
 }
 
   // ======================================================== macro call (c.4 MACRO branch, c.13 #13)
