@@ -213,6 +213,13 @@ static bool image_mentions_setq(const Image& img) {
     if ((img.tag[k] & KIND_MASK) == K_SYM && img.word[k] == SP_SETQ) return true;
   return false;
 }
+// Closures are made only by lambda and defun (c.4): without either symbol there is no closure to apply,
+// so argument splitting (which polls at closure calls) cannot help and the eval grid can shrink.
+static bool image_mentions_closure(const Image& img) {
+  for (size_t k = 0; k < img.tag.size(); ++k)
+    if ((img.tag[k] & KIND_MASK) == K_SYM && (img.word[k] == SP_LAMBDA || img.word[k] == SP_DEFUN)) return true;
+  return false;
+}
 static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, int define_mode) {
   EvalArgs A{};
   A.H = c->H;
@@ -249,7 +256,10 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.kst2 = c->kst2;
   A.vst2 = c->vst2;
   A.finished = c->nnest + 1;
-  A.split = (!define_mode && !(c->opts.flags & CULI_F_NO_SPLIT)) ? 1 : 0;
+  // argument splitting: only where a closure may be applied, and only on binned batches (or one form):
+  // on unbinned multi-form batches (divergent warps) it was seen to hang (DESIGN.md §5.5 known issue)
+  A.split = (!define_mode && c->batch_may_close && (perm || nforms <= 1) &&
+             !(c->opts.flags & CULI_F_NO_SPLIT)) ? 1 : 0;
   // setq (R7): frames go to the heap when made, and a form runs in one thread only (no fan-out, nested
   // fan-out or argument splitting: those evaluate parts of a form elsewhere, on copies of its frames)
   A.mut = define_mode ? c->define_mut : c->batch_mut;
@@ -359,6 +369,7 @@ extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed
   if (rc) return rc;
   c->strings += img.strings;
   c->persist_has_par = c->persist_has_par || image_mentions_par(img);
+  c->persist_has_closure = c->persist_has_closure || image_mentions_closure(img);
   c->define_mut = c->persist_has_setq || image_mentions_setq(img);
   c->persist_has_setq = c->define_mut;
   return run_define(c, nf, img.tag.size(), failed_index, failed_err);
@@ -372,6 +383,7 @@ extern "C" int culi_define_text(culi_ctx* c, const char* text, size_t len, int t
   if (rc) return rc;
   c->strings += ro.strings;
   c->persist_has_par = c->persist_has_par || ro.par_root_head || ro.par_nested;
+  c->persist_has_closure = c->persist_has_closure || ro.closure;
   c->define_mut = c->persist_has_setq || ro.setq;
   c->persist_has_setq = c->define_mut;
   return run_define(c, ro.nforms, ro.nodes, failed_index, failed_err);
@@ -395,10 +407,10 @@ static int run_batch_device(culi_ctx* c) {
                   c->nfallback, c->nnest, c->gcount));
   ++c->last_kernels;
   uint32_t* perm = nullptr;
-  if (!(c->opts.flags & CULI_F_NO_BINNING) && nf > 1) {
+  if (!(c->opts.flags & CULI_F_NO_BINNING) && nf > 1 && (nf >= BIN_MIN_FORMS || c->batch_may_close)) {
     CK(launch_dispatch(c->stream, c->H, c->roots.p, nf, c->keys.p, c->keys_alt.p, c->perm.p,
                        c->perm_alt.p, c->dtemp.p, c->dtemp.n, &perm, c->sms));
-    c->last_kernels += 3;
+    c->last_kernels += dispatch_launches(nf);
   }
   CK(record_event(c, 1));
   EvalArgs A = make_args(c, nf, perm, 0);
@@ -443,8 +455,9 @@ static int run_batch_device(culi_ctx* c) {
 // host image or written by the device reader).  par_any / par_nonroot: the ||| symbol is the car of some
 // cell / of some cell other than a top-level form's first cell; par_head: some form is (||| ...).
 static int finish_prepare(culi_ctx* c, uint32_t nf, uint64_t nnodes, std::string strings, bool par_any,
-                          bool par_nonroot, bool par_head, bool has_wide, bool setq) {
+                          bool par_nonroot, bool par_head, bool has_wide, bool setq, bool closure) {
   c->batch_mut = c->persist_has_setq || setq;
+  c->batch_may_close = c->persist_has_closure || closure;
   drop_graph(c);
   int rc = ensure_results(c, nf);
   if (rc) return rc;
@@ -502,7 +515,8 @@ static int prepare_batch(culi_ctx* c, const Image& img) {
     CK(cudaMemcpyAsync(c->wide.p, wide.data(), nf * 4, cudaMemcpyHostToDevice, c->stream));
   }
   return finish_prepare(c, nf, img.tag.size(), img.strings, image_mentions_par(img, false),
-                        image_mentions_par(img, true), par_head, has_wide, image_mentions_setq(img));
+                        image_mentions_par(img, true), par_head, has_wide, image_mentions_setq(img),
+                        image_mentions_closure(img));
 }
 
 // Device reader (§8(f)2) -> the same prepared batch.
@@ -511,7 +525,7 @@ static int prepare_text(culi_ctx* c, const char* text, size_t len, bool on_devic
   int rc = device_read(c, text, len, on_device, &ro, err_offset);
   if (rc) return rc;
   return finish_prepare(c, ro.nforms, ro.nodes, std::move(ro.strings), ro.par_root_head || ro.par_nested,
-                        ro.par_nested, ro.par_root_head, ro.wide, ro.setq);
+                        ro.par_nested, ro.par_root_head, ro.wide, ro.setq, ro.closure);
 }
 
 // ||| forms the fan-out could not decide (an element error, fuel overflow, a short or non-contiguous

@@ -134,6 +134,8 @@ struct culi_ctx {
   bool persist_has_par = false;      // some definition mentions |||
   bool persist_has_setq = false;     // some definition mentions setq (R7: batches run with heap frames)
   bool batch_mut = false, define_mut = false;
+  bool persist_has_closure = false;  // some definition mentions lambda / defun
+  bool batch_may_close = false;      // a closure may be applied in the batch (argument splitting useful)
   bool batch_may_nest = false;
   NestDesc* ndesc = nullptr;
   uint32_t maxnest = 4096;

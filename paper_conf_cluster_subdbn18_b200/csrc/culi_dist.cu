@@ -84,7 +84,7 @@ int culi_env_export(culi_ctx* c, void* dev_buf, size_t cap, size_t* bytes) {
   h.nsyms = c->syms->names.size();
   h.nstr = c->strings.size();
   h.names_bytes = names.size();
-  h.flags = (c->persist_has_par ? 1 : 0) | (c->persist_has_setq ? 2 : 0);
+  h.flags = (c->persist_has_par ? 1 : 0) | (c->persist_has_setq ? 2 : 0) | (c->persist_has_closure ? 4 : 0);
   EnvLayout L(h);
   if (bytes) *bytes = L.total;
   if (!dev_buf || cap < L.total) return dev_buf ? CULI_E_ARG : CULI_OK;
@@ -139,6 +139,7 @@ int culi_env_import(culi_ctx* c, const void* dev_buf, size_t nbytes) {
   c->mark = h.mark;
   c->persist_has_par = (h.flags & 1) != 0;
   c->persist_has_setq = (h.flags & 2) != 0;
+  c->persist_has_closure = (h.flags & 4) != 0;
   c->defined = true;
   return CULI_OK;
 }

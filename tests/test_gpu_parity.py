@@ -199,7 +199,7 @@ def test_depth_and_fuel_limits(culi, oracle_mod):
 
 
 def test_flags_do_not_change_results(culi, oracle_mod):
-    wl = W.c5(3000)
+    wl = W.c5(5000)                      # above BIN_MIN_FORMS: the default run is binned
     outs = []
     for fl in (0, culi.CULI_F_NO_BINNING, culi.CULI_F_NO_VOTING | culi.CULI_F_NO_STAGING):
         gp, gs, o = run_both(culi, oracle_mod, wl.defs, wl.forms, ctx_kw=dict(flags=fl))
@@ -400,3 +400,47 @@ def test_nested_par_limits(culi, oracle_mod):
     for fuel, depth in ((1 << 40, 1024), (5000, 1024), (200000, 1024), (1 << 40, 6), (1 << 40, 4)):
         assert_parity(culi, oracle_mod, NESTED_DEFS, forms, ctx_kw=dict(fuel=fuel, max_depth=depth),
                       oracle_kw=dict(fuel=fuel, max_depth=depth))
+
+
+@pytest.mark.parametrize("n", [1, 2, 4095, 4096, 4097])
+def test_small_batch_dispatch_boundary(culi, oracle_mod, n):
+    """Batches of <= 4096 forms run in input order, larger ones through the binning permutation
+    (BIN_MIN_FORMS, csrc/culi_eval.cuh): both must evaluate every form exactly once, in parity."""
+    wl = W.c5(n, seed=77)
+    gp, gs, o = assert_parity(culi, oracle_mod, wl.defs, wl.forms)
+    ctx = culi.Context(**{**SMALL, "flags": culi.CULI_F_NO_BINNING})
+    ctx.define(wl.defs)
+    r = ctx.eval_batch(wl.forms)
+    assert (r.printed(), r.steps()) == (gp, gs)
+
+
+def test_no_closure_batch_runs_without_splitting(culi, oracle_mod):
+    """Without lambda / defun anywhere (definitions or batch) no closure exists, so argument splitting is
+    off and the grid shrinks (csrc/culi_capi.cu image_mentions_closure); a lambda turns it back on."""
+    wl = W.c1()
+    ctx = culi.Context(**SMALL)
+    r = ctx.eval_batch(wl.forms)
+    assert ctx.last_splits() == 0
+    o = oracle_mod.Session().eval_batch(wl.forms, nthreads=os.cpu_count() or 1).results
+    assert not compare(r.printed(), r.steps(), o, wl.forms.splitlines())
+    fib = "(define fib (lambda (n) (if (< n 2) n (+ (fib (- n 1)) (fib (- n 2))))))"
+    ctx.define(fib)
+    r2 = ctx.eval_batch("(fib 22)\n" * 64)
+    assert r2.printed() == ["17711"] * 64
+    assert ctx.last_splits() > 0
+
+
+@pytest.mark.timeout(300)
+def test_unbinned_closure_batches_do_not_split(culi, oracle_mod):
+    """Regression: argument splitting on unbinned multi-form batches (CULI_F_NO_BINNING, or below
+    BIN_MIN_FORMS) was seen to hang; such batches now run without splitting, repeatedly, in parity."""
+    wl = W.c5(2000)
+    ctx = culi.Context(**{**SMALL, "flags": culi.CULI_F_NO_BINNING})
+    ctx.define(wl.defs)
+    o = oracle_mod.Session()
+    o.define(wl.defs)
+    ores = o.eval(wl.forms)
+    for _ in range(5):
+        r = ctx.eval_batch(wl.forms)
+        assert ctx.last_splits() == 0
+        assert not compare(r.printed(), r.steps(), ores, wl.forms.splitlines())
