@@ -81,6 +81,9 @@ typedef struct {
 #define CULI_F_NO_SPLIT  32u   /* no argument splitting: each form is evaluated by one thread only        */
 #define CULI_F_NO_GC     64u   /* do not compact the persistent heap segment after culi_define (§8(f)3)  */
 #define CULI_F_NO_GRAPH 128u   /* culi_eval_uploaded issues its launches directly (no CUDA-graph replay)  */
+/* Without flags: batches of <= 4,096 forms with no lambda / defun in them or in any definition run in
+ * input order (no dispatch) and without argument splitting; argument splitting only runs where a closure
+ * can exist, and only in binned batches or single forms (so never with CULI_F_NO_BINNING) — DESIGN.md §5.5. */
 
 /* Fill *opts with defaults (device 0, default stream, default sizes). */
 void culi_default_opts(culi_opts* opts);
@@ -218,7 +221,8 @@ int culi_last_stats(const culi_ctx* ctx, uint32_t* fanout_forms, uint32_t* fallb
 /* Argument splitting (an implementation choice, not a paper mechanism): the number of
  * split groups the last fetched batch published — each group is up to 32 pending arguments of one warp
  * that an idle warp offered to evaluate (evaluated by it, or taken back by the owners).  Results, steps
- * and errors are identical with CULI_F_NO_SPLIT. */
+ * and errors are identical with CULI_F_NO_SPLIT.  0 for batches that do not split (see the note after
+ * the CULI_F_* flags). */
 int culi_last_splits(const culi_ctx* ctx, uint32_t* groups);
 
 #ifdef __cplusplus
