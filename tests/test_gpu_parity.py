@@ -444,3 +444,39 @@ def test_unbinned_closure_batches_do_not_split(culi, oracle_mod):
         r = ctx.eval_batch(wl.forms)
         assert ctx.last_splits() == 0
         assert not compare(r.printed(), r.steps(), ores, wl.forms.splitlines())
+
+
+DEFUN_DEFS = "\n".join([
+    "(defun sq (x) (* x x))",
+    "(defun k42 () 42)",
+    "(defun two (x) (+ x 1) (* x 2))",
+    "(defun fibd (n) (if (< n 2) n (+ (fibd (- n 1)) (fibd (- n 2)))))",
+    "(defun factd (n) (if (< n 2) 1 (* n (factd (- n 1)))))",
+    "(defun add3 (a b c) (+ a (* 10 b) (* 100 c)))",
+    "(defun mk (k) (lambda (x) (+ x k)))",
+])
+
+
+def test_defun_definitions(culi, oracle_mod):
+    """defun (SURVEY c.13 #12): functions defined with defun, through the host
+    reader and the device reader, against the oracle and the closed forms pinned in test_oracle_pins."""
+    forms = ["(sq 7)", "(k42)", "(two 5)", "(add3 1 2 3)", "sq", "(sq)", "(sq 'a)", "((mk 3) 4)",
+             "(||| 4 sq '(1 2 3 4))", "(||| 3 (mk 10) '(1 2 3))", "(defun z (x) x)"]
+    forms += ["(fibd %d)" % (n % 19) for n in range(600)] + ["(factd %d)" % (n % 22) for n in range(300)]
+    text = "\n".join(forms)
+    gp, gs, _ = assert_parity(culi, oracle_mod, DEFUN_DEFS, text)
+    assert gp[:5] == ["49", "42", "10", "321", "#<lambda>"] and gs[:4] == [7, 3, 11, 16]
+    assert gp[10] == "#<error DEFINE_IN_BATCH>"
+    for f, p, s in zip(forms, gp, gs):
+        if f.startswith("(fibd"):
+            n = int(f[6:-1])
+            assert (int(p), s) == (fib_py(n), 27 * fib_py(n + 1) - 17), f
+    ctx = culi.Context(**SMALL)
+    ctx.define_text(DEFUN_DEFS)
+    r = ctx.eval_text(text)
+    assert (r.printed(), r.steps()) == (gp, gs)
+    # redefinition through defun is seen by existing callers (late binding, L447-448)
+    ctx.define_text("(defun h (x) (sq (sq x)))")
+    assert ctx.eval_batch("(h 3)").printed() == ["81"]
+    ctx.define("(defun sq (x) (+ x x))")
+    assert ctx.eval_batch("(h 3)").printed() == ["12"]

@@ -117,32 +117,6 @@ def test_fuel_limit(oracle_mod):
     assert s2.eval1("(fib 5)").printed == "5"
 
 
-# ---- brute force: every arithmetic tree of op-depth <= 2 over {+,-,*} and ints {-2..2} -----------------
-def _trees(depth):
-    leaves = [str(v) for v in range(-2, 3)]
-    if depth == 0:
-        for l in leaves:
-            yield l, int(l), 0
-        return
-    subs = list(_trees(depth - 1))
-    for op in "+-*":
-        for (ta, va, oa), (tb, vb, ob) in itertools.product(subs, subs):
-            v = {"+": va + vb, "-": va - vb, "*": va * vb}[op]
-            yield "(%s %s %s)" % (op, ta, tb), v, oa + ob + 1
-
-
-def test_bruteforce_arith_trees(sess):
-    trees = [t for t in _trees(1)] + [t for t in _trees(2)]
-    # keep depth-2 trees exhaustive for the two left shapes, sample the rest deterministically
-    rnd = random.Random(7)
-    if len(trees) > 6000:
-        trees = trees[:2000] + rnd.sample(trees[2000:], 4000)
-    res = sess.eval("\n".join(t for t, _, _ in trees))
-    for (text, val, ops), r in zip(trees, res):
-        assert int(r.printed) == wrap64(val), text
-        assert r.steps == 3 * ops + 1, text          # 2 per list (list + head) + 1 per leaf; leaves = ops+1
-
-
 def test_int64_wrap_random(sess):
     rnd = random.Random(11)
     forms, exp = [], []
@@ -412,3 +386,139 @@ def test_setq_forms_are_independent(oracle_mod):
     s.define(SETQ_DEFS)
     out = [r.printed for r in s.eval("(let ((c (make-counter))) (c) (c))\n(let ((c (make-counter))) (c))")]
     assert out == ["2", "1"]
+
+
+# ---- defun (§III-A.b: function forms "stored in the global environment by the
+# keyword defun"; SURVEY c.5 / c.13 #12: defun is sugar for define + lambda, no extra steps) --------------
+DEFUN_DEFS = "\n".join([
+    "(defun sq (x) (* x x))",
+    "(defun k42 () 42)",
+    "(defun two (x) (+ x 1) (* x 2))",
+    "(defun fibd (n) (if (< n 2) n (+ (fibd (- n 1)) (fibd (- n 2)))))",
+    "(defun factd (n) (if (< n 2) 1 (* n (factd (- n 1)))))",
+    "(defun add3 (a b c) (+ a (* 10 b) (* 100 c)))",
+    "(defun firstp (a a) a)",
+])
+
+
+@pytest.fixture(scope="module")
+def defun_sess(oracle_mod):
+    s = oracle_mod.Session()
+    s.define(DEFUN_DEFS)
+    return s
+
+
+def test_defun_hand_derived(defun_sess):
+    # steps by c.4: (sq 7) = list 1 + head 1 + arg 1 + body (* x x) 4 = 7; (k42) = 2 + body atom 1 = 3;
+    # (two 5) = 3 + (+ x 1) 4 + (* x 2) 4 = 11; (add3 1 2 3) = 5 + body: list+head 2, a 1, (* 10 b) 4,
+    # (* 100 c) 4 = 16
+    cases = [("(sq 7)", "49", 7), ("(k42)", "42", 3), ("(two 5)", "10", 11), ("(add3 1 2 3)", "321", 16),
+             ("(firstp 1 2)", "1", 5), ("sq", "#<lambda>", 1), ("(sq)", "#<error ARITY>", 2),
+             ("(sq 1 2)", "#<error ARITY>", 4), ("(k42 1)", "#<error ARITY>", 3),
+             ("(sq 'a)", "#<error TYPE>", 8)]
+    res = defun_sess.eval("\n".join(c[0] for c in cases))
+    assert [(r.printed, r.steps) for r in res] == [(c[1], c[2]) for c in cases]
+
+
+def test_defun_closed_forms(defun_sess):
+    # the recurrences of c.12 hold unchanged for the defun-defined functions (defun adds no steps)
+    ns = list(range(0, 21))
+    res = defun_sess.eval("\n".join("(fibd %d)" % n for n in ns))
+    for n, r in zip(ns, res):
+        assert (int(r.printed), r.steps) == (fib_py(n), 27 * fib_py(n + 1) - 17)
+    res = defun_sess.eval("\n".join("(factd %d)" % n for n in ns))
+    for n, r in zip(ns, res):
+        assert (int(r.printed), r.steps) == (wrap64(math.factorial(n)), 15 * n - 5 if n >= 2 else 10)
+
+
+def test_defun_equals_define_lambda(oracle_mod, defun_sess):
+    # c.13 #12: defun is sugar — same value and same step count as the define + lambda spelling
+    s = oracle_mod.Session()
+    s.define("\n".join([
+        "(define sq (lambda (x) (* x x)))", "(define two (lambda (x) (+ x 1) (* x 2)))",
+        "(define fibd (lambda (n) (if (< n 2) n (+ (fibd (- n 1)) (fibd (- n 2))))))"]))
+    forms = "\n".join(["(sq 12)", "(two -3)", "(fibd 12)", "(list (sq 3) (two 4))", "(||| 3 sq '(1 2 3))"])
+    a = [(r.printed, r.steps) for r in s.eval(forms)]
+    b = [(r.printed, r.steps) for r in defun_sess.eval(forms)]
+    assert a == b
+
+
+def test_defun_syntax_errors(oracle_mod):
+    # reserved name, non-list parameters, reserved parameter, missing body: SYNTAX (c.5), no binding made
+    for bad in ["(defun if (x) x)", "(defun f x x)", "(defun f (car) car)", "(defun f)", "(defun 5 (x) x)"]:
+        s = oracle_mod.Session()
+        with pytest.raises(oracle_mod.OracleError, match="SYNTAX"):
+            s.define(bad)
+    s = oracle_mod.Session()
+    s.define("(defun f () )")                               # empty body -> nil (c.4)
+    assert (s.eval1("(f)").printed, s.eval1("(f)").steps) == ("nil", 2)
+
+
+def test_defun_redefinition_late_binding(oracle_mod):
+    # PAPER L98-101 / L447-448: a redefinition via defun is seen by existing callers
+    s = oracle_mod.Session()
+    s.define("(defun g (x) (+ x 1))\n(defun h (x) (g (g x)))")
+    assert s.eval1("(h 1)").printed == "3"
+    s.define("(defun g (x) (* x 10))")
+    assert s.eval1("(h 1)").printed == "100"
+
+
+# ---- comparisons (c.6: numeric, mixed -> f64, IEEE: nan compares false) against Python --------------------
+_CMP_INTS = [-2, -1, 0, 1, 2, 9007199254740992, 9007199254740993, -2**63, 2**63 - 1]
+_CMP_FLOATS = ["-1.5", "-0.0", "0.0", "0.5", "1.0", "2.0", "9007199254740992.0", "1e300", "-1e300"]
+_CMP_SPECIAL = {"(/ 1 0.0)": math.inf, "(/ -1 0.0)": -math.inf, "(/ 0 0.0)": math.nan}
+
+
+def _cmp_py(op, a, b):
+    if isinstance(a, float) or isinstance(b, float):
+        a, b = float(a), float(b)                             # Python int -> float rounds to nearest even
+    return {"=": a == b, "<": a < b, ">": a > b, "<=": a <= b, ">=": a >= b}[op]
+
+
+def test_comparisons_bruteforce(sess):
+    vals = [(str(v), v) for v in _CMP_INTS] + [(t, float(t)) for t in _CMP_FLOATS] + list(_CMP_SPECIAL.items())
+    forms, exp = [], []
+    for op in ("=", "<", ">", "<=", ">="):
+        for (ta, va), (tb, vb) in itertools.product(vals, vals):
+            forms.append("(%s %s %s)" % (op, ta, tb))
+            exp.append("T" if _cmp_py(op, va, vb) else "nil")
+    res = sess.eval("\n".join(forms))
+    got = [r.printed for r in res]
+    bad = [(f, g, e) for f, g, e in zip(forms, got, exp) if g != e]
+    assert not bad, bad[:10]
+    # steps: list + head + 2 atom args = 4 for atom operands
+    assert all(r.steps == 4 for f, r in zip(forms, res) if "(/" not in f)
+
+
+def test_comparison_errors(sess):
+    cases = [("(< 1)", "#<error ARITY>"), ("(>= 1 2 3)", "#<error ARITY>"), ("(<=)", "#<error ARITY>"),
+             ("(= 1 'a)", "#<error TYPE>"), ("(> nil 1)", "#<error TYPE>"), ("(< \"s\" 1)", "#<error TYPE>"),
+             ("(<= (list 1) 2)", "#<error TYPE>")]
+    assert [r.printed for r in sess.eval("\n".join(c[0] for c in cases))] == [c[1] for c in cases]
+
+
+# ---- brute force, exhaustive: EVERY arithmetic tree of op-depth <= 2 (mixed depths included) --------------
+def _trees_upto(depth):
+    """All trees of op-depth <= depth over {+,-,*} and leaves -2..2: (text, python value, op count)."""
+    leaves = [(str(v), v, 0) for v in range(-2, 3)]
+    if depth == 0:
+        return leaves
+    subs = _trees_upto(depth - 1)
+    out = list(subs)
+    seen = {t for t, _, _ in subs}
+    for op in "+-*":
+        for (ta, va, oa), (tb, vb, ob) in itertools.product(subs, subs):
+            text = "(%s %s %s)" % (op, ta, tb)
+            if text in seen:
+                continue
+            seen.add(text)
+            out.append((text, {"+": va + vb, "-": va - vb, "*": va * vb}[op], oa + ob + 1))
+    return out
+
+
+def test_bruteforce_arith_trees_exhaustive(sess):
+    trees = _trees_upto(2)
+    assert len(trees) == 5 + 75 + 3 * (80 * 80 - 25)        # leaves, depth-1, depth-2 (any child mix)
+    res = sess.eval("\n".join(t for t, _, _ in trees))
+    for (text, val, ops), r in zip(trees, res):
+        assert (int(r.printed), r.steps) == (wrap64(val), 3 * ops + 1), text
