@@ -82,8 +82,8 @@ typedef struct {
 #define CULI_F_NO_GC     64u   /* do not compact the persistent heap segment after culi_define (§8(f)3)  */
 #define CULI_F_NO_GRAPH 128u   /* culi_eval_uploaded issues its launches directly (no CUDA-graph replay)  */
 /* Without flags: batches of <= 4,096 forms with no lambda / defun in them or in any definition run in
- * input order (no dispatch) and without argument splitting; argument splitting only runs where a closure
- * can exist, and only in binned batches or single forms (so never with CULI_F_NO_BINNING) — DESIGN.md §5.5. */
+ * input order (no dispatch) and without argument splitting; argument splitting runs wherever a closure can
+ * exist (binned or not, CULI_F_NO_BINNING included) — DESIGN.md §5.5. */
 
 /* Fill *opts with defaults (device 0, default stream, default sizes). */
 void culi_default_opts(culi_opts* opts);
@@ -112,6 +112,8 @@ void culi_image_free(culi_image* img);
  * Stops at the first form whose evaluation errors: returns CULI_E_DEFINE, *failed_index = its index,
  * *failed_err = its culi_err; that binding is not created (earlier ones stay). */
 int culi_define(culi_ctx* ctx, const culi_image* defs, uint32_t* failed_index, uint8_t* failed_err);
+/* (culi_define / culi_define_text while a batch is uploaded with culi_upload*: CULI_E_STATE — the new
+ * definitions would land below the uploaded batch; culi_release it first.) */
 
 /* ---- eval (device, data-parallel) ------------------------------------------------------------------
  * Evaluate the image's forms as N independent evaluations (one thread each; top-level ||| forms fan out
@@ -224,6 +226,13 @@ int culi_last_stats(const culi_ctx* ctx, uint32_t* fanout_forms, uint32_t* fallb
  * and errors are identical with CULI_F_NO_SPLIT.  0 for batches that do not split (see the note after
  * the CULI_F_* flags). */
 int culi_last_splits(const culi_ctx* ctx, uint32_t* groups);
+/* Every wait of one warp on another (an owner joining a split argument, a thief reading a queue entry, a
+ * nested ||| waiting for its elements) is bounded by 10 s (env CULI_WAIT_MS).  A wait that gives up
+ * recovers exactly — the owner evaluates the argument itself / the form goes to the sequential fallback —
+ * so results are unaffected; it is counted here for the last fetched batch (*timeouts; 0 in a healthy
+ * run), and diag9 (if non-NULL, 9 entries) receives the first one's state: kind (1 join, 2 queue entry,
+ * 3 nested), group, lane, form, group state, task mask, owners remaining, task done flag, thief warp. */
+int culi_last_waits(const culi_ctx* ctx, uint32_t* timeouts, uint32_t* diag9);
 
 #ifdef __cplusplus
 }

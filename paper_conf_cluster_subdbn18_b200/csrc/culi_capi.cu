@@ -83,6 +83,7 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   c->stream = (cudaStream_t)o.stream;
   if (const char* e = getenv("CULI_SPLIT_POLL")) c->split_poll = std::max(1, atoi(e));      // tuning knobs
   if (const char* e = getenv("CULI_SPLIT_SLEEP")) c->split_sleep = std::max(32, atoi(e));
+  if (const char* e = getenv("CULI_WAIT_MS")) c->wait_ns = (unsigned long long)std::max(1, atoi(e)) * 1000000ull;
   bool ok = true;
   ok &= cudaMalloc(&c->H.tag, o.heap_nodes) == cudaSuccess;
   ok &= cudaMalloc(&c->H.word, o.heap_nodes * 8) == cudaSuccess;
@@ -101,8 +102,8 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   ok &= cudaMalloc(&c->nnest, 2 * sizeof(uint32_t)) == cudaSuccess;
   ok &= cudaMalloc(&c->ndesc, (size_t)c->maxnest * sizeof(NestDesc)) == cudaSuccess;
   ok &= cudaMalloc(&c->groups, (size_t)c->nslots / 32 * SPLIT_GPW * sizeof(SplitGroup)) == cudaSuccess;
-  ok &= cudaMalloc(&c->gqueue, (size_t)c->gqcap * sizeof(uint32_t)) == cudaSuccess;
-  ok &= cudaMalloc(&c->gcount, 4 * sizeof(uint32_t)) == cudaSuccess;
+  ok &= cudaMalloc(&c->gqueue, (size_t)c->gqcap * sizeof(unsigned long long)) == cudaSuccess;
+  ok &= cudaMalloc(&c->sctl, sizeof(SplitCtl)) == cudaSuccess;
   for (int k = 0; k < 4 && ok; ++k) ok &= cudaEventCreate(&c->ev[k]) == cudaSuccess;
   if (!ok) { culi_shutdown(c); return CULI_E_CUDA; }
   c->H.cap = o.heap_nodes;
@@ -115,8 +116,8 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
              cudaMemsetAsync(c->H.gtag, K_UNBOUND, GCAP, c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->flags, 0, 8 * sizeof(int), c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->groups, 0xff, (size_t)c->nslots / 32 * SPLIT_GPW * sizeof(SplitGroup), c->stream) == cudaSuccess &&
-             cudaMemsetAsync(c->gqueue, 0, (size_t)c->gqcap * sizeof(uint32_t), c->stream) == cudaSuccess &&
-             cudaMemsetAsync(c->gcount, 0, 4 * sizeof(uint32_t), c->stream) == cudaSuccess &&
+             cudaMemsetAsync(c->gqueue, 0, (size_t)c->gqcap * sizeof(unsigned long long), c->stream) == cudaSuccess &&
+             cudaMemsetAsync(c->sctl, 0, sizeof(SplitCtl), c->stream) == cudaSuccess &&
              cudaStreamSynchronize(c->stream) == cudaSuccess;
   if (!ok2) { culi_shutdown(c); return CULI_E_CUDA; }
   *out = c;
@@ -144,7 +145,7 @@ void culi_shutdown(culi_ctx* c) {
   cudaFree(c->ndesc);
   cudaFree(c->groups);
   cudaFree(c->gqueue);
-  cudaFree(c->gcount);
+  cudaFree(c->sctl);
   cudaFree(c->kst2);
   cudaFree(c->vst2);
   c->fallback.release();
@@ -256,10 +257,9 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.kst2 = c->kst2;
   A.vst2 = c->vst2;
   A.finished = c->nnest + 1;
-  // argument splitting: only where a closure may be applied, and only on binned batches (or one form):
-  // on unbinned multi-form batches (divergent warps) it was seen to hang (DESIGN.md §5.5 known issue)
-  A.split = (!define_mode && c->batch_may_close && (perm || nforms <= 1) &&
-             !(c->opts.flags & CULI_F_NO_SPLIT)) ? 1 : 0;
+  // argument splitting: where a closure may be applied (the poll sits at closure calls), binned or not
+  (void)perm;
+  A.split = (!define_mode && c->batch_may_close && !(c->opts.flags & CULI_F_NO_SPLIT)) ? 1 : 0;
   // setq (R7): frames go to the heap when made, and a form runs in one thread only (no fan-out, nested
   // fan-out or argument splitting: those evaluate parts of a form elsewhere, on copies of its frames)
   A.mut = define_mode ? c->define_mut : c->batch_mut;
@@ -275,8 +275,8 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.groups = c->groups;
   A.gqueue = c->gqueue;
   A.gqcap = c->gqcap;
-  A.gcount = c->gcount;
-  A.hungry = reinterpret_cast<int*>(c->gcount + 2);
+  A.sctl = c->sctl;
+  A.wait_ns = c->wait_ns;
   A.payload = c->payload.p;
   A.pcount = c->pcount;
   A.pcap = c->payload.n;
@@ -333,7 +333,7 @@ static int run_define(culi_ctx* c, uint32_t nf, uint64_t nnodes, uint32_t* faile
   int rc = ensure_results(c, nf);
   if (rc) return rc;
   CK(launch_reset(c->stream, c->H.top, c->mark + nnodes, c->next, c->pcount, c->flags, c->npend,
-                  c->nfallback, c->nnest, c->gcount));
+                  c->nfallback, c->nnest, c->sctl));
   EvalArgs A = make_args(c, nf, nullptr, 1);
   if (nf) CK(launch_define(c->stream, A));
   int flags[8];
@@ -362,6 +362,7 @@ static int run_define(culi_ctx* c, uint32_t nf, uint64_t nnodes, uint32_t* faile
 extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed_index,
                            uint8_t* failed_err) {
   if (!c || !defs) return CULI_E_ARG;
+  if (c->have_batch) return CULI_E_STATE;            // definitions go below an uploaded batch: release it first
   const Image& img = defs->img;
   uint32_t nf = (uint32_t)img.roots.size();
   uint32_t str_base = (uint32_t)c->strings.size();
@@ -378,6 +379,7 @@ extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed
 extern "C" int culi_define_text(culi_ctx* c, const char* text, size_t len, int text_on_device,
                                 uint32_t* failed_index, uint8_t* failed_err, size_t* err_offset) {
   if (!c || (!text && len)) return CULI_E_ARG;
+  if (c->have_batch) return CULI_E_STATE;
   ReadOut ro;
   int rc = device_read(c, text, len, text_on_device != 0, &ro, err_offset);
   if (rc) return rc;
@@ -404,7 +406,7 @@ static int run_batch_device(culi_ctx* c) {
   c->last_kernels = 0;
   CK(record_event(c, 0));
   CK(launch_reset(c->stream, c->H.top, c->mark + c->batch_nodes, c->next, c->pcount, c->flags, c->npend,
-                  c->nfallback, c->nnest, c->gcount));
+                  c->nfallback, c->nnest, c->sctl));
   ++c->last_kernels;
   uint32_t* perm = nullptr;
   if (!(c->opts.flags & CULI_F_NO_BINNING) && nf > 1 && (nf >= BIN_MIN_FORMS || c->batch_may_close)) {
@@ -562,9 +564,10 @@ static int fetch(culi_ctx* c, culi_results** out) {
   for (int attempt = 0; attempt < 4; ++attempt) {
     int flags[8];
     unsigned long long pc = 0, top = 0;
-    uint32_t nfb = 0, npend = 0, nnest = 0, ngroups = 0;
+    uint32_t nfb = 0, npend = 0, nnest = 0;
+    SplitCtl sc{};
     CK(cudaMemcpyAsync(&npend, c->npend, 4, cudaMemcpyDeviceToHost, c->stream));
-    if (attempt == 0) CK(cudaMemcpyAsync(&ngroups, c->gcount, 4, cudaMemcpyDeviceToHost, c->stream));
+    if (attempt == 0) CK(cudaMemcpyAsync(&sc, c->sctl, sizeof sc, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(&nnest, c->nnest, 4, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(flags, c->flags, sizeof flags, cudaMemcpyDeviceToHost, c->stream));
     CK(cudaMemcpyAsync(&pc, c->pcount, 8, cudaMemcpyDeviceToHost, c->stream));
@@ -577,7 +580,9 @@ static int fetch(culi_ctx* c, culi_results** out) {
       c->last_fanout = (c->batch_has_par && !(c->opts.flags & CULI_F_NO_FANOUT)) ? std::min(npend, c->maxdesc) : 0;
       c->last_fallback = 0;
       c->last_nested = c->batch_may_nest ? std::min(nnest, c->maxnest) : 0;
-      c->last_splits = ngroups;
+      c->last_splits = sc.published;
+      c->last_timeouts = sc.timeouts;
+      std::memcpy(c->last_diag, sc.diag, sizeof sc.diag);
     }
     if (nfb && !flags[3]) {
       c->last_fallback += nfb;
@@ -825,6 +830,13 @@ int culi_last_stats(const culi_ctx* c, uint32_t* fanout_forms, uint32_t* fallbac
 int culi_last_splits(const culi_ctx* c, uint32_t* groups) {
   if (!c || !groups) return CULI_E_ARG;
   *groups = c->last_splits;
+  return CULI_OK;
+}
+
+int culi_last_waits(const culi_ctx* c, uint32_t* timeouts, uint32_t* diag9) {
+  if (!c) return CULI_E_ARG;
+  if (timeouts) *timeouts = c->last_timeouts;
+  if (diag9) std::memcpy(diag9, c->last_diag, sizeof c->last_diag);
   return CULI_OK;
 }
 

@@ -145,9 +145,12 @@ struct culi_ctx {
   uint32_t last_fanout = 0, last_fallback = 0, last_nested = 0, last_splits = 0;
   // argument splitting
   SplitGroup* groups = nullptr;      // SPLIT_GPW per warp of the grid
-  uint32_t* gqueue = nullptr;
+  unsigned long long* gqueue = nullptr;
   uint32_t gqcap = 1u << 18;
-  uint32_t* gcount = nullptr;        // [0] queue tail (groups published), [1] queue head, [2] hungry (int)
+  SplitCtl* sctl = nullptr;          // queue counters (persist across launches), tokens, stats, diagnostics
+  unsigned long long wait_ns = 10ull * 1000 * 1000 * 1000;   // bounded inter-warp waits (env CULI_WAIT_MS)
+  uint32_t last_timeouts = 0;
+  uint32_t last_diag[9] = {0};
   uint32_t split_poll = 64;          // closure calls between polls (env CULI_SPLIT_POLL)
   uint32_t split_sleep = 4096;       // idle-warp back-off cap in ns (env CULI_SPLIT_SLEEP)
   DevBuf<uint32_t> wide;

@@ -89,10 +89,10 @@ struct EvalArgs {
   uint32_t split_poll;         // closure calls between two polls of the idle-warp counter
   uint32_t split_sleep;        // longest back-off (ns) of an idle warp polling for split groups
   struct SplitGroup* groups;   // SPLIT_GPW group slots per warp of the grid (slot reused after its join)
-  uint32_t* gqueue;            // ring of published group ids + 1 (0 = empty), gqcap entries
+  unsigned long long* gqueue;  // ring of published groups: ticket << 32 | (group + 1), gqcap entries
   uint32_t gqcap;              // power of two
-  uint32_t* gcount;            // [0] queue tail (groups published), [1] queue head (next entry a thief takes)
-  int* hungry;                 // idle thief warps minus open groups (owners split while > 0)
+  struct SplitCtl* sctl;       // queue counters, idle-warp tokens, statistics, bounded-wait diagnostics
+  unsigned long long wait_ns;  // longest wait for another warp (join, queue entry, nested |||) before giving up
 };
 
 // One top-level (||| n f l1 .. lm) form whose arguments have been evaluated.
@@ -151,9 +151,23 @@ struct SplitGroup {
   uint32_t remaining;                  // owner lanes that have not joined yet (0: the slot is free again)
   uint32_t mask;                       // lanes with a task
   uint32_t form;
+  uint32_t claimer;                    // global warp id of the thief (diagnostics)
+  uint32_t pad[3];
   SplitTask t[32];
 };
 constexpr uint32_t SPLIT_GPW = 8;      // group slots per warp
+// Queue counters live across launches: tickets are never reused, so an entry left in the ring by an earlier
+// launch (or an earlier lap of the ring) can never be mistaken for the one a thief is waiting for; the reset
+// kernel drops unclaimed entries by setting head = tail.
+struct SplitCtl {
+  unsigned long long tail;             // tickets handed out to publishers (monotonic)
+  unsigned long long head;             // next ticket a thief takes
+  int hungry;                          // idle thief warps minus open groups (owners split while > 0)
+  uint32_t published;                  // groups published in this launch (statistics)
+  uint32_t timeouts;                   // bounded waits that gave up in this launch (0 in a healthy run)
+  uint32_t diag[9];                    // the first one: kind, group, lane, form, state, mask, remaining, done, claimer
+};
+constexpr uint32_t WAIT_JOIN = 1, WAIT_QUEUE = 2, WAIT_NEST = 3;
 constexpr uint32_t SPLIT_OPEN = 0, SPLIT_CLAIMED = 1, SPLIT_TAKEN = 2;
 
 struct ExportArgs {
@@ -180,7 +194,7 @@ cudaError_t launch_define(cudaStream_t s, const EvalArgs& A);
 cudaError_t launch_export(cudaStream_t s, const ExportArgs& X, uint32_t blocks);
 cudaError_t launch_reset(cudaStream_t s, unsigned long long* top, unsigned long long top_value,
                          uint32_t* next, unsigned long long* pcount, int* flags, uint32_t* npend,
-                         uint32_t* nfallback, uint32_t* nnest, uint32_t* gcount);
+                         uint32_t* nfallback, uint32_t* nnest, struct SplitCtl* sctl);
 cudaError_t launch_fanout(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
 cudaError_t launch_nest_clear(cudaStream_t s, struct NestDesc* d, uint32_t n);
 cudaError_t launch_flat_export(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
@@ -192,8 +206,8 @@ uint32_t dispatch_launches(uint32_t nforms);   // kernels launch_dispatch issues
 // Batches of at most this many forms in which no closure can exist (no lambda / defun) are evaluated in
 // input order: with <= 128 warps (fewer than the 148 SMs) the eval time is the slowest warp's either way,
 // and the binning permutation scatters the warps' node loads.  Measured on C1 (1,024 forms): dispatch
-// 35 us + eval 51 us binned, eval 42 us not.  Batches with closures stay binned: argument splitting runs
-// only on binned batches (known issue: on unbinned multi-form batches it was seen to hang).
+// 35 us + eval 51 us binned, eval 42 us not.  Batches with closures stay binned: recursive forms of equal
+// shape and argument then share warps (converged lanes), which pays for the sort.
 constexpr uint32_t BIN_MIN_FORMS = 4097;
 
 struct V {

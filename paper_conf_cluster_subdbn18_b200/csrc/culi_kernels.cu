@@ -99,23 +99,37 @@ __device__ __forceinline__ bool nest_help_any(const EvalArgs& A, const Ctx& C2, 
 }
 
 // ---- argument splitting: a warp with no form left is a thief -----------------------------
-// It has offered itself (A.hungry += 1); lane 0 claims published groups in order (queue head A.gcount[1]).
-// Returns the group, or 0xffffffff once every form of the batch is finished.
-// Idle warps back off exponentially (up to A.split_sleep ns) so that they do not hammer the L2 line of the
-// queue counters.  A queue entry whose group is no longer open (taken back, or reused and already
-// claimed) is skipped.
+// It has offered itself (A.sctl->hungry += 1); lane 0 takes tickets in order (queue head) and claims the
+// group of the entry stamped with that ticket.  Returns the group, or 0xffffffff once every form of the
+// batch is finished.  Idle warps back off exponentially (up to A.split_sleep ns) so that they do not hammer
+// the L2 line of the queue counters.  An entry whose group is no longer open (taken back by its owners, or
+// reused and already claimed) is skipped; so is a ticket whose entry does not appear within A.wait_ns.
 __device__ __noinline__ uint32_t split_claim(const EvalArgs& A) {
+  SplitCtl* Q = A.sctl;
   uint32_t ns = 64;
   for (;;) {
-    uint32_t h = *(volatile uint32_t*)&A.gcount[1];
-    uint32_t n = *(volatile uint32_t*)&A.gcount[0];
+    unsigned long long h = *(volatile unsigned long long*)&Q->head;
+    unsigned long long n = *(volatile unsigned long long*)&Q->tail;
     if (h < n) {
-      if (atomicCAS(&A.gcount[1], h, h + 1) == h) {
-        uint32_t* qe = &A.gqueue[h & (A.gqcap - 1)];
-        uint32_t e;
-        while ((e = ld_acquire(qe)) == 0) __nanosleep(32);
-        *qe = 0;
-        if (atomicCAS(&A.groups[e - 1].state, SPLIT_OPEN, SPLIT_CLAIMED) == SPLIT_OPEN) return e - 1;
+      if (atomicCAS(&Q->head, h, h + 1) == h) {
+        unsigned long long* qe = &A.gqueue[h & (A.gqcap - 1)];
+        unsigned long long e = 0, t0 = 0;
+        bool ok = true;
+        for (uint32_t spin = 1;; ++spin) {
+          asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(e) : "l"(qe) : "memory");
+          if ((uint32_t)(e >> 32) == (uint32_t)h && (uint32_t)e != 0) break;
+          __nanosleep(32);
+          if ((spin & 63) == 0) {
+            unsigned long long now = gtime();
+            if (!t0) t0 = now;
+            else if (now - t0 > A.wait_ns) { wait_gave_up(A, WAIT_QUEUE, (uint32_t)h, 0); ok = false; break; }
+          }
+        }
+        uint32_t g = (uint32_t)e - 1;
+        if (ok && atomicCAS(&A.groups[g].state, SPLIT_OPEN, SPLIT_CLAIMED) == SPLIT_OPEN) {
+          A.groups[g].claimer = (blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+          return g;
+        }
       }
       ns = 64;
       continue;
@@ -168,7 +182,7 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
       if (b >= A.nforms) {
         if (!SPLIT) break;
         forms_left = false;
-        if (lane == 0) atomicAdd(A.hungry, 1);                 // offer this warp to the busy ones
+        if (lane == 0) atomicAdd(&A.sctl->hungry, 1);          // offer this warp to the busy ones
         continue;
       }
       uint32_t i = b + lane;
@@ -202,8 +216,14 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
         o = eval_form<FANOUT, false, NEST, SPLIT>(C, root, f, 0, 0, fuel, d, resume, R, env);
         if (!NEST || o.err != E_SUSPEND) break;
         NestDesc* D = A.ndesc + o.aux;                  // suspended on a nested |||: help until done
-        while (*(volatile uint32_t*)&D->done < D->n)
-          if (!nest_help_any(A, C2, D)) __nanosleep(128);
+        unsigned long long t0 = 0;
+        while (*(volatile uint32_t*)&D->done < D->n) {
+          if (nest_help_any(A, C2, D)) { t0 = 0; continue; }
+          __nanosleep(128);
+          unsigned long long now = gtime();                   // bounded: an element that never finishes
+          if (!t0) t0 = now;                                    // sends the form to the sequential fallback
+          else if (now - t0 > A.wait_ns) { wait_gave_up(A, WAIT_NEST, o.aux, f); atomicOr(&D->bad, 4u); break; }
+        }
         __threadfence();
         uint64_t s = D->steps0 + *(volatile unsigned long long*)&D->total;
         if (*(volatile uint32_t*)&D->bad || s > A.fuel) {   // decide exactly: sequential re-evaluation
@@ -231,7 +251,7 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
     }
     if (SPLIT && !forms_left) {
       __syncwarp();
-      if (lane == 0) atomicAdd(A.hungry, 1);                   // ready for the next group
+      if (lane == 0) atomicAdd(&A.sctl->hungry, 1);            // ready for the next group
     }
   }
   if (NEST) {                                           // no forms left: help until every form is done
@@ -310,9 +330,15 @@ __global__ void __launch_bounds__(128) culi_export_kernel(ExportArgs X) {
 
 __global__ void culi_reset_kernel(unsigned long long* top, unsigned long long top_value, uint32_t* next,
                                   unsigned long long* pcount, int* flags, uint32_t* npend,
-                                  uint32_t* nfallback, uint32_t* nnest, uint32_t* gcount) {
+                                  uint32_t* nfallback, uint32_t* nnest, SplitCtl* sctl) {
   *top = top_value;
-  if (gcount) { gcount[0] = 0; gcount[1] = 0; gcount[2] = 0; }
+  if (sctl) {                                         // tickets continue; unclaimed entries are dropped
+    sctl->head = sctl->tail;
+    sctl->hungry = 0;
+    sctl->published = 0;
+    sctl->timeouts = 0;
+    for (int k = 0; k < 9; ++k) sctl->diag[k] = 0;
+  }
   *next = 0;
   *pcount = 0;
   *npend = 0;
@@ -544,8 +570,8 @@ cudaError_t launch_export(cudaStream_t s, const ExportArgs& X, uint32_t blocks) 
 
 cudaError_t launch_reset(cudaStream_t s, unsigned long long* top, unsigned long long top_value,
                          uint32_t* next, unsigned long long* pcount, int* flags, uint32_t* npend,
-                         uint32_t* nfallback, uint32_t* nnest, uint32_t* gcount) {
-  culi_reset_kernel<<<1, 1, 0, s>>>(top, top_value, next, pcount, flags, npend, nfallback, nnest, gcount);
+                         uint32_t* nfallback, uint32_t* nnest, SplitCtl* sctl) {
+  culi_reset_kernel<<<1, 1, 0, s>>>(top, top_value, next, pcount, flags, npend, nfallback, nnest, sctl);
   return cudaGetLastError();
 }
 

@@ -806,6 +806,33 @@ __device__ __forceinline__ void st_release(uint32_t* p, uint32_t v) {
   asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
 }
 
+__device__ __forceinline__ unsigned long long gtime() {
+  unsigned long long t;
+  asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+  return t;
+}
+
+// A bounded wait gave up: count it and keep the first occurrence's state for diagnosis.
+// Every wait on another warp is bounded by EvalArgs.wait_ns, so a protocol bug shows up as a counter and a
+// status (culi_last_waits), never as a frozen GPU.
+__device__ CULI_COLD void wait_gave_up(const EvalArgs& A, uint32_t kind, uint32_t g, uint32_t form) {
+  if (atomicAdd(&A.sctl->timeouts, 1u) != 0) return;
+  uint32_t* d = A.sctl->diag;
+  d[0] = kind;
+  d[1] = g;
+  d[2] = threadIdx.x & 31;
+  d[3] = form;
+  if (kind == WAIT_JOIN) {
+    const SplitGroup* G = A.groups + g;
+    d[4] = *(volatile const uint32_t*)&G->state;
+    d[5] = *(volatile const uint32_t*)&G->mask;
+    d[6] = *(volatile const uint32_t*)&G->remaining;
+    d[7] = *(volatile const uint32_t*)&G->t[threadIdx.x & 31].done;
+    d[8] = *(volatile const uint32_t*)&G->claimer;
+  }
+  __threadfence();
+}
+
 // In-use bits of the SPLIT_GPW group slots of each warp of the block (the block has 4 warps); cleared by
 // the kernel prologue, set by try_split, cleared by the last owner lane that joins the group.
 __shared__ uint32_t culi_split_busy[4];
@@ -816,22 +843,32 @@ __shared__ uint32_t culi_split_busy[4];
 // the heap (promote) and publishes the argument as task `lane` of the group; the frame becomes KF_JOIN and
 // its V-stack header records the group.  The owner later joins (RET KF_JOIN): it takes the group back if
 // no thief claimed it.
+// The lanes that call this together are those of __activemask(): in a diverged warp several lane groups
+// can be here at once, each with its own leader.  The slot is therefore claimed with an atomic
+// test-and-set of its busy bit (a plain read-then-set let two lane groups share one slot: the second
+// overwrote mask / remaining of the first, whose owners then waited for tasks no thief ran).
 __device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t fuel, uint32_t form) {
   const EvalArgs& A = *C.A;
   unsigned mask = __activemask();
   int lane = threadIdx.x & 31;
   int leader = __ffs(mask) - 1;
   uint32_t* busy = &culi_split_busy[threadIdx.x >> 5];
+  SplitCtl* Q = A.sctl;
   int j = -1;
-  if (lane == leader && *(volatile int*)A.hungry > 0) {
-    uint32_t freeb = ~*(volatile uint32_t*)busy & ((1u << SPLIT_GPW) - 1u);
-    if (freeb) {
-      if (atomicSub(A.hungry, 1) > 0) {
-        j = __ffs(freeb) - 1;
-        atomicOr(busy, 1u << j);
+  if (lane == leader && *(volatile int*)&Q->hungry > 0 &&
+      *(volatile unsigned long long*)&Q->tail - *(volatile unsigned long long*)&Q->head < A.gqcap / 2) {
+    for (;;) {
+      uint32_t freeb = ~*(volatile uint32_t*)busy & ((1u << SPLIT_GPW) - 1u);
+      if (!freeb) break;
+      uint32_t bit = freeb & (0u - freeb);
+      if (atomicOr(busy, bit) & bit) continue;                  // another lane group took it: retry
+      if (atomicSub(&Q->hungry, 1) > 0) {
+        j = __ffs(bit) - 1;
       } else {
-        atomicAdd(A.hungry, 1);
+        atomicAdd(&Q->hungry, 1);
+        atomicAnd(busy, ~bit);
       }
+      break;
     }
   }
   j = __shfl_sync(mask, j, leader);
@@ -851,7 +888,7 @@ __device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t
   if (!part) {                                                  // nothing to split: return slot and token
     if (lane == leader) {
       atomicAnd(busy, ~(1u << j));
-      atomicAdd(A.hungry, 1);
+      atomicAdd(&Q->hungry, 1);
     }
     return;
   }
@@ -873,10 +910,13 @@ __device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t
     G->mask = part;
     G->remaining = __popc(part);
     G->form = form;
+    G->claimer = 0xffffffffu;
     __threadfence();
     st_release(&G->state, SPLIT_OPEN);
-    uint32_t q = atomicAdd(&A.gcount[0], 1u);
-    st_release(&A.gqueue[q & (A.gqcap - 1)], g + 1);
+    unsigned long long q = atomicAdd(&Q->tail, 1ull);
+    atomicAdd(&Q->published, 1u);
+    unsigned long long e = ((q & 0xffffffffull) << 32) | (g + 1);
+    asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(&A.gqueue[q & (A.gqcap - 1)]), "l"(e) : "memory");
   }
   __syncwarp(mask);
 }
@@ -885,6 +925,37 @@ __device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t
 __device__ __forceinline__ void split_release(const EvalArgs& A, uint32_t g) {
   if (atomicSub(&A.groups[g].remaining, 1u) == 1u)
     atomicAnd(&culi_split_busy[threadIdx.x >> 5], ~(1u << (g % SPLIT_GPW)));
+}
+
+// Owner side of a join whose group a thief claimed: wait for this lane's task (bounded).  false = the
+// wait gave up; the owner then evaluates the argument itself and leaves the slot busy for the rest of the
+// launch, so a late thief can never write into a reused group.
+__device__ CULI_COLD bool join_wait(const EvalArgs& A, SplitTask* T, uint32_t g, uint32_t form) {
+  unsigned long long t0 = gtime();
+  for (uint32_t spin = 1;; ++spin) {
+    if (ld_acquire(&T->done) != 0) return true;
+    __nanosleep(200);
+    if ((spin & 63) == 0 && gtime() - t0 > A.wait_ns) {
+      wait_gave_up(A, WAIT_JOIN, g, form);
+      return false;
+    }
+  }
+}
+
+// A lane leaves its evaluation with an error while KF_JOIN frames are on its stack: hand their groups
+// back (still open: take it back, return the token, release the slot) so a warp whose forms fail does not
+// lose its slots; a group already claimed stays busy until the launch ends (its thief still writes it).
+__device__ CULI_COLD void abandon_joins(Ctx C, uint32_t sp, uint4 ktop) {
+  const EvalArgs& A = *C.A;
+  for (uint32_t i = 0; i < sp; ++i) {
+    uint4 f = i + 1 == sp ? ktop : *KS(C, i);
+    if (kkind(f.w) != KF_JOIN) continue;
+    uint32_t g = VS(C, f.z)->z - 1;
+    if (atomicCAS(&A.groups[g].state, SPLIT_OPEN, SPLIT_TAKEN) == SPLIT_OPEN) {
+      atomicAdd(&A.sctl->hungry, 1);
+      split_release(A, g);
+    }
+  }
 }
 
 struct FormOut {
@@ -1285,11 +1356,11 @@ RET:
       uint32_t st = ld_acquire(&G->state);
       if (st == SPLIT_OPEN) {                                   // unclaimed: take it back, evaluate here
         st = atomicCAS(&G->state, SPLIT_OPEN, SPLIT_TAKEN);
-        if (st == SPLIT_OPEN) { atomicAdd(C.A->hungry, 1); st = SPLIT_TAKEN; }
+        if (st == SPLIT_OPEN) { atomicAdd(&C.A->sctl->hungry, 1); st = SPLIT_TAKEN; }
       }
       if (st == SPLIT_TAKEN) { split_release(*C.A, g); goto ARGS; }
       SplitTask* T = &G->t[threadIdx.x & 31];
-      while (ld_acquire(&T->done) == 0) __nanosleep(200);
+      if (ld_acquire(&T->done) == 0 && !join_wait(*C.A, T, g, form)) goto ARGS;   // gave up: evaluate here
       uint64_t ts = T->rsteps;
       uint32_t te = T->rerr;
       V tv = mkv(T->rt, T->rw);
@@ -1594,6 +1665,7 @@ PAR_NEXT: {
 
 
 done:
+  if (SPLIT && err != 0 && err != E_PENDING && err != E_SUSPEND && sp > 0) abandon_joins(C, sp, ktop);
 #undef FAIL
 #undef STEP
 #undef KPUSH

@@ -33,7 +33,7 @@ SYMBOLS = [
     "culi_result_int", "culi_result_float", "culi_print", "culi_results_totals", "culi_results_free",
     "culi_env_export", "culi_env_import", "culi_results_serialize", "culi_results_merge",
     "culi_status_string", "culi_error_name", "culi_last_timing", "culi_records_device",
-    "culi_last_stats", "culi_last_splits", "culi_image_pin", "culi_results_wire_bytes",
+    "culi_last_stats", "culi_last_splits", "culi_last_waits", "culi_image_pin", "culi_results_wire_bytes",
     "culi_define_text", "culi_eval_text", "culi_upload_text", "culi_last_read", "culi_collect",
     "culi_heap_usage",
 ]
@@ -95,6 +95,7 @@ def load(path: str = LIB_PATH) -> ctypes.CDLL:
         "culi_records_device": (I, [P, P, SZ, pp(SZ)]),
         "culi_last_stats": (I, [P, pp(U32), pp(U32), pp(U32)]),
         "culi_last_splits": (I, [P, pp(U32)]),
+        "culi_last_waits": (I, [P, pp(U32), pp(U32)]),
         "culi_image_pin": (I, [P, pp(U64)]),
         "culi_results_wire_bytes": (I, [P, pp(U64)]),
         "culi_define_text": (I, [P, P, SZ, I, pp(U32), pp(ctypes.c_uint8), pp(SZ)]),
@@ -397,6 +398,15 @@ class Context:
         g = ctypes.c_uint32()
         _check(load().culi_last_splits(self._p, ctypes.byref(g)), "culi_last_splits")
         return g.value
+
+    def last_waits(self) -> tuple[int, list[int]]:
+        """Bounded inter-warp waits that gave up in the last fetched batch (0 in a healthy run) and the first
+        one's state: [kind (1 join, 2 queue, 3 nested), group, lane, form, state, mask, remaining, done,
+        claimer]."""
+        n = ctypes.c_uint32()
+        d = (ctypes.c_uint32 * 9)()
+        _check(load().culi_last_waits(self._p, ctypes.byref(n), d), "culi_last_waits")
+        return n.value, list(d)
 
     def records_device(self, dev_ptr: int | None, cap: int = 0) -> int:
         need = ctypes.c_size_t(0)

@@ -5,6 +5,7 @@ from __future__ import annotations
 import os
 import random
 
+import numpy as np
 import pytest
 
 from paper_conf_cluster_subdbn18_b200 import workloads as W
@@ -430,20 +431,74 @@ def test_no_closure_batch_runs_without_splitting(culi, oracle_mod):
     assert ctx.last_splits() > 0
 
 
-@pytest.mark.timeout(300)
-def test_unbinned_closure_batches_do_not_split(culi, oracle_mod):
-    """Regression: argument splitting on unbinned multi-form batches (CULI_F_NO_BINNING, or below
-    BIN_MIN_FORMS) was seen to hang; such batches now run without splitting, repeatedly, in parity."""
+@pytest.mark.timeout(600)
+@pytest.mark.parametrize("flags", ["NO_BINNING", "binned"])
+def test_unbinned_closure_batches_split(culi, oracle_mod, flags):
+    """Regression (round 1: argument splitting on unbinned multi-form batches hung, so it was gated off):
+    unbinned (diverged warps) and binned closure batches now split, repeatedly, in parity, and no bounded
+    inter-warp wait ever gives up (atomic slot pick, ticket-stamped queue entries)."""
     wl = W.c5(2000)
-    ctx = culi.Context(**{**SMALL, "flags": culi.CULI_F_NO_BINNING})
+    fl = culi.CULI_F_NO_BINNING if flags == "NO_BINNING" else 0
+    ctx = culi.Context(**{**SMALL, "flags": fl})
     ctx.define(wl.defs)
     o = oracle_mod.Session()
     o.define(wl.defs)
     ores = o.eval(wl.forms)
-    for _ in range(5):
+    total = 0
+    for _ in range(8):
         r = ctx.eval_batch(wl.forms)
-        assert ctx.last_splits() == 0
+        total += ctx.last_splits()
+        assert ctx.last_waits()[0] == 0, ctx.last_waits()
         assert not compare(r.printed(), r.steps(), ores, wl.forms.splitlines())
+    assert total > 0
+    h = ctx.upload(wl.forms)                       # graph replay of the same unbinned step
+    for _ in range(50):
+        ctx.eval_uploaded(h)
+    r = ctx.fetch_results(h)
+    ctx.release(h)
+    assert ctx.last_waits()[0] == 0
+    assert not compare(r.printed(), r.steps(), ores, wl.forms.splitlines())
+
+
+@pytest.mark.timeout(600)
+def test_split_with_failing_forms_unbinned(culi, oracle_mod):
+    """Forms that fail while split groups are pending (abandon_joins) mixed with recursive forms in the same
+    warps, unbinned and repeated: parity, splits happen, no wait gives up."""
+    defs = "\n".join([W.FIB_DEF, W.SUM_DEF])
+    rng = np.random.default_rng(3)
+    kinds = ["(+ (fib %d) (fib %d))", "(+ (fib %d) (car %d))", "(list (fib %d) (sum 400) %d)",
+             "(+ (sum %d) (fib %d) (/ 1 0))", "(- (fib %d) (fib %d))"]
+    forms = []
+    for _ in range(3000):
+        k = kinds[rng.integers(0, len(kinds))]
+        forms.append(k % (rng.integers(8, 19), rng.integers(5, 16)))
+    text = "\n".join(forms)
+    gp, gs, o = run_both(culi, oracle_mod, defs, text, ctx_kw=dict(flags=culi.CULI_F_NO_BINNING))
+    assert not compare(gp, gs, o, forms)
+    ctx = culi.Context(**{**SMALL, "flags": culi.CULI_F_NO_BINNING})
+    ctx.define(defs)
+    splits = 0
+    for _ in range(6):
+        r = ctx.eval_batch(text)
+        splits += ctx.last_splits()
+        assert ctx.last_waits()[0] == 0, ctx.last_waits()
+        assert (r.printed(), r.steps()) == (gp, gs)
+    assert splits > 0
+
+
+def test_define_while_uploaded_is_a_state_error(culi):
+    """culi_define while a batch is uploaded would put definitions below the batch: CULI_E_STATE."""
+    ctx = culi.Context(**SMALL)
+    ctx.define(W.FIB_DEF)
+    h = ctx.upload("(fib 10)")
+    with pytest.raises(culi.CuliError) as ei:
+        ctx.define("(define x 1)")
+    assert ei.value.status == -7
+    with pytest.raises(culi.CuliError):
+        ctx.define_text("(define x 1)")
+    ctx.release(h)
+    ctx.define("(define x 1)")
+    assert ctx.eval_batch("(+ x (fib 10))").printed() == ["56"]
 
 
 DEFUN_DEFS = "\n".join([

@@ -11,7 +11,7 @@ from __future__ import annotations
 import struct
 
 MAGIC = 0x31534552494C5543
-RESERVED = ["quote", "if", "define", "defun", "defmacro", "lambda", "let", "progn",
+RESERVED = ["quote", "if", "define", "defun", "defmacro", "lambda", "let", "progn", "setq",
             "+", "-", "*", "/", "rem", "mod", "sqrt", "float", "trunc",
             "=", "<", ">", "<=", ">=", "eq", "equal", "null", "not",
             "atom", "consp", "numberp", "symbolp", "cons", "car", "cdr", "list",
