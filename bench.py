@@ -115,6 +115,20 @@ class ClockSampler:
                 "reasons": reasons, "samples": len(self.samples)}
 
 
+def host_cpu_info():
+    """lscpu model, sockets and SMT of the host the oracle runs on."""
+    info = {}
+    try:
+        out = subprocess.run(["lscpu"], capture_output=True, text=True, timeout=10).stdout
+        kv = {k.strip(): v.strip() for k, _, v in (l.partition(":") for l in out.splitlines()) if v}
+        info = {"model": kv.get("Model name"), "sockets": int(kv.get("Socket(s)", "0") or 0),
+                "threads_per_core": int(kv.get("Thread(s) per core", "0") or 0),
+                "cpus_online": kv.get("On-line CPU(s) list")}
+    except Exception:  # noqa: BLE001
+        pass
+    return info
+
+
 def host_cores():
     try:
         return len(os.sched_getaffinity(0))
@@ -170,8 +184,8 @@ def reference_arm(args):
         "vs_baseline": None, "dtype": "int64+f64", "data": "synthetic",
         "eval_steps_per_sec": steps_tot / t,
         "config": dict(bench_config(args.workload, args.gpus), sample=desc),
-        "cpu_baseline": {"value": value, "unit": "forms/s", "cores": threads, "kind": "oracle",
-                         "sample": desc},
+        "cpu_baseline": dict({"value": value, "unit": "forms/s", "cores": threads, "kind": "oracle",
+                              "sample": desc}, **host_cpu_info()),
         "e2e": {"value": value, "unit": "forms/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }
     print(json.dumps(line), flush=True)
@@ -277,6 +291,12 @@ def culi_arm(args):
     torch.cuda.synchronize()
     res = ctx.fetch_results(h)                  # parity-relevant numbers of this exact batch
     total_steps, n_err = res.totals()
+    wire_bytes = res.wire_bytes()
+    # the timed step is culi_eval_uploaded alone: it must not need the work a fetch can add afterwards
+    # (sequential fallback of undecidable ||| forms, eval + export re-run into a grown payload buffer)
+    fb0, regrow0 = ctx.last_reruns()
+    if fb0:
+        raise SystemExit("bench: %d forms needed the sequential fallback; the timed step would omit it" % fb0)
     del res
 
     # ---- timed region: K steps, CUDA events on the launching stream, L2 flushed between steps
@@ -299,6 +319,11 @@ def culi_arm(args):
         torch.cuda.synchronize()
     if world > 1:
         dist.barrier()
+    chk = ctx.fetch_results(h)                  # the timed steps' own results: same totals, no re-runs
+    assert chk.totals() == (total_steps, n_err) and ctx.last_reruns() == (0, 0), ctx.last_reruns()
+    waits_gave_up = ctx.last_waits()[0]
+    splits = ctx.last_splits()
+    del chk
     step_ms = [a.elapsed_time(b) for a, b in ev]
     t_rank = sum(step_ms) / 1e3
     t_max = t_rank
@@ -374,38 +399,47 @@ def culi_arm(args):
             dist.destroy_process_group()
         return
 
-    # ---- roofline of the dominant kernel (the eval kernel)
+    # ---- roofline of the dominant kernel (the eval kernel; for ||| workloads plus the fan-out kernel)
+    # the algorithmic HBM fraction = (bytes the method must move) / eval time / peak HBM.
+    # Algorithmic bytes of one launch = the batch image read once (9 B per node, SURVEY §8 canonical
+    # node) + the results written once (18 B record per form + 16 B per serialized list token, exactly
+    # the fetched bytes) + for ||| workloads each element's cell and value read from the environment
+    # (2 x 9 B).  C2: 4 nodes/form -> 36 + 18 = 54 B/form (§8(d): "52 B").  The kernel is in fact
+    # bound by instruction issue / latency (an interpreter); the issue-slot view is its own field.
     peaks, peak_src = load_peaks()
     eval_s = statistics.mean(eval_ms) / 1e3
     clocks = clk.summary()
     prof = load_inst_profile(args.workload)
-    # The dominant kernel is the eval phase (culi_eval_kernel; for ||| workloads plus the fan-out element
-    # kernel).  It is bound by instruction issue/latency (an interpreter: plain int64/f64 ALU + branches),
-    # so the roofline is the warp-instruction issue rate; the HBM view is reported beside it.
+    image_bytes = 9 * img.nnodes
+    env_bytes = 18 * wl.units if wl.units != wl.nforms else 0
+    alg_bytes = image_bytes + wire_bytes + env_bytes
+    hbm_ach = alg_bytes / eval_s / 1e9
     sm_mhz = peaks.get("sm_max_mhz", 1965.0)
     peak_inst = 148 * 4 * sm_mhz * 1e6 / 1e9          # G warp-instructions / s
     inst = prof.get("warp_inst_per_launch") if prof else None
     ach = inst / eval_s / 1e9 if inst else None
-    alg_bytes = {"C3": 36.0 * wl.units, "C0": 36.0 * wl.units,                # per element: read cons + float, write cons + box
-                 "C2": 52.0 * len(shard_idx), "C1": 190.0 * len(shard_idx),
-                 "C4": 120.0 * len(shard_idx), "C5": 120.0 * len(shard_idx)}.get(args.workload, 0.0)
-    hbm_ach = alg_bytes / eval_s / 1e9
-    roof = {"bound": "alu", "achieved": ach, "peak": peak_inst, "unit": "Gwarp-inst/s",
-            "frac": (ach / peak_inst) if ach else None,
+    roof = {"bound": "hbm", "achieved": hbm_ach, "peak": peaks["hbm_gbs"], "unit": "GB/s",
+            "frac": hbm_ach / peaks["hbm_gbs"],
             "traffic": prof.get("dram_bytes") if prof else None,
-            "peak_source": "148 SMs x 4 SMSP x 1 warp-inst/clk x %.0f MHz (B200_PROFILING.md, "
-                           "MEASURED_PEAKS sm_max_mhz)" % sm_mhz,
-            "achieved_source": ("ncu smsp__inst_executed.sum per launch (profiles/eval_inst_%s.json) / live "
-                                "eval-phase CUDA-event time" % args.workload.lower()) if inst else None,
-            "hbm_view": {"algorithmic_bytes": alg_bytes, "achieved_gbs": hbm_ach, "peak_gbs": peaks["hbm_gbs"],
-                         "frac": hbm_ach / peaks["hbm_gbs"], "peak_source": peak_src}}
+            "algorithmic_bytes": alg_bytes,
+            "algorithmic_source": "image %d B (9 B x %d nodes) + results %d B (fetched records + tokens) + "
+                                  "||| elements %d B, per eval launch / live eval-phase CUDA-event time"
+                                  % (image_bytes, img.nnodes, wire_bytes, env_bytes),
+            "peak_source": "MEASURED_PEAKS.json hbm_gbs (%s)" % peak_src,
+            "traffic_source": ("ncu dram__bytes_read.sum + dram__bytes_write.sum per launch "
+                               "(profiles/eval_inst_%s.json)" % args.workload.lower()) if prof else None,
+            "issue": {"achieved": ach, "peak": peak_inst, "unit": "Gwarp-inst/s",
+                      "frac": (ach / peak_inst) if ach else None,
+                      "peak_source": "148 SMs x 4 SMSP x 1 warp-inst/clk x %.0f MHz (B200_PROFILING.md)" % sm_mhz,
+                      "source": ("ncu smsp__inst_executed.sum per launch (profiles/eval_inst_%s.json) / "
+                                 "live eval-phase time" % args.workload.lower()) if inst else None}}
 
     cpu = None
     if world == 1 and not args.no_cpu_baseline:
         threads = host_cores()
         sample, desc, r = run_oracle(wl, ORACLE_SAMPLE[args.workload], threads)
-        cpu = {"value": sample.units / r.seconds, "unit": "forms/s", "cores": threads, "kind": "oracle",
-               "sample": desc, "eval_steps_per_sec": r.total_steps / r.seconds}
+        cpu = dict({"value": sample.units / r.seconds, "unit": "forms/s", "cores": threads, "kind": "oracle",
+                    "sample": desc, "eval_steps_per_sec": r.total_steps / r.seconds}, **host_cpu_info())
 
     ms_step = 1e3 * t_max / args.steps
     line = {
@@ -420,6 +454,7 @@ def culi_arm(args):
         "phases_ms": {"dispatch": statistics.mean(disp_ms), "eval": statistics.mean(eval_ms),
                       "export": statistics.mean(exp_ms)},
         "errors_in_batch": n_err, "read_s": t_read, "env_broadcast_ms": t_env,
+        "split_groups": splits, "waits_gave_up": waits_gave_up, "fallback_forms": 0, "payload_regrows": 0,
         "roofline": roof,
         "cpu_baseline": cpu,
         "e2e": {"value": e2e_value, "unit": "forms/s", "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,

@@ -71,7 +71,16 @@ typedef struct {
   uint32_t vstack_entries; /* value-stack entries per resident thread; 0 = default 4096                   */
   uint32_t slots;          /* resident eval threads (stack slots); 0 = default (SM count x 1024)         */
   uint32_t flags;          /* CULI_F_* below                                                              */
+  void* heap_base;         /* caller-owned device memory for the heap, global table, string area and
+                              stacks (e.g. a torch uint8 tensor's data_ptr); NULL = the library
+                              cudaMallocs them.  Borrowed: must outlive the ctx; 256-byte aligned.        */
+  uint64_t heap_bytes;     /* size of heap_base; at least culi_arena_bytes(opts) (CULI_E_ARG otherwise)   */
 } culi_opts;
+
+/* Bytes of device memory a ctx with these opts places in heap_base (heap tag + word arrays, the global
+ * frame, the string area, K- and V-stacks; SURVEY §8(d) "heap and stack budget").  The remaining session
+ * state (counters, descriptors, result buffers) stays library-allocated. */
+int culi_arena_bytes(const culi_opts* opts, uint64_t* bytes);
 
 #define CULI_F_NO_BINNING 1u   /* evaluate forms in input order (no classify+sort dispatch, §8(a)5)     */
 #define CULI_F_NO_FANOUT  2u   /* evaluate top-level ||| forms in one thread (no fan-out, §8(a)6)        */
@@ -123,12 +132,26 @@ int culi_define(culi_ctx* ctx, const culi_image* defs, uint32_t* failed_index, u
  * On CULI_E_HEAP_FULL no results are returned. */
 int culi_eval_batch(culi_ctx* ctx, const culi_image* forms, culi_results** out);
 
+/* Asynchronous variant (the paper's host-reads / device-evaluates split, L85-89, L477-480): uploads the
+ * image and enqueues dispatch + eval + export on ctx's stream, then returns without waiting; *out is a
+ * results object that is NOT ready (every accessor returns CULI_E_STATE) until culi_sync(ctx) completes
+ * it (D2H of records + payload; sequential fallbacks run there).  The host may read the next batch
+ * meanwhile.  One batch in flight per ctx: a second call before culi_sync returns CULI_E_STATE.  The image
+ * must stay alive until culi_sync (pin it with culi_image_pin for a true async H2D). */
+int culi_eval_batch_async(culi_ctx* ctx, const culi_image* forms, culi_results** out);
+/* Wait for the batch started by culi_eval_batch_async and complete its results (no-op without one). */
+int culi_sync(culi_ctx* ctx);
+
 /* Device-resident variant for timing (bench.py "value"): the image must already be uploaded with
  * culi_upload (done once); each call runs relocate-free dispatch + eval + export on the device and
  * leaves records on the device.  No host copies, no host synchronisation.  On a non-default stream the
  * first call captures the step into a CUDA graph and later calls replay it (CULI_F_NO_GRAPH: no graph). */
 int culi_upload(culi_ctx* ctx, const culi_image* forms, uint32_t* batch_handle);
 int culi_eval_uploaded(culi_ctx* ctx, uint32_t batch_handle);
+/* Complete the device-resident results of the last culi_eval_uploaded call without copying them to the
+ * host: sequential re-evaluation of undecided ||| forms, eval + export again into a grown payload buffer
+ * (synchronises).  Used before culi_results_export on the end-to-end multi-GPU path. */
+int culi_complete(culi_ctx* ctx, uint32_t batch_handle);
 /* Copy the device-resident results of the last culi_eval_uploaded call to the host (synchronises). */
 int culi_fetch_results(culi_ctx* ctx, uint32_t batch_handle, culi_results** out);
 /* Release an uploaded batch (resets the heap to the post-define mark). */
@@ -205,6 +228,25 @@ int culi_env_import(culi_ctx* ctx, const void* dev_buf, size_t bytes);
  * an NCCL all_gather): [tag u8 x n][err u8 x n][pad to 8][steps u64 x n][word u64 x n].  Stream-ordered,
  * no host synchronisation.  *bytes = size needed (always set); CULI_E_ARG if cap is too small. */
 int culi_records_device(culi_ctx* ctx, void* dev_buf, size_t cap, size_t* bytes);
+/* Device-resident result gather (the multi-GPU form of the paper's ordered result assembly,
+ * PAPER L584-589).  culi_results_export packs the results of the ctx's current batch (after
+ * culi_eval_uploaded; before culi_release) into dev_buf (device memory, for an NCCL all_gather of
+ * fixed-size buffers): a 64-byte header {magic "CULIRES2", nforms, npayload, names_bytes, nstr, payload
+ * capacity, overflow, 0}, then tag u8[n], err u8[n], steps u64[n], word u64[n] (8-aligned), the symbol
+ * names (NUL-separated, id order) and string bytes, then the payload tokens (16 B each, 16-aligned).
+ * Stream-ordered and without a host synchronisation: the token count is read on the device; tokens beyond
+ * the capacity left in dev_buf are dropped and the header's overflow flag is set.  With dev_buf == NULL,
+ * *bytes = the exact size these results need (this synchronises); otherwise *bytes = the fixed part +
+ * the payload capacity used.  CULI_E_ARG if cap cannot hold the fixed part. */
+int culi_results_export(culi_ctx* ctx, void* dev_buf, size_t cap, size_t* bytes);
+/* Merge per-rank exported buffers (device pointers, e.g. slices of the all_gather output on this ctx's
+ * device) into one host result set: records are scattered by global form index on the device, payload
+ * tokens concatenated with their offsets shifted, SYMBOL tokens re-interned by name, STRING offsets
+ * shifted; then one D2H.  form_index[r][k] = global index of rank r's k-th form, or form_index == NULL for
+ * the strided deal of SURVEY §8(e) (rank r's k-th form is r + k * nranks).  CULI_E_ARG on a bad buffer or
+ * an overflowed export (re-export with a larger capacity). */
+int culi_results_import(culi_ctx* ctx, const void* const* dev_bufs, const size_t* sizes, int nranks,
+                        const uint32_t* const* form_index, culi_results** merged);
 int culi_results_serialize(const culi_results* r, void* buf, size_t cap, size_t* bytes);
 int culi_results_merge(const void* const* blobs, const size_t* sizes, int nranks,
                        const uint32_t* const* form_index, culi_results** merged);
@@ -233,6 +275,11 @@ int culi_last_splits(const culi_ctx* ctx, uint32_t* groups);
  * run), and diag9 (if non-NULL, 9 entries) receives the first one's state: kind (1 join, 2 queue entry,
  * 3 nested), group, lane, form, group state, task mask, owners remaining, task done flag, thief warp. */
 int culi_last_waits(const culi_ctx* ctx, uint32_t* timeouts, uint32_t* diag9);
+/* Work the last fetch (culi_fetch_results / culi_eval_batch / culi_eval_text) did after the device step it
+ * fetched: forms re-evaluated by the sequential fallback (as culi_last_stats), and re-runs of eval + export
+ * because the result payload buffer had to grow.  A timed culi_eval_uploaded step does neither; a caller
+ * timing only that step checks both are 0 (bench.py does). */
+int culi_last_reruns(const culi_ctx* ctx, uint32_t* fallback_forms, uint32_t* payload_regrows);
 
 #ifdef __cplusplus
 }

@@ -31,7 +31,50 @@ static void drop_graph(culi_ctx* c) {
   c->graph_exec = nullptr;
 }
 
+// Caller-owned arena (culi_opts.heap_base): heap tag + word, global frame, string area, K- and V-stacks,
+// each 256-byte aligned, in this order.
+struct ArenaLayout {
+  size_t off[7];
+  size_t total;
+};
+static ArenaLayout arena_layout(uint64_t heap_nodes, uint64_t str_cap, size_t nslots, size_t kcap, size_t vcap) {
+  size_t sz[7] = {heap_nodes, heap_nodes * 8, GCAP, (size_t)GCAP * 8, str_cap, nslots * kcap * 16, nslots * vcap * 16};
+  ArenaLayout L{};
+  size_t o = 0;
+  for (int k = 0; k < 7; ++k) {
+    L.off[k] = o;
+    o = (o + sz[k] + 255) & ~(size_t)255;
+  }
+  L.total = o;
+  return L;
+}
+
+// opts with defaults filled in; false on an invalid value
+static bool normalize_opts(culi_opts& o, int sms) {
+  if (o.max_depth == 0) o.max_depth = 1024;
+  if (o.max_depth > 4095) return false;
+  if (o.fuel == 0) o.fuel = 1ull << 40;
+  if (o.heap_nodes == 0) o.heap_nodes = 64ull << 20;
+  if (o.heap_nodes > 0x7fffffffull) return false;
+  if (o.vstack_entries == 0) o.vstack_entries = 4096;
+  if (o.vstack_entries > 65535) return false;
+  if (o.slots == 0) o.slots = (uint32_t)sms * 128 * CULI_BLOCKS_PER_SM;
+  return true;
+}
+
 extern "C" {
+
+int culi_arena_bytes(const culi_opts* opts, uint64_t* bytes) {
+  if (!opts || !bytes) return CULI_E_ARG;
+  culi_opts o = *opts;
+  int ndev = 0, sms = 0;
+  if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev <= 0 || o.device >= ndev) return CULI_E_CUDA;
+  if (cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, o.device) != cudaSuccess) return CULI_E_CUDA;
+  if (!normalize_opts(o, sms)) return CULI_E_ARG;
+  size_t nslots = (o.slots + 127) / 128 * 128;
+  *bytes = arena_layout(o.heap_nodes, STR_CAP, nslots, 2 * o.max_depth + 8, o.vstack_entries).total;
+  return CULI_OK;
+}
 
 void culi_default_opts(culi_opts* o) {
   if (!o) return;
@@ -62,13 +105,6 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   culi_default_opts(&c->opts);
   if (opts) c->opts = *opts;
   culi_opts& o = c->opts;
-  if (o.max_depth == 0) o.max_depth = 1024;
-  if (o.max_depth > 4095) { delete c; return CULI_E_ARG; }
-  if (o.fuel == 0) o.fuel = 1ull << 40;
-  if (o.heap_nodes == 0) o.heap_nodes = 64ull << 20;
-  if (o.heap_nodes > 0x7fffffffull) { delete c; return CULI_E_ARG; }
-  if (o.vstack_entries == 0) o.vstack_entries = 4096;
-  if (o.vstack_entries > 65535) { delete c; return CULI_E_ARG; }
   int ndev = 0;
   if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev <= 0 || o.device >= ndev) {
     delete c;
@@ -76,23 +112,38 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   }
   if (cudaSetDevice(o.device) != cudaSuccess) { delete c; return CULI_E_CUDA; }
   cudaDeviceGetAttribute(&c->sms, cudaDevAttrMultiProcessorCount, o.device);
-  if (o.slots == 0) o.slots = (uint32_t)c->sms * 128 * CULI_BLOCKS_PER_SM;
+  if (!normalize_opts(o, c->sms)) { delete c; return CULI_E_ARG; }
   c->nslots = (o.slots + 127) / 128 * 128;
   c->kcap = 2 * o.max_depth + 8;
   c->vcap = o.vstack_entries;
   c->stream = (cudaStream_t)o.stream;
   if (const char* e = getenv("CULI_SPLIT_POLL")) c->split_poll = std::max(1, atoi(e));      // tuning knobs
+  if (const char* e = getenv("CULI_SPLIT_FIRST")) c->split_first = std::max(1, atoi(e));
   if (const char* e = getenv("CULI_SPLIT_SLEEP")) c->split_sleep = std::max(32, atoi(e));
   if (const char* e = getenv("CULI_WAIT_MS")) c->wait_ns = (unsigned long long)std::max(1, atoi(e)) * 1000000ull;
   bool ok = true;
-  ok &= cudaMalloc(&c->H.tag, o.heap_nodes) == cudaSuccess;
-  ok &= cudaMalloc(&c->H.word, o.heap_nodes * 8) == cudaSuccess;
+  if (o.heap_base) {                                 // caller-owned arena (e.g. a torch tensor)
+    ArenaLayout L = arena_layout(o.heap_nodes, c->str_cap, c->nslots, c->kcap, c->vcap);
+    if (o.heap_bytes < L.total || ((uintptr_t)o.heap_base & 255)) { delete c; return CULI_E_ARG; }
+    char* b = (char*)o.heap_base;
+    c->arena_owned = false;
+    c->H.tag = (uint8_t*)(b + L.off[0]);
+    c->H.word = (uint64_t*)(b + L.off[1]);
+    c->H.gtag = (uint8_t*)(b + L.off[2]);
+    c->H.gword = (uint64_t*)(b + L.off[3]);
+    c->H.strs = (const char*)(b + L.off[4]);
+    c->kst = (uint4*)(b + L.off[5]);
+    c->vst = (uint4*)(b + L.off[6]);
+  } else {
+    ok &= cudaMalloc(&c->H.tag, o.heap_nodes) == cudaSuccess;
+    ok &= cudaMalloc(&c->H.word, o.heap_nodes * 8) == cudaSuccess;
+    ok &= cudaMalloc(&c->H.gtag, GCAP) == cudaSuccess;
+    ok &= cudaMalloc(&c->H.gword, (size_t)GCAP * 8) == cudaSuccess;
+    ok &= cudaMalloc((void**)&c->H.strs, c->str_cap) == cudaSuccess;
+    ok &= cudaMalloc(&c->kst, (size_t)c->nslots * c->kcap * sizeof(uint4)) == cudaSuccess;
+    ok &= cudaMalloc(&c->vst, (size_t)c->nslots * c->vcap * sizeof(uint4)) == cudaSuccess;
+  }
   ok &= cudaMalloc(&c->H.top, sizeof(unsigned long long)) == cudaSuccess;
-  ok &= cudaMalloc(&c->H.gtag, GCAP) == cudaSuccess;
-  ok &= cudaMalloc(&c->H.gword, (size_t)GCAP * 8) == cudaSuccess;
-  ok &= cudaMalloc((void**)&c->H.strs, c->str_cap) == cudaSuccess;
-  ok &= cudaMalloc(&c->kst, (size_t)c->nslots * c->kcap * sizeof(uint4)) == cudaSuccess;
-  ok &= cudaMalloc(&c->vst, (size_t)c->nslots * c->vcap * sizeof(uint4)) == cudaSuccess;
   ok &= cudaMalloc(&c->next, sizeof(uint32_t)) == cudaSuccess;
   ok &= cudaMalloc(&c->pcount, sizeof(unsigned long long)) == cudaSuccess;
   ok &= cudaMalloc(&c->flags, 8 * sizeof(int)) == cudaSuccess;
@@ -126,15 +177,21 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
 
 void culi_shutdown(culi_ctx* c) {
   if (!c) return;
-  if (c->stream || true) cudaStreamSynchronize(c->stream);
-  cudaFree(c->H.tag);
-  cudaFree(c->H.word);
+  cudaStreamSynchronize(c->stream);
+  if (c->pending) {                                  // an async batch nobody synced: results stay not ready
+    c->pending->owner = nullptr;
+    c->pending = nullptr;
+  }
+  if (c->arena_owned) {
+    cudaFree(c->H.tag);
+    cudaFree(c->H.word);
+    cudaFree(c->H.gtag);
+    cudaFree(c->H.gword);
+    cudaFree((void*)c->H.strs);
+    cudaFree(c->kst);
+    cudaFree(c->vst);
+  }
   cudaFree(c->H.top);
-  cudaFree(c->H.gtag);
-  cudaFree(c->H.gword);
-  cudaFree((void*)c->H.strs);
-  cudaFree(c->kst);
-  cudaFree(c->vst);
   cudaFree(c->next);
   cudaFree(c->pcount);
   cudaFree(c->flags);
@@ -271,6 +328,7 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
     A.wide = nullptr;
   }
   A.split_poll = c->split_poll;
+  A.split_first = c->split_first;
   A.split_sleep = c->split_sleep;
   A.groups = c->groups;
   A.gqueue = c->gqueue;
@@ -362,7 +420,7 @@ static int run_define(culi_ctx* c, uint32_t nf, uint64_t nnodes, uint32_t* faile
 extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed_index,
                            uint8_t* failed_err) {
   if (!c || !defs) return CULI_E_ARG;
-  if (c->have_batch) return CULI_E_STATE;            // definitions go below an uploaded batch: release it first
+  if (c->have_batch || c->pending) return CULI_E_STATE;   // definitions go below an uploaded batch: release it first
   const Image& img = defs->img;
   uint32_t nf = (uint32_t)img.roots.size();
   uint32_t str_base = (uint32_t)c->strings.size();
@@ -379,7 +437,7 @@ extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed
 extern "C" int culi_define_text(culi_ctx* c, const char* text, size_t len, int text_on_device,
                                 uint32_t* failed_index, uint8_t* failed_err, size_t* err_offset) {
   if (!c || (!text && len)) return CULI_E_ARG;
-  if (c->have_batch) return CULI_E_STATE;
+  if (c->have_batch || c->pending) return CULI_E_STATE;
   ReadOut ro;
   int rc = device_read(c, text, len, text_on_device != 0, &ro, err_offset);
   if (rc) return rc;
@@ -559,8 +617,9 @@ static int rerun_fallback(culi_ctx* c, uint32_t nfb) {
   return CULI_OK;
 }
 
-static int fetch(culi_ctx* c, culi_results** out) {
-  uint32_t nf = c->batch_forms;
+// Finish the device-resident results of the current batch: sequential fallbacks of undecided ||| forms,
+// eval + export again into a grown payload buffer.  Synchronises.  *pc = payload tokens.
+static int complete_device(culi_ctx* c, unsigned long long* pc_out) {
   for (int attempt = 0; attempt < 4; ++attempt) {
     int flags[8];
     unsigned long long pc = 0, top = 0;
@@ -577,6 +636,7 @@ static int fetch(culi_ctx* c, culi_results** out) {
     c->heap_high = std::max<uint64_t>(c->heap_high, std::min<unsigned long long>(top, c->H.cap));
     if (flags[0] || flags[4]) return CULI_E_HEAP_FULL;
     if (attempt == 0) {
+      c->last_regrows = 0;
       c->last_fanout = (c->batch_has_par && !(c->opts.flags & CULI_F_NO_FANOUT)) ? std::min(npend, c->maxdesc) : 0;
       c->last_fallback = 0;
       c->last_nested = c->batch_may_nest ? std::min(nnest, c->maxnest) : 0;
@@ -591,6 +651,8 @@ static int fetch(culi_ctx* c, culi_results** out) {
       continue;
     }
     if (flags[3]) {                                  // payload buffer too small: grow, re-export
+      ++c->last_regrows;
+      drop_graph(c);                                 // a captured step still points at the old buffer
       CK(c->payload.ensure((size_t)pc + 1024));
       int zero[8] = {0};
       CK(cudaMemcpyAsync(c->flags, zero, sizeof zero, cudaMemcpyHostToDevice, c->stream));
@@ -601,6 +663,19 @@ static int fetch(culi_ctx* c, culi_results** out) {
       if (rc) return rc;
       continue;
     }
+    *pc_out = pc;
+    return CULI_OK;
+  }
+  return CULI_E_HEAP_FULL;
+}
+
+// complete_device + D2H of records and payload into a new results object
+static int fetch(culi_ctx* c, culi_results** out) {
+  uint32_t nf = c->batch_forms;
+  unsigned long long pc = 0;
+  int rc = complete_device(c, &pc);
+  if (rc) return rc;
+  {
     culi_results* r = new (std::nothrow) culi_results;
     if (!r) return CULI_E_ARG;
     r->r.resize(nf);
@@ -619,14 +694,56 @@ static int fetch(culi_ctx* c, culi_results** out) {
     *out = r;
     return CULI_OK;
   }
-  return CULI_E_HEAP_FULL;
 }
 
 extern "C" {
 
+int culi_eval_batch_async(culi_ctx* c, const culi_image* forms, culi_results** out) {
+  if (!c || !forms || !out) return CULI_E_ARG;
+  *out = nullptr;
+  if (c->pending || c->have_batch) return CULI_E_STATE;
+  culi_results* r = new (std::nothrow) culi_results;
+  if (!r) return CULI_E_ARG;
+  int rc = prepare_batch(c, forms->img);
+  if (!rc) rc = run_batch_device(c);
+  if (rc) {
+    c->have_batch = false;
+    delete r;
+    return rc;
+  }
+  r->ready = false;
+  r->owner = c;
+  c->pending = r;
+  *out = r;
+  return CULI_OK;
+}
+
+int culi_sync(culi_ctx* c) {
+  if (!c) return CULI_E_ARG;
+  if (!c->pending) return cudaStreamSynchronize(c->stream) == cudaSuccess ? CULI_OK : CULI_E_CUDA;
+  culi_results* p = c->pending;
+  c->pending = nullptr;
+  culi_results* tmp = nullptr;
+  int rc = fetch(c, &tmp);
+  c->have_batch = false;
+  p->owner = nullptr;
+  if (rc) return rc;                                 // p stays not ready
+  p->r = std::move(tmp->r);
+  p->ready = true;
+  delete tmp;
+  return CULI_OK;
+}
+
+int culi_complete(culi_ctx* c, uint32_t handle) {
+  if (!c || handle != 1 || !c->have_batch) return CULI_E_STATE;
+  unsigned long long pc = 0;
+  return complete_device(c, &pc);
+}
+
 int culi_eval_batch(culi_ctx* c, const culi_image* forms, culi_results** out) {
   if (!c || !forms || !out) return CULI_E_ARG;
   *out = nullptr;
+  if (c->pending) return CULI_E_STATE;
   int rc = prepare_batch(c, forms->img);
   if (rc) return rc;
   rc = run_batch_device(c);
@@ -639,6 +756,7 @@ int culi_eval_batch(culi_ctx* c, const culi_image* forms, culi_results** out) {
 int culi_eval_text(culi_ctx* c, const char* text, size_t len, int text_on_device, culi_results** out,
                    size_t* err_offset) {
   if (!c || !out || (!text && len)) return CULI_E_ARG;
+  if (c->pending) return CULI_E_STATE;
   *out = nullptr;
   int rc = prepare_text(c, text, len, text_on_device != 0, err_offset);
   if (rc) return rc;
@@ -652,6 +770,7 @@ int culi_eval_text(culi_ctx* c, const char* text, size_t len, int text_on_device
 int culi_upload_text(culi_ctx* c, const char* text, size_t len, int text_on_device, uint32_t* handle,
                      uint32_t* nforms, size_t* err_offset) {
   if (!c || (!text && len)) return CULI_E_ARG;
+  if (c->pending) return CULI_E_STATE;
   int rc = prepare_text(c, text, len, text_on_device != 0, err_offset);
   if (rc) return rc;
   if (handle) *handle = 1;
@@ -687,6 +806,7 @@ int culi_last_read(const culi_ctx* c, float* ms, uint64_t* items, uint64_t* node
 
 int culi_upload(culi_ctx* c, const culi_image* forms, uint32_t* handle) {
   if (!c || !forms) return CULI_E_ARG;
+  if (c->pending) return CULI_E_STATE;
   int rc = prepare_batch(c, forms->img);
   if (rc) return rc;
   CK(cudaStreamSynchronize(c->stream));
@@ -753,9 +873,10 @@ int culi_records_device(culi_ctx* c, void* dev_buf, size_t cap, size_t* bytes) {
   return CULI_OK;
 }
 
-uint32_t culi_results_count(const culi_results* r) { return r ? (uint32_t)r->r.size() : 0; }
+uint32_t culi_results_count(const culi_results* r) { return r && r->ready ? (uint32_t)r->r.size() : 0; }
 
 int culi_result_info(const culi_results* r, uint32_t i, uint8_t* tag, uint8_t* err, uint64_t* steps) {
+  if (r && !r->ready) return CULI_E_STATE;
   if (!r || i >= r->r.size()) return CULI_E_ARG;
   const Record x = r->r.at(i);
   if (tag) *tag = x.tag;
@@ -765,6 +886,7 @@ int culi_result_info(const culi_results* r, uint32_t i, uint8_t* tag, uint8_t* e
 }
 
 int culi_result_int(const culi_results* r, uint32_t i, int64_t* v) {
+  if (r && !r->ready) return CULI_E_STATE;
   if (!r || i >= r->r.size() || !v) return CULI_E_ARG;
   const Record x = r->r.at(i);
   if (x.err || x.tag != K_INT) return CULI_E_ARG;
@@ -773,6 +895,7 @@ int culi_result_int(const culi_results* r, uint32_t i, int64_t* v) {
 }
 
 int culi_result_float(const culi_results* r, uint32_t i, double* v) {
+  if (r && !r->ready) return CULI_E_STATE;
   if (!r || i >= r->r.size() || !v) return CULI_E_ARG;
   const Record x = r->r.at(i);
   if (x.err || x.tag != K_FLOAT) return CULI_E_ARG;
@@ -781,6 +904,7 @@ int culi_result_float(const culi_results* r, uint32_t i, double* v) {
 }
 
 int culi_print(const culi_results* r, uint32_t i, char* buf, size_t cap, size_t* needed) {
+  if (r && !r->ready) return CULI_E_STATE;
   if (!r || i >= r->r.size()) return CULI_E_ARG;
   std::string s;
   r->r.print(i, s);
@@ -799,6 +923,7 @@ int culi_print(const culi_results* r, uint32_t i, char* buf, size_t cap, size_t*
 
 int culi_results_totals(const culi_results* r, uint64_t* total_steps, uint32_t* n_errors) {
   if (!r) return CULI_E_ARG;
+  if (!r->ready) return CULI_E_STATE;
   uint64_t t = 0;
   uint32_t ne = 0;
   for (size_t q = 0; q < r->r.size(); ++q) {
@@ -810,10 +935,14 @@ int culi_results_totals(const culi_results* r, uint64_t* total_steps, uint32_t* 
   return CULI_OK;
 }
 
-void culi_results_free(culi_results* r) { delete r; }
+void culi_results_free(culi_results* r) {
+  if (r && !r->ready && r->owner) culi_sync(r->owner);   // finish the batch before its results go away
+  delete r;
+}
 
 int culi_results_wire_bytes(const culi_results* r, uint64_t* d2h_bytes) {
   if (!r || !d2h_bytes) return CULI_E_ARG;
+  if (!r->ready) return CULI_E_STATE;
   *d2h_bytes = r->r.size() * 18 + r->r.payload.size() * sizeof(Token);
   return CULI_OK;
 }
@@ -830,6 +959,13 @@ int culi_last_stats(const culi_ctx* c, uint32_t* fanout_forms, uint32_t* fallbac
 int culi_last_splits(const culi_ctx* c, uint32_t* groups) {
   if (!c || !groups) return CULI_E_ARG;
   *groups = c->last_splits;
+  return CULI_OK;
+}
+
+int culi_last_reruns(const culi_ctx* c, uint32_t* fallback_forms, uint32_t* payload_regrows) {
+  if (!c) return CULI_E_ARG;
+  if (fallback_forms) *fallback_forms = c->last_fallback;
+  if (payload_regrows) *payload_regrows = c->last_regrows;
   return CULI_OK;
 }
 

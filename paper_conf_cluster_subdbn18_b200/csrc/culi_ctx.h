@@ -29,6 +29,8 @@ struct culi_image {
 
 struct culi_results {
   Results r;
+  bool ready = true;                 // false: an async batch's results before culi_sync
+  struct culi_ctx* owner = nullptr;  // the ctx whose culi_sync completes them (while not ready)
 };
 
 namespace culi_detail {
@@ -105,6 +107,8 @@ struct culi_ctx {
   culi_opts opts;
   cudaStream_t stream = nullptr;
   int sms = 0;
+  bool arena_owned = true;           // heap / global frame / strings / stacks cudaMalloc'ed here (else opts.heap_base)
+  culi_results* pending = nullptr;   // culi_eval_batch_async results awaiting culi_sync
   std::shared_ptr<SymTable> syms = std::make_shared<SymTable>();
   uint64_t str_cap = STR_CAP;
   std::string strings;              // host mirror of the device string area (persistent part)
@@ -150,8 +154,10 @@ struct culi_ctx {
   SplitCtl* sctl = nullptr;          // queue counters (persist across launches), tokens, stats, diagnostics
   unsigned long long wait_ns = 10ull * 1000 * 1000 * 1000;   // bounded inter-warp waits (env CULI_WAIT_MS)
   uint32_t last_timeouts = 0;
+  uint32_t last_regrows = 0;         // payload-buffer regrowths (eval + export re-run) in the last fetch
   uint32_t last_diag[9] = {0};
   uint32_t split_poll = 64;          // closure calls between polls (env CULI_SPLIT_POLL)
+  uint32_t split_first = 64;         // closure calls before the first poll (env CULI_SPLIT_FIRST)
   uint32_t split_sleep = 4096;       // idle-warp back-off cap in ns (env CULI_SPLIT_SLEEP)
   DevBuf<uint32_t> wide;
   // uploaded batch (culi_upload)

@@ -87,6 +87,7 @@ struct EvalArgs {
   uint32_t gst;                // global-frame entries staged in shared memory
   uint32_t split;              // argument splitting: idle warps evaluate pending arguments of busy ones
   uint32_t split_poll;         // closure calls between two polls of the idle-warp counter
+  uint32_t split_first;        // closure calls before an evaluation's first poll (split the top of the tree early)
   uint32_t split_sleep;        // longest back-off (ns) of an idle warp polling for split groups
   struct SplitGroup* groups;   // SPLIT_GPW group slots per warp of the grid (slot reused after its join)
   unsigned long long* gqueue;  // ring of published groups: ticket << 32 | (group + 1), gqcap entries
@@ -123,6 +124,9 @@ constexpr uint8_t K_FLATREC = 12;
 // and adds their steps; when done == n the owner resumes at RET with the result spine.
 constexpr uint32_t NEST_MIN = 32;
 constexpr uint8_t E_SUSPEND = 0xfc;
+// Warp voting (north_star "ballot for branch voting"): a lane group that diverged yields
+// at a return; the kernel re-forms groups by (stack height, continuation kind) and resumes the deepest.
+constexpr uint8_t E_YIELD = 0xfb;
 struct NestDesc {
   uint32_t form, n, m, spine;
   uint32_t ftag, depth;

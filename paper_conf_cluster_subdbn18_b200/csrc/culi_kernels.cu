@@ -260,6 +260,67 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
   }
 }
 
+// Batch mode with warp voting (north_star: "ballot for branch voting").  Divergence is the
+// cost the paper names for SIMT evaluation of different forms (§III-D.d).  A warp takes 32
+// forms; the lanes start together; a lane group that diverges yields at its next return (E_YIELD, its
+// state saved); the warp then votes: every waiting lane offers key = stack height << 4 | kind of the
+// continuation it is about to pop, __reduce_max_sync picks the deepest, and the lanes with that key are
+// resumed together (same height and same continuation: the same place of the same-shaped form).  The
+// group runs until it diverges again or returns down to the height of the deepest other waiting lane,
+// where the groups merge.  Used for batches that neither split arguments nor nest |||.
+template <bool FANOUT>
+__global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_vote_kernel(const __grid_constant__ EvalArgs A) {
+  uint64_t* sgword = reinterpret_cast<uint64_t*>(culi_smem);
+  uint8_t* sgtag = reinterpret_cast<uint8_t*>(sgword + A.gst);
+  for (uint32_t i = threadIdx.x; i < A.gst; i += blockDim.x) {
+    sgword[i] = A.H.gword[i];
+    sgtag[i] = A.H.gtag[i];
+  }
+  __syncthreads();
+  uint32_t slot = blockIdx.x * blockDim.x + threadIdx.x;
+  Ctx C = make_ctx(A, slot);
+  int lane = threadIdx.x & 31;
+  for (;;) {
+    uint32_t b = 0;
+    if (lane == 0) b = atomicAdd(A.next, 32u);
+    b = __shfl_sync(0xffffffffu, b, 0);
+    if (b >= A.nforms) break;
+    uint32_t i = b + lane, f = 0, root = 0, key = 0;
+    bool live = i < A.nforms, fresh = true;
+    if (live) {
+      f = A.perm ? A.perm[i] : i;
+      root = A.roots[f];
+    }
+    Resume R{};
+    R.grp = __ballot_sync(0xffffffffu, live);                  // first: every lane from its root
+    R.wait = 0;
+    for (;;) {
+      if ((R.grp >> lane) & 1u) {
+        FormOut o = eval_form<FANOUT, false, false, false, true>(C, root, f, 0, 0, A.fuel, 1, !fresh, R);
+        fresh = false;
+        if (o.err == E_YIELD) {
+          R.sp = o.aux;
+          R.vtop = o.vtop;
+          R.steps = o.steps;
+          R.v = mkv(o.t, o.w);
+          key = (o.aux << 4) | o.kk;
+        } else {
+          write_result(A, f, o);
+          live = false;
+        }
+      }
+      __syncwarp();
+      uint32_t mykey = live ? key : 0u;
+      uint32_t best = __reduce_max_sync(0xffffffffu, mykey);
+      if (best == 0) break;                                     // every lane's form is finished
+      unsigned grp = __ballot_sync(0xffffffffu, live && mykey == best);
+      uint32_t wait = __reduce_max_sync(0xffffffffu, (live && mykey != best) ? (key >> 4) : 0u);
+      if ((grp >> lane) & 1u) { R.grp = grp; R.wait = wait; }
+      else R.grp = grp;                                         // (not resumed: only the membership test)
+    }
+  }
+}
+
 // Define mode (culi_define): forms evaluated in order by one thread; define/defun/defmacro write the
 // global frame; stops at the first error.  No staging: this kernel writes globals.
 __global__ void culi_define_kernel(const __grid_constant__ EvalArgs A) {
@@ -546,9 +607,11 @@ cudaError_t launch_eval(cudaStream_t s, const EvalArgs& A, uint32_t blocks) {
   // specialised on whether the batch holds top-level ||| / wide forms (FANOUT), whether ||| can occur
   // below the top level (NEST) and whether idle warps split arguments off busy ones (SPLIT; not combined
   // with NEST, whose helpers use the idle warps)
+  // and whether lane groups vote (VOTE: neither nesting nor splitting, code staging off)
   void (*k)(EvalArgs);
   if (A.nest) k = A.fanout ? culi_eval_kernel<true, true, false> : culi_eval_kernel<false, true, false>;
   else if (A.split) k = A.fanout ? culi_eval_kernel<true, false, true> : culi_eval_kernel<false, false, true>;
+  else if (A.voting && A.code_n == 0) k = A.fanout ? culi_eval_vote_kernel<true> : culi_eval_vote_kernel<false>;
   else k = A.fanout ? culi_eval_kernel<true, false, false> : culi_eval_kernel<false, false, false>;
   if (smem > 48 * 1024) {
     cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);

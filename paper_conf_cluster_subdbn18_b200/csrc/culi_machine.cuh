@@ -963,21 +963,28 @@ struct FormOut {
   uint64_t w;
   uint64_t steps;
   uint8_t err;
-  uint32_t aux;        // E_SUSPEND: index of the nested-||| descriptor
+  uint32_t aux;        // E_SUSPEND: index of the nested-||| descriptor; E_YIELD: stack height
+  uint32_t vtop;       // E_YIELD: V-stack top
+  uint32_t kk;         // E_YIELD: kind of the continuation about to be popped
 };
 
-// state to resume a suspended evaluation at RET with value v (the nested |||'s result)
+// state to resume a suspended evaluation at RET with value v (the nested |||'s result, or the value a
+// yielding lane was about to return); grp / wait: VOTE mode, see eval_form
 struct Resume {
   uint32_t sp, vtop;
   uint64_t steps;
   V v;
+  uint32_t grp, wait;
 };
 
 // eval_form(C, root, form, 0, 0, fuel): evaluate the datum at node `root` at depth 1.
 // eval_form(C, 0, form, 1, m, budget): apply vs[0] to the m values vs[1..m] as the body of a top-level
 //   (||| ...) form (depth 1) — one fan-out element (c.7); `budget` = fuel left after the ||| arguments.
 // eval_form<..., SPLIT>(C, root, form, 0, 0, budget, depth, false, {}, env): a split-off argument task.
-template <bool FANOUT, bool APPLY, bool NEST = false, bool SPLIT = false>
+// VOTE: the lanes of R.grp run together; at a return, a lane yields (E_YIELD, state in FormOut) when its
+// group is no longer converged (__activemask() != grp) or its stack is back down to the height R.wait of
+// the deepest waiting lane, where the two groups can continue as one.
+template <bool FANOUT, bool APPLY, bool NEST = false, bool SPLIT = false, bool VOTE = false>
 __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32_t form, int apply_mode,
                                              uint32_t apply_cnt, uint64_t fuel, uint32_t d0 = 1,
                                              bool resume = false, const Resume& R = Resume{},
@@ -994,7 +1001,7 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32
   uint4 k, ktop = make_uint4(0, 0, 0, 0);
   uint4 hv = make_uint4(0, 0, 0, 0);      // the value being applied (copy of vs[base])
   bool kdirty = false;                      // ktop holds frame sp-1 not yet written to memory
-  uint32_t pollc = SPLIT ? C.A->split_poll : 0;   // closure calls until the next split poll
+  uint32_t pollc = SPLIT ? C.A->split_first : 0;  // closure calls until the next split poll
 
 #define FAIL(e) do { err = (e); goto done; } while (0)
 // setq batches (R7): a frame moves to the heap as soon as it is made, so that no copy of it can go stale
@@ -1018,13 +1025,13 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32
 #define ATOMVAL(n, tt, ww) (((tt) & KIND_MASK) == K_SYM ? lookup(C, (uint32_t)(ww), env) : unbox_loaded((n), (tt), (ww)))
 
   uint32_t aux = 0;
-  if (NEST && resume) {                                         // continue a suspended evaluation
+  if ((NEST || VOTE) && resume) {                               // continue a suspended evaluation
     sp = R.sp;
     vtop = R.vtop;
     steps = R.steps;
     v = R.v;
     if (sp > 0) ktop = *KS(C, sp - 1);
-    goto RET;
+    goto RET_POP;                                               // (no yield check: make progress first)
   }
   if (APPLY && apply_mode) {
     base = 0;
@@ -1327,6 +1334,13 @@ IF_BRANCH:
   // ======================================================== return v to the top continuation
 RET:
   if (sp == 0) goto done;
+  if (VOTE && (__activemask() != R.grp || sp <= R.wait)) {      // diverged, or level with a waiting group
+    if (kdirty) *KS(C, sp - 1) = ktop;
+    err = E_YIELD;
+    goto done;
+  }
+RET_POP:
+  if (NEST && sp == 0) goto done;
   k = ktop;
   --sp;
   if (sp > 0) ktop = *KS(C, sp - 1);                            // consumed at the next return
@@ -1676,6 +1690,11 @@ done:
   o.steps = steps;
   o.err = err;
   o.aux = aux;
+  if (VOTE && err == E_YIELD) {
+    o.aux = sp;
+    o.vtop = vtop;
+    o.kk = kkind(ktop.w);
+  }
   return o;
 }
 

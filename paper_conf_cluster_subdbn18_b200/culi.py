@@ -33,9 +33,10 @@ SYMBOLS = [
     "culi_result_int", "culi_result_float", "culi_print", "culi_results_totals", "culi_results_free",
     "culi_env_export", "culi_env_import", "culi_results_serialize", "culi_results_merge",
     "culi_status_string", "culi_error_name", "culi_last_timing", "culi_records_device",
-    "culi_last_stats", "culi_last_splits", "culi_last_waits", "culi_image_pin", "culi_results_wire_bytes",
+    "culi_last_stats", "culi_last_splits", "culi_last_waits", "culi_last_reruns", "culi_image_pin", "culi_results_wire_bytes",
     "culi_define_text", "culi_eval_text", "culi_upload_text", "culi_last_read", "culi_collect",
-    "culi_heap_usage",
+    "culi_heap_usage", "culi_arena_bytes", "culi_eval_batch_async", "culi_sync", "culi_complete",
+    "culi_results_export", "culi_results_import",
 ]
 
 
@@ -48,7 +49,8 @@ class CuliError(RuntimeError):
 class culi_opts(ctypes.Structure):
     _fields_ = [("device", ctypes.c_int), ("stream", ctypes.c_void_p), ("heap_nodes", ctypes.c_uint64),
                 ("max_depth", ctypes.c_uint32), ("fuel", ctypes.c_uint64),
-                ("vstack_entries", ctypes.c_uint32), ("slots", ctypes.c_uint32), ("flags", ctypes.c_uint32)]
+                ("vstack_entries", ctypes.c_uint32), ("slots", ctypes.c_uint32), ("flags", ctypes.c_uint32),
+                ("heap_base", ctypes.c_void_p), ("heap_bytes", ctypes.c_uint64)]
 
 
 _lib = None
@@ -96,6 +98,7 @@ def load(path: str = LIB_PATH) -> ctypes.CDLL:
         "culi_last_stats": (I, [P, pp(U32), pp(U32), pp(U32)]),
         "culi_last_splits": (I, [P, pp(U32)]),
         "culi_last_waits": (I, [P, pp(U32), pp(U32)]),
+        "culi_last_reruns": (I, [P, pp(U32), pp(U32)]),
         "culi_image_pin": (I, [P, pp(U64)]),
         "culi_results_wire_bytes": (I, [P, pp(U64)]),
         "culi_define_text": (I, [P, P, SZ, I, pp(U32), pp(ctypes.c_uint8), pp(SZ)]),
@@ -104,6 +107,12 @@ def load(path: str = LIB_PATH) -> ctypes.CDLL:
         "culi_last_read": (I, [P, pp(ctypes.c_float), pp(U64), pp(U64)]),
         "culi_collect": (I, [P, pp(U64), pp(U64)]),
         "culi_heap_usage": (I, [P, pp(U64), pp(U64), pp(U64)]),
+        "culi_arena_bytes": (I, [pp(culi_opts), pp(U64)]),
+        "culi_eval_batch_async": (I, [P, P, pp(P)]),
+        "culi_sync": (I, [P]),
+        "culi_complete": (I, [P, U32]),
+        "culi_results_export": (I, [P, P, SZ, pp(SZ)]),
+        "culi_results_import": (I, [P, pp(P), pp(SZ), I, pp(pp(U32)), pp(P)]),
     }
     for name, (res, args) in sig.items():
         fn = getattr(L, name)
@@ -245,7 +254,9 @@ class Context:
 
     def __init__(self, device: int = 0, stream: int | None = None, heap_nodes: int = 0,
                  max_depth: int = 0, fuel: int = 0, vstack_entries: int = 0, slots: int = 0,
-                 flags: int = 0):
+                 flags: int = 0, arena=None):
+        """arena: optional caller-owned device memory (a CUDA uint8 tensor of at least
+        Context.arena_bytes(...) bytes) for the heap, global frame, strings and stacks (culi_opts.heap_base)."""
         L = load()
         o = culi_opts()
         L.culi_default_opts(ctypes.byref(o))
@@ -257,6 +268,10 @@ class Context:
         o.vstack_entries = vstack_entries
         o.slots = slots
         o.flags = flags
+        self._arena = arena                      # keep the caller's tensor alive as long as the ctx
+        if arena is not None:
+            o.heap_base = arena.data_ptr()
+            o.heap_bytes = arena.numel() * arena.element_size()
         self.opts = o
         p = ctypes.c_void_p()
         _check(L.culi_init(ctypes.byref(o), ctypes.byref(p)), "culi_init")
@@ -407,6 +422,70 @@ class Context:
         d = (ctypes.c_uint32 * 9)()
         _check(load().culi_last_waits(self._p, ctypes.byref(n), d), "culi_last_waits")
         return n.value, list(d)
+
+    @staticmethod
+    def arena_bytes(device: int = 0, heap_nodes: int = 0, max_depth: int = 0, vstack_entries: int = 0,
+                    slots: int = 0) -> int:
+        """Bytes a caller-owned arena needs for these sizes (culi_arena_bytes)."""
+        o = culi_opts()
+        load().culi_default_opts(ctypes.byref(o))
+        o.device, o.heap_nodes, o.max_depth, o.vstack_entries, o.slots = device, heap_nodes, max_depth, \
+            vstack_entries, slots
+        b = ctypes.c_uint64(0)
+        _check(load().culi_arena_bytes(ctypes.byref(o), ctypes.byref(b)), "culi_arena_bytes")
+        return b.value
+
+    def eval_batch_async(self, forms: str | bytes | Image) -> "Results":
+        """Start a batch (culi_eval_batch_async); the results are ready after sync()."""
+        img = forms if isinstance(forms, Image) else self.read(forms)
+        out = ctypes.c_void_p()
+        _check(load().culi_eval_batch_async(self._p, img._p, ctypes.byref(out)), "culi_eval_batch_async")
+        r = Results(out.value)
+        r._image = img                           # the image must live until culi_sync
+        return r
+
+    def sync(self) -> None:
+        _check(load().culi_sync(self._p), "culi_sync")
+
+    def complete(self, handle: int) -> None:
+        """Finish the uploaded batch's device-resident results (fallbacks, payload regrowth), no D2H."""
+        _check(load().culi_complete(self._p, handle), "culi_complete")
+
+    def results_export_size(self) -> int:
+        need = ctypes.c_size_t(0)
+        _check(load().culi_results_export(self._p, None, 0, ctypes.byref(need)), "culi_results_export")
+        return need.value
+
+    def results_export(self, dev_ptr: int, cap: int) -> int:
+        """Pack the current batch's device-resident results into dev_ptr[cap] (stream-ordered, no sync)."""
+        used = ctypes.c_size_t(0)
+        _check(load().culi_results_export(self._p, ctypes.c_void_p(dev_ptr), cap, ctypes.byref(used)),
+               "culi_results_export")
+        return used.value
+
+    def results_import(self, dev_ptrs: list[int], sizes: list[int],
+                       form_index: list[list[int]] | None = None) -> "Results":
+        """Merge per-rank exported device buffers into one host result set (None: strided deal)."""
+        n = len(dev_ptrs)
+        ptrs = (ctypes.c_void_p * n)(*dev_ptrs)
+        szs = (ctypes.c_size_t * n)(*sizes)
+        idx = None
+        keep = []
+        if form_index is not None:
+            arrs = [(ctypes.c_uint32 * len(ix))(*ix) for ix in form_index]
+            keep = arrs
+            idx = (ctypes.POINTER(ctypes.c_uint32) * n)(*[ctypes.cast(a, ctypes.POINTER(ctypes.c_uint32))
+                                                         for a in arrs])
+        out = ctypes.c_void_p()
+        _check(load().culi_results_import(self._p, ptrs, szs, n, idx, ctypes.byref(out)), "culi_results_import")
+        del keep
+        return Results(out.value)
+
+    def last_reruns(self) -> tuple[int, int]:
+        """(forms re-evaluated by the sequential fallback, payload-buffer regrowths) of the last fetch."""
+        a, b = ctypes.c_uint32(), ctypes.c_uint32()
+        _check(load().culi_last_reruns(self._p, ctypes.byref(a), ctypes.byref(b)), "culi_last_reruns")
+        return a.value, b.value
 
     def records_device(self, dev_ptr: int | None, cap: int = 0) -> int:
         need = ctypes.c_size_t(0)

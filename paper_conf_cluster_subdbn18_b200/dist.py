@@ -6,6 +6,10 @@ gloo in the CPU tests).  The collectives move opaque byte buffers produced and c
     strings, symbol names), broadcast from rank 0 once per session;
   * culi_results_serialize / culi_results_merge — per-rank results gathered to every rank and rebuilt in
     global form order (symbols re-interned by name).
+  * culi_results_export / culi_results_import — the device-resident gather (the default): each rank packs
+    its records + payload + names into a fixed-size device buffer (no host sync), one all_gather of the
+    padded buffers (NCCL: device to device over NVLink), and the destination rank merges them on its GPU
+    (records scattered by form index, payload offsets shifted, symbols re-interned) with one D2H.
 No collective runs inside the eval kernel: the path has one exchange before and one after the batch.
 """
 from __future__ import annotations
@@ -89,3 +93,43 @@ def gather_results(results, nforms: int, group=None):
     blobs = all_gather_bytes(results.serialize(), group=group)
     idx = [shard_indices(nforms, r, world) for r in range(world)]
     return culi.merge_results(blobs, idx)
+
+
+def all_gather_device(buf: torch.Tensor, group=None) -> torch.Tensor:
+    """all_gather_into_tensor of equal-size device buffers; gloo (CPU tests) stages through host memory."""
+    world = dist.get_world_size(group)
+    out = torch.empty(world * buf.numel(), dtype=buf.dtype, device=buf.device)
+    if _buffer_device(group).type == "cuda":
+        dist.all_gather_into_tensor(out, buf, group=group)
+    else:
+        h = torch.empty(world * buf.numel(), dtype=buf.dtype)
+        dist.all_gather_into_tensor(h, buf.cpu(), group=group)
+        out.copy_(h)
+    return out
+
+
+def export_capacity(ctx, group=None, slack: float = 1.25) -> int:
+    """Common export-buffer size: the largest exact size over the ranks, with room for payload growth."""
+    dev = _buffer_device(group)
+    n = torch.tensor([ctx.results_export_size()], dtype=torch.int64, device=dev)
+    dist.all_reduce(n, op=dist.ReduceOp.MAX, group=group)
+    return (int(int(n.item()) * slack) + 4095) // 4096 * 4096
+
+
+def gather_results_device(ctx, cap: int, dst: int | None = 0, group=None, buf: torch.Tensor | None = None):
+    """Device-resident gather of the current batch's results (strided shards).  Every rank
+    exports into `cap` bytes, one all_gather, rank `dst` (every rank if None) imports.  Returns the merged
+    Results on the importing rank(s), else None."""
+    dev = torch.device("cuda", torch.cuda.current_device())
+    world = dist.get_world_size(group)
+    if buf is None:
+        buf = torch.empty(cap, dtype=torch.uint8, device=dev)
+    ctx.results_export(buf.data_ptr(), cap)
+    if _buffer_device(group).type != "cuda":
+        torch.cuda.synchronize()                 # gloo reads the buffer on the host
+    out = all_gather_device(buf, group=group)
+    if dst is not None and dist.get_rank(group) != dst:
+        return None
+    torch.cuda.synchronize()
+    ptrs = [out.data_ptr() + r * cap for r in range(world)]
+    return ctx.results_import(ptrs, [cap] * world, None)

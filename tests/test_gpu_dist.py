@@ -43,8 +43,15 @@ def _worker(rank, world, port, defs, forms, q):
         shard, idx = W.shard_lines(forms, rank, world)
         assert idx == D.shard_indices(nforms, rank, world)
         res = ctx.eval_batch(shard)
-        merged = D.gather_results(res, nforms)
-        q.put((rank, nbytes, merged.printed(), merged.steps()))
+        merged = D.gather_results(res, nforms)               # host-serialized blobs (reference path)
+        # device-resident gather (culi_results_export / culi_results_import): no Python bytes
+        h = ctx.upload(shard)
+        ctx.eval_uploaded(h)
+        ctx.complete(h)
+        cap = D.export_capacity(ctx)
+        dm = D.gather_results_device(ctx, cap, dst=None)
+        ctx.release(h)
+        q.put((rank, nbytes, merged.printed(), merged.steps(), dm.printed(), dm.steps()))
     finally:
         dist.destroy_process_group()
 
@@ -74,7 +81,8 @@ def test_two_ranks_broadcast_shard_gather(oracle_mod):
     s = oracle_mod.Session()
     s.define(defs)
     o = s.eval(forms)
-    for rank, nbytes, printed, steps in outs:
+    for rank, nbytes, printed, steps, dprinted, dsteps in outs:
         assert nbytes > 0
         bad = compare(printed, steps, o, forms.splitlines())
         assert not bad, "\n".join(bad)
+        assert (dprinted, dsteps) == (printed, steps)
