@@ -263,17 +263,20 @@ int culi_last_timing(const culi_ctx* ctx, float* ms3, uint32_t* kernels, uint64_
 int culi_last_stats(const culi_ctx* ctx, uint32_t* fanout_forms, uint32_t* fallback_forms,
                     uint32_t* nested_forms);
 /* Argument splitting (an implementation choice, not a paper mechanism): the number of
- * split groups the last fetched batch published — each group is up to 32 pending arguments of one warp
- * that an idle warp offered to evaluate (evaluated by it, or taken back by the owners).  Results, steps
- * and errors are identical with CULI_F_NO_SPLIT.  0 for batches that do not split (see the note after
- * the CULI_F_* flags). */
+ * split groups the last fetched batch published — each group is the pending arguments of the lanes of one
+ * warp that polled together while an idle warp waited for work; the idle warp evaluates the group (or the
+ * owners take it back).  Results, steps and errors are identical with CULI_F_NO_SPLIT.  0 for batches that
+ * do not split (see the note after the CULI_F_* flags). */
 int culi_last_splits(const culi_ctx* ctx, uint32_t* groups);
-/* Every wait of one warp on another (an owner joining a split argument, a thief reading a queue entry, a
+/* Of those, the groups an idle warp claimed and evaluated (the others were taken back by their owners). */
+int culi_last_split_claims(const culi_ctx* ctx, uint32_t* claimed);
+/* Every wait of one lane on another (an owner joining a split argument, a thief waiting for its group, a
  * nested ||| waiting for its elements) is bounded by 10 s (env CULI_WAIT_MS).  A wait that gives up
  * recovers exactly — the owner evaluates the argument itself / the form goes to the sequential fallback —
  * so results are unaffected; it is counted here for the last fetched batch (*timeouts; 0 in a healthy
  * run), and diag9 (if non-NULL, 9 entries) receives the first one's state: kind (1 join, 2 queue entry,
- * 3 nested), group, lane, form, group state, task mask, owners remaining, task done flag, thief warp. */
+ * 3 nested), group (or descriptor), lane, form, group state, task mask, owners remaining, task done
+ * flag, thief warp. */
 int culi_last_waits(const culi_ctx* ctx, uint32_t* timeouts, uint32_t* diag9);
 /* Work the last fetch (culi_fetch_results / culi_eval_batch / culi_eval_text) did after the device step it
  * fetched: forms re-evaluated by the sequential fallback (as culi_last_stats), and re-runs of eval + export

@@ -23,7 +23,11 @@ def _stale(target: str, deps: list[str]) -> bool:
     return any(os.path.getmtime(d) > t for d in deps)
 
 
-def build(verbose: bool = False, force: bool = False, ptxas_v: bool = False) -> str:
+def build(verbose: bool = False, force: bool = False, ptxas_v: bool = False, defines: list[str] | None = None,
+          out: str | None = None) -> str:
+    """defines / out: debug or A/B variants (e.g. ["CULI_WATCHDOG=20000"], "scratch/libculi_wd.so")."""
+    if defines or out:
+        return _build_variant(defines or [], out or LIB, verbose)
     if HERE not in sys.path:
         sys.path.insert(0, HERE)
     import gen_pow5
@@ -46,6 +50,21 @@ def build(verbose: bool = False, force: bool = False, ptxas_v: bool = False) -> 
     for o in objs:
         os.remove(o)
     return LIB
+
+
+def _build_variant(defines: list[str], out: str, verbose: bool) -> str:
+    import tempfile
+    tmp = tempfile.mkdtemp()
+    objs = []
+    for src in SOURCES:
+        obj = os.path.join(tmp, src + ".o")
+        cmd = [NVCC, *ARCH, *FLAGS, *["-D" + d for d in defines], "-c", os.path.join(CSRC, src), "-o", obj]
+        if verbose:
+            print(" ".join(cmd), file=sys.stderr)
+        subprocess.check_call(cmd)
+        objs.append(obj)
+    subprocess.check_call([NVCC, *ARCH, "-shared", "-o", out, *objs, "-lcudart"])
+    return out
 
 
 if __name__ == "__main__":

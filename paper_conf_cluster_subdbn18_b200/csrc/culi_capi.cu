@@ -4,6 +4,7 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <cstdio>
 #include <cstdlib>
 #include <cstring>
 #include <memory>
@@ -120,6 +121,7 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   if (const char* e = getenv("CULI_SPLIT_POLL")) c->split_poll = std::max(1, atoi(e));      // tuning knobs
   if (const char* e = getenv("CULI_SPLIT_FIRST")) c->split_first = std::max(1, atoi(e));
   if (const char* e = getenv("CULI_SPLIT_SLEEP")) c->split_sleep = std::max(32, atoi(e));
+  if (const char* e = getenv("CULI_STEAL_GATE")) c->steal_gate = atoi(e) != 0;
   if (const char* e = getenv("CULI_WAIT_MS")) c->wait_ns = (unsigned long long)std::max(1, atoi(e)) * 1000000ull;
   bool ok = true;
   if (o.heap_base) {                                 // caller-owned arena (e.g. a torch tensor)
@@ -329,6 +331,7 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   }
   A.split_poll = c->split_poll;
   A.split_first = c->split_first;
+  A.steal_gate = c->steal_gate;
   A.split_sleep = c->split_sleep;
   A.groups = c->groups;
   A.gqueue = c->gqueue;
@@ -642,7 +645,15 @@ static int complete_device(culi_ctx* c, unsigned long long* pc_out) {
       c->last_nested = c->batch_may_nest ? std::min(nnest, c->maxnest) : 0;
       c->last_splits = sc.published;
       c->last_timeouts = sc.timeouts;
+      c->last_claimed = sc.claimed;
+      if (getenv("CULI_SPLIT_STATS"))
+        fprintf(stderr, "[culi split] groups published %u claimed %u; idle rounds %u (lanes missing %u)\n",
+                sc.published, sc.claimed, sc.stat[0], sc.stat[1]);
       std::memcpy(c->last_diag, sc.diag, sizeof sc.diag);
+#if CULI_WATCHDOG
+      if (sc.wd[0]) fprintf(stderr, "[culi watchdog] %u lanes fired; first: form %u steps(lo) %u sp %u depth %u root %u thief %u finished %u\n",
+                            sc.wd[0], sc.wd[1], sc.wd[2], sc.wd[3], sc.wd[4], sc.wd[5], sc.wd[6], sc.wd[7]);
+#endif
     }
     if (nfb && !flags[3]) {
       c->last_fallback += nfb;
@@ -959,6 +970,12 @@ int culi_last_stats(const culi_ctx* c, uint32_t* fanout_forms, uint32_t* fallbac
 int culi_last_splits(const culi_ctx* c, uint32_t* groups) {
   if (!c || !groups) return CULI_E_ARG;
   *groups = c->last_splits;
+  return CULI_OK;
+}
+
+int culi_last_split_claims(const culi_ctx* c, uint32_t* claimed) {
+  if (!c || !claimed) return CULI_E_ARG;
+  *claimed = c->last_claimed;
   return CULI_OK;
 }
 

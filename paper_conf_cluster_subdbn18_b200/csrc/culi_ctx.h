@@ -150,14 +150,16 @@ struct culi_ctx {
   // argument splitting
   SplitGroup* groups = nullptr;      // SPLIT_GPW per warp of the grid
   unsigned long long* gqueue = nullptr;
-  uint32_t gqcap = 1u << 18;
+  uint32_t gqcap = 1u << 18;         // > outstanding tickets (<= warps of the grid + racing publishers)
   SplitCtl* sctl = nullptr;          // queue counters (persist across launches), tokens, stats, diagnostics
   unsigned long long wait_ns = 10ull * 1000 * 1000 * 1000;   // bounded inter-warp waits (env CULI_WAIT_MS)
   uint32_t last_timeouts = 0;
+  uint32_t last_claimed = 0;         // split tasks a thief claimed in the last fetch
   uint32_t last_regrows = 0;         // payload-buffer regrowths (eval + export re-run) in the last fetch
   uint32_t last_diag[9] = {0};
   uint32_t split_poll = 64;          // closure calls between polls (env CULI_SPLIT_POLL)
   uint32_t split_first = 64;         // closure calls before the first poll (env CULI_SPLIT_FIRST)
+  uint32_t steal_gate = 1;           // steal only from fully idle warps (env CULI_STEAL_GATE)
   uint32_t split_sleep = 4096;       // idle-warp back-off cap in ns (env CULI_SPLIT_SLEEP)
   DevBuf<uint32_t> wide;
   // uploaded batch (culi_upload)

@@ -88,8 +88,9 @@ struct EvalArgs {
   uint32_t split;              // argument splitting: idle warps evaluate pending arguments of busy ones
   uint32_t split_poll;         // closure calls between two polls of the idle-warp counter
   uint32_t split_first;        // closure calls before an evaluation's first poll (split the top of the tree early)
-  uint32_t split_sleep;        // longest back-off (ns) of an idle warp polling for split groups
-  struct SplitGroup* groups;   // SPLIT_GPW group slots per warp of the grid (slot reused after its join)
+  uint32_t split_sleep;        // longest back-off (ns) of an idle warp waiting for its ticket's group
+  uint32_t steal_gate;         // idle lanes steal only when their whole warp is idle
+  struct SplitGroup* groups;   // SPLIT_GPW group slots per warp of the grid
   unsigned long long* gqueue;  // ring of published groups: ticket << 32 | (group + 1), gqcap entries
   uint32_t gqcap;              // power of two
   struct SplitCtl* sctl;       // queue counters, idle-warp tokens, statistics, bounded-wait diagnostics
@@ -139,40 +140,54 @@ struct NestDesc {
   uint32_t next, done, bad, ready;            // ready: fields published, elements claimable
 };
 
-// Argument splitting.  A busy warp that sees idle warps turns the lowest pending
-// argument of each lane's K-stack (the biggest unevaluated chunk: the next argument of the outermost
-// KF_ARGS frame) into a task; an idle warp claims the whole group and lane i evaluates task i.  Arguments
-// are pure (no mutation inside a batch, c.3/c.13 #25), so only steps, the first error and fuel need care:
-// the owner adds the task's steps at the join and decides errors/fuel exactly (c.4, c.10).
+// Argument splitting.  When idle warps wait for work, the lanes of a busy warp that poll
+// together turn the lowest pending argument of their K-stacks (the biggest unevaluated chunk: the next
+// argument of the outermost KF_ARGS frame) into tasks, one group per poll, published with one ticket; an
+// idle warp holding that ticket claims the whole group and its lanes evaluate the tasks on their own
+// stacks.  Arguments are pure (no mutation inside a batch, c.3/c.13 #25), so only steps, the first error
+// and fuel need care: each owner lane adds its task's steps at the join and decides errors/fuel exactly
+// (c.4, c.10).  A group is claimed or taken back as a whole, so the owner lanes of a converged warp stay
+// converged.  No warp-wide barrier takes part (round 1 deadlocked on one): the idle
+// warps' rounds use a shared-memory counter, and the only warp intrinsics are a ballot and shuffles over
+// __activemask() with no other collective in between.
 struct SplitTask {
   uint32_t expr, env, depth, pad;      // argument node, heap env, depth of its evaluation
   unsigned long long budget;           // fuel left at the fork
   unsigned long long rw, rsteps;       // result word, steps
   uint32_t rt, rerr, done, pad2;
+  uint32_t pad3[2];
 };
+static_assert(sizeof(SplitTask) == 64, "one task per 64-byte line");
 struct SplitGroup {
-  uint32_t state;                      // 0 open, 1 claimed by a thief warp, 2 taken back by the owners
+  uint32_t state;                      // SPLIT_OPEN / SPLIT_CLAIMED / SPLIT_TAKEN
   uint32_t remaining;                  // owner lanes that have not joined yet (0: the slot is free again)
   uint32_t mask;                       // lanes with a task
   uint32_t form;
   uint32_t claimer;                    // global warp id of the thief (diagnostics)
-  uint32_t pad[3];
+  uint32_t pad[11];
   SplitTask t[32];
 };
-constexpr uint32_t SPLIT_GPW = 8;      // group slots per warp
-// Queue counters live across launches: tickets are never reused, so an entry left in the ring by an earlier
-// launch (or an earlier lap of the ring) can never be mistaken for the one a thief is waiting for; the reset
-// kernel drops unclaimed entries by setting head = tail.
+constexpr uint32_t SPLIT_GPW = 8;      // group slots per warp (outstanding polls of one warp)
+constexpr uint32_t SPLIT_OPEN = 0, SPLIT_CLAIMED = 1, SPLIT_TAKEN = 2;
+// Ticket queue (a FAA queue): an idle warp takes ticket h = head++ and waits for the entry stamped h; busy
+// warps publish while head > tail (an idle warp waits) at ticket q = tail++.  Counters live across
+// launches and tickets are never reused, so an entry left by an earlier launch (or lap of the ring) never
+// matches; the reset kernel sets head = tail = max.  Outstanding tickets <= warps < ring capacity.
 struct SplitCtl {
   unsigned long long tail;             // tickets handed out to publishers (monotonic)
-  unsigned long long head;             // next ticket a thief takes
-  int hungry;                          // idle thief warps minus open groups (owners split while > 0)
+  unsigned long long head;             // tickets handed out to idle lanes (monotonic)
   uint32_t published;                  // groups published in this launch (statistics)
   uint32_t timeouts;                   // bounded waits that gave up in this launch (0 in a healthy run)
   uint32_t diag[9];                    // the first one: kind, group, lane, form, state, mask, remaining, done, claimer
+  uint32_t claimed;                    // groups an idle warp claimed (the rest were taken back by their owners)
+  uint32_t stat[4];                    // statistics: thief rounds, rounds with < 32 lanes present, -, -
+  unsigned long long t0;               // globaltimer at the launch's reset (debug watchdog, CULI_WATCHDOG builds)
+  uint32_t wd[8];                      // debug watchdog: count, form, steps lo, sp, depth, root, thief, finished
 };
 constexpr uint32_t WAIT_JOIN = 1, WAIT_QUEUE = 2, WAIT_NEST = 3;
-constexpr uint32_t SPLIT_OPEN = 0, SPLIT_CLAIMED = 1, SPLIT_TAKEN = 2;
+#ifndef CULI_WATCHDOG
+#define CULI_WATCHDOG 0            // debug builds: forms running past CULI_WATCHDOG ms fail and are recorded
+#endif
 
 struct ExportArgs {
   const uint8_t* tag;

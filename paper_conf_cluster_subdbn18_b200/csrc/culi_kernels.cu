@@ -98,53 +98,78 @@ __device__ __forceinline__ bool nest_help_any(const EvalArgs& A, const Ctx& C2, 
   return false;
 }
 
-// ---- argument splitting: a warp with no form left is a thief -----------------------------
-// It has offered itself (A.sctl->hungry += 1); lane 0 takes tickets in order (queue head) and claims the
-// group of the entry stamped with that ticket.  Returns the group, or 0xffffffff once every form of the
-// batch is finished.  Idle warps back off exponentially (up to A.split_sleep ns) so that they do not hammer
-// the L2 line of the queue counters.  An entry whose group is no longer open (taken back by its owners, or
-// reused and already claimed) is skipped; so is a ticket whose entry does not appear within A.wait_ns.
-__device__ __noinline__ uint32_t split_claim(const EvalArgs& A) {
+// ---- argument splitting: a warp with no form left steals ----------------------------
+// Its lanes, once every lane of the warp is idle, work in rounds, coordinated through shared memory only
+// (no warp intrinsic: lanes of a warp in different spin loops must never meet in a collective): each lane
+// arrives at the warp's round counter; the last to arrive is the round's leader, takes ticket h = head++,
+// waits for the entry stamped h and claims its group (OPEN -> CLAIMED) unless the owners took it back
+// first, then publishes the result in the warp's mailbox and bumps the round generation; the others wait
+// for the generation.  All 32 lanes are in every round, so lane i runs task i of the group (owner lane i's
+// argument: converged, like the owners).  Returns the group, 0xfffffffe for no group this round, or
+// 0xffffffff once every form of the batch is finished.  Waits back off exponentially (A.split_sleep ns).
+__shared__ uint32_t culi_warp_idle[4];       // lanes of each warp with no form left (kernel prologue: 0)
+__shared__ uint32_t culi_warp_round[4];      // arrivals at the idle warps' round barrier
+__shared__ uint32_t culi_warp_gen[4];        // rounds whose group is in the mailbox
+__shared__ uint32_t culi_warp_mail[4];       // the round's group (or 0xfffffffe / 0xffffffff)
+
+__device__ __noinline__ uint32_t claim_group(const EvalArgs& A) {
   SplitCtl* Q = A.sctl;
+  unsigned long long h = atomicAdd(&Q->head, 1ull);
+  const unsigned long long* qe = &A.gqueue[h & (A.gqcap - 1)];
   uint32_t ns = 64;
-  for (;;) {
-    unsigned long long h = *(volatile unsigned long long*)&Q->head;
-    unsigned long long n = *(volatile unsigned long long*)&Q->tail;
-    if (h < n) {
-      if (atomicCAS(&Q->head, h, h + 1) == h) {
-        unsigned long long* qe = &A.gqueue[h & (A.gqcap - 1)];
-        unsigned long long e = 0, t0 = 0;
-        bool ok = true;
-        for (uint32_t spin = 1;; ++spin) {
-          asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(e) : "l"(qe) : "memory");
-          if ((uint32_t)(e >> 32) == (uint32_t)h && (uint32_t)e != 0) break;
-          __nanosleep(32);
-          if ((spin & 63) == 0) {
-            unsigned long long now = gtime();
-            if (!t0) t0 = now;
-            else if (now - t0 > A.wait_ns) { wait_gave_up(A, WAIT_QUEUE, (uint32_t)h, 0); ok = false; break; }
-          }
-        }
-        uint32_t g = (uint32_t)e - 1;
-        if (ok && atomicCAS(&A.groups[g].state, SPLIT_OPEN, SPLIT_CLAIMED) == SPLIT_OPEN) {
-          A.groups[g].claimer = (blockIdx.x * blockDim.x + threadIdx.x) >> 5;
-          return g;
-        }
-      }
-      ns = 64;
-      continue;
+  for (uint32_t spin = 0;; ++spin) {
+    unsigned long long e = ld_acquire64(qe);
+    if ((uint32_t)(e >> 32) == (uint32_t)h && (uint32_t)e != 0) {   // (0: never written)
+      uint32_t g = (uint32_t)e - 1;
+      if (atomicCAS(&A.groups[g].state, SPLIT_OPEN, SPLIT_CLAIMED) != SPLIT_OPEN) return 0xfffffffeu;
+      A.groups[g].claimer = my_slot() >> 5;
+      atomicAdd(&Q->claimed, 1u);
+      return g;
     }
-    if (*(volatile uint32_t*)A.finished >= A.nforms) return 0xffffffffu;
+    if ((spin & 7) == 0 && *(volatile uint32_t*)A.finished >= A.nforms) return 0xffffffffu;
+#if CULI_WATCHDOG
+    if (gtime() - *(volatile unsigned long long*)&Q->t0 > (unsigned long long)CULI_WATCHDOG * 1000000ull + 2000000000ull) {
+      if (atomicAdd(&Q->wd[0], 1u) == 0) { Q->wd[6] = 1; Q->wd[7] = *(volatile uint32_t*)A.finished; }
+      return 0xffffffffu;
+    }
+#endif
     __nanosleep(ns);
     ns = ns * 2 > A.split_sleep ? A.split_sleep : ns * 2;
   }
 }
 
+__device__ __noinline__ uint32_t split_claim(const EvalArgs& A, uint32_t& round) {
+  uint32_t w = threadIdx.x >> 5;
+  uint32_t r = ++round;
+  // wait until the whole warp is idle (the first round only has to)
+  for (uint32_t ns = 64; A.steal_gate && *(volatile uint32_t*)&culi_warp_idle[w] < 32;) {
+    if (*(volatile uint32_t*)A.finished >= A.nforms) return 0xffffffffu;
+    __nanosleep(ns);
+    ns = ns * 2 > A.split_sleep ? A.split_sleep : ns * 2;
+  }
+  if (atomicAdd(&culi_warp_round[w], 1u) == 32u * r - 1u) {   // last to arrive: this round's leader
+    uint32_t g = claim_group(A);
+    *(volatile uint32_t*)&culi_warp_mail[w] = g;
+    __threadfence_block();
+    *(volatile uint32_t*)&culi_warp_gen[w] = r;
+    return g;
+  }
+  for (uint32_t ns = 64; *(volatile uint32_t*)&culi_warp_gen[w] < r;) {
+    // (a lane that found every form finished leaves without arriving: so does everyone after it)
+    if (*(volatile uint32_t*)A.finished >= A.nforms) return 0xffffffffu;
+    __nanosleep(ns);
+    ns = ns * 2 > A.split_sleep ? A.split_sleep : ns * 2;
+  }
+  __threadfence_block();
+  return *(volatile uint32_t*)&culi_warp_mail[w];
+}
+
 // Batch mode.  Shared memory per block: the persistent code segment [code_lo, code_lo + code_n) as
-// {w.lo, w.hi, tag, 0} and the global frame [0, gst) ("stage").  Each warp takes 32
-// consecutive forms of the (binned) order with one atomicAdd and runs them to completion.  With SPLIT, a
-// warp that finds no form left becomes a thief: lane i of it evaluates task i of a claimed split group on
-// the warp's own stacks (one eval_form call site serves forms and tasks).
+// {w.lo, w.hi, tag, 0} and the global frame [0, gst) ("stage").  Every lane takes its next
+// form with a warp-aggregated counter (converged lanes of the binned order get consecutive forms) and runs
+// it to completion; no warp-wide barrier anywhere, so diverged lanes never wait on each other.  With SPLIT,
+// a lane that finds no form left is a thief: it evaluates split-off arguments of busy lanes on its own
+// stacks (one eval_form call site serves forms and tasks).
 template <bool FANOUT, bool NEST, bool SPLIT>
 __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(const __grid_constant__ EvalArgs A) {
   uint4* scode = culi_smem;
@@ -158,9 +183,14 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
     sgword[i] = A.H.gword[i];
     sgtag[i] = A.H.gtag[i];
   }
-  if (SPLIT && threadIdx.x < 4) culi_split_busy[threadIdx.x] = 0;
+  if (SPLIT && threadIdx.x < 4) {
+    culi_split_busy[threadIdx.x] = 0;
+    culi_warp_idle[threadIdx.x] = 0;
+    culi_warp_round[threadIdx.x] = 0;
+    culi_warp_gen[threadIdx.x] = 0;
+  }
   __syncthreads();
-  uint32_t slot = blockIdx.x * blockDim.x + threadIdx.x;
+  uint32_t slot = my_slot();
   Ctx C = make_ctx(A, slot);
   Ctx C2;
   if (NEST) {
@@ -168,90 +198,81 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
     C2.kb = A.kst2 + slot;
     C2.vb = A.vst2 + slot;
   }
-  int lane = threadIdx.x & 31;
   bool forms_left = true;
+  uint32_t round = 0;                                   // idle rounds taken (split_claim)
+  SplitGroup* G = nullptr;                              // the claimed group whose tasks this lane runs
+  uint32_t todo = 0;                                    // its task positions left for this lane
   for (;;) {
     uint32_t f = 0, root = 0, env = 0, d = 1;
     uint64_t fuel = A.fuel;
-    bool run;
     SplitTask* T = nullptr;
     if (!SPLIT || forms_left) {
-      uint32_t b = 0;
-      if (lane == 0) b = atomicAdd(A.next, 32u);
-      b = __shfl_sync(0xffffffffu, b, 0);
-      if (b >= A.nforms) {
+      uint32_t i = fetch_add_lanes32(A.next);
+      if (i >= A.nforms) {
         if (!SPLIT) break;
         forms_left = false;
-        if (lane == 0) atomicAdd(&A.sctl->hungry, 1);          // offer this warp to the busy ones
+        atomicAdd(&culi_warp_idle[threadIdx.x >> 5], 1u);
         continue;
       }
-      uint32_t i = b + lane;
-      run = i < A.nforms;
-      if (run) {
-        f = A.perm ? A.perm[i] : i;
-        root = A.roots[f];
-      }
+      f = A.perm ? A.perm[i] : i;
+      root = A.roots[f];
     } else {
-      uint32_t g = 0;
-      if (lane == 0) g = split_claim(A);
-      g = __shfl_sync(0xffffffffu, g, 0);
-      if (g == 0xffffffffu) break;
-      SplitGroup* G = A.groups + g;
-      ld_acquire(&G->state);                                   // acquire the owners' task and env writes
-      run = (G->mask >> lane) & 1u;
-      if (run) {
-        T = &G->t[lane];
-        f = G->form;
-        root = T->expr;
-        env = T->env;
-        d = T->depth;
-        fuel = T->budget;
+      if (!todo) {
+        uint32_t g = split_claim(A, round);
+        if (g == 0xffffffffu) break;
+        if (g == 0xfffffffeu) continue;
+        G = A.groups + g;
+        ld_acquire(&G->state);                          // acquire the owners' task and env writes
+        todo = G->mask & (1u << (threadIdx.x & 31));   // lane i runs owner lane i's task
+        if (!todo) continue;
       }
+      uint32_t p = __ffs(todo) - 1;
+      todo &= todo - 1;
+      T = &G->t[p];
+      f = G->form;
+      root = T->expr;
+      env = T->env;
+      d = T->depth;
+      fuel = T->budget;
     }
-    if (run) {
-      FormOut o;
-      bool resume = false;
-      Resume R{};
-      for (;;) {
-        o = eval_form<FANOUT, false, NEST, SPLIT>(C, root, f, 0, 0, fuel, d, resume, R, env);
-        if (!NEST || o.err != E_SUSPEND) break;
-        NestDesc* D = A.ndesc + o.aux;                  // suspended on a nested |||: help until done
-        unsigned long long t0 = 0;
-        while (*(volatile uint32_t*)&D->done < D->n) {
-          if (nest_help_any(A, C2, D)) { t0 = 0; continue; }
-          __nanosleep(128);
-          unsigned long long now = gtime();                   // bounded: an element that never finishes
-          if (!t0) t0 = now;                                    // sends the form to the sequential fallback
-          else if (now - t0 > A.wait_ns) { wait_gave_up(A, WAIT_NEST, o.aux, f); atomicOr(&D->bad, 4u); break; }
-        }
-        __threadfence();
-        uint64_t s = D->steps0 + *(volatile unsigned long long*)&D->total;
-        if (*(volatile uint32_t*)&D->bad || s > A.fuel) {   // decide exactly: sequential re-evaluation
-          A.fallback[atomicAdd(A.nfallback, 1u)] = f;
-          o.err = E_PENDING;
-          break;
-        }
-        R.sp = D->sp;
-        R.vtop = D->vtop;
-        R.steps = s;
-        R.v = mkv(K_CONS, D->spine);
-        resume = true;
+    FormOut o;
+    bool resume = false;
+    Resume R{};
+    for (;;) {
+      o = eval_form<FANOUT, false, NEST, SPLIT>(C, root, f, 0, 0, fuel, d, resume, R, env);
+      if (!NEST || o.err != E_SUSPEND) break;
+      NestDesc* D = A.ndesc + o.aux;                    // suspended on a nested |||: help until done
+      unsigned long long t0 = 0;
+      while (*(volatile uint32_t*)&D->done < D->n) {
+        if (nest_help_any(A, C2, D)) { t0 = 0; continue; }
+        __nanosleep(128);
+        unsigned long long now = gtime();                     // bounded: an element that never finishes
+        if (!t0) t0 = now;                                    // sends the form to the sequential fallback
+        else if (now - t0 > A.wait_ns) { wait_gave_up(A, WAIT_NEST, o.aux, f); atomicOr(&D->bad, 4u); break; }
       }
-      if (SPLIT && T) {                                 // a split-off argument: hand it to its owner
-        T->rt = o.t;
-        T->rw = o.w;
-        T->rsteps = o.steps;
-        T->rerr = o.err;
-        __threadfence();
-        st_release(&T->done, 1u);
-      } else {
-        write_result(A, f, o);
-        if (NEST || SPLIT) atomicAdd(A.finished, 1u);
+      __threadfence();
+      uint64_t s = D->steps0 + *(volatile unsigned long long*)&D->total;
+      if (*(volatile uint32_t*)&D->bad || s > A.fuel) {   // decide exactly: sequential re-evaluation
+        A.fallback[atomicAdd(A.nfallback, 1u)] = f;
+        o.err = E_PENDING;
+        break;
       }
+      R.sp = D->sp;
+      R.vtop = D->vtop;
+      R.steps = s;
+      R.v = mkv(K_CONS, D->spine);
+      resume = true;
     }
-    if (SPLIT && !forms_left) {
-      __syncwarp();
-      if (lane == 0) atomicAdd(&A.sctl->hungry, 1);            // ready for the next group
+    if (SPLIT && T) {                                   // a split-off argument: hand it to its owner
+      T->rt = o.t;
+      T->rw = o.w;
+      T->rsteps = o.steps;
+      T->rerr = o.err;
+      __threadfence();
+      st_release(&T->done, 1u);
+    } else {
+      write_result(A, f, o);
+      if (NEST || SPLIT) atomicAdd(A.finished, 1u);
     }
   }
   if (NEST) {                                           // no forms left: help until every form is done
@@ -394,11 +415,16 @@ __global__ void culi_reset_kernel(unsigned long long* top, unsigned long long to
                                   uint32_t* nfallback, uint32_t* nnest, SplitCtl* sctl) {
   *top = top_value;
   if (sctl) {                                         // tickets continue; unclaimed entries are dropped
-    sctl->head = sctl->tail;
-    sctl->hungry = 0;
+    unsigned long long t = sctl->tail > sctl->head ? sctl->tail : sctl->head;
+    sctl->head = t;
+    sctl->tail = t;
     sctl->published = 0;
+    sctl->claimed = 0;
+    for (int k = 0; k < 4; ++k) sctl->stat[k] = 0;
     sctl->timeouts = 0;
     for (int k = 0; k < 9; ++k) sctl->diag[k] = 0;
+    for (int k = 0; k < 8; ++k) sctl->wd[k] = 0;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(sctl->t0));
   }
   *next = 0;
   *pcount = 0;

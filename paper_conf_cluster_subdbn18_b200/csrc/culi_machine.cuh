@@ -129,7 +129,9 @@ __device__ __forceinline__ uint32_t cdr_of(const Ctx& C, uint32_t c) { return hi
 // receive adjacent ranges, so their node stores coalesce.
 __device__ __forceinline__ bool heap_alloc(const DevHeap& H, uint32_t n, uint32_t* out) {
   unsigned mask = __activemask();
-  unsigned peers = __match_any_sync(mask, n);
+  // (& mask: a lane group of another call converged onto this instruction must not leak into the result,
+  // see try_split)
+  unsigned peers = __match_any_sync(mask, n) & mask;
   int lane = threadIdx.x & 31;
   int leader = __ffs(peers) - 1;
   unsigned rank = __popc(peers & ((1u << lane) - 1u));
@@ -811,9 +813,43 @@ __device__ __forceinline__ unsigned long long gtime() {
   asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
   return t;
 }
+__device__ __forceinline__ unsigned long long ld_acquire64(const unsigned long long* p) {
+  unsigned long long v;
+  asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ unsigned long long ld_relaxed64(const unsigned long long* p) {
+  unsigned long long v;
+  asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+
+// Warp-aggregated fetch-and-add of 1 per calling lane (the lanes executing it together share one atomic
+// and get consecutive values in lane order).  Safe in diverged code: the mask is the lanes present, and no
+// other collective can run between __activemask and the shuffle (the leader's branch holds only the atomic).
+__device__ __forceinline__ unsigned long long fetch_add_lanes(unsigned long long* p) {
+  unsigned mask = __activemask();
+  int lane = threadIdx.x & 31;
+  int leader = __ffs(mask) - 1;
+  unsigned rank = __popc(mask & ((1u << lane) - 1u));
+  unsigned long long base = 0;
+  if (lane == leader) base = atomicAdd(p, (unsigned long long)__popc(mask));
+  base = __shfl_sync(mask, base, leader);
+  return base + rank;
+}
+__device__ __forceinline__ uint32_t fetch_add_lanes32(uint32_t* p) {
+  unsigned mask = __activemask();
+  int lane = threadIdx.x & 31;
+  int leader = __ffs(mask) - 1;
+  unsigned rank = __popc(mask & ((1u << lane) - 1u));
+  uint32_t base = 0;
+  if (lane == leader) base = atomicAdd(p, (uint32_t)__popc(mask));
+  base = __shfl_sync(mask, base, leader);
+  return base + rank;
+}
 
 // A bounded wait gave up: count it and keep the first occurrence's state for diagnosis.
-// Every wait on another warp is bounded by EvalArgs.wait_ns, so a protocol bug shows up as a counter and a
+// Every wait on another lane is bounded by EvalArgs.wait_ns, so a protocol bug shows up as a counter and a
 // status (culi_last_waits), never as a frozen GPU.
 __device__ CULI_COLD void wait_gave_up(const EvalArgs& A, uint32_t kind, uint32_t g, uint32_t form) {
   if (atomicAdd(&A.sctl->timeouts, 1u) != 0) return;
@@ -833,68 +869,71 @@ __device__ CULI_COLD void wait_gave_up(const EvalArgs& A, uint32_t kind, uint32_
   __threadfence();
 }
 
+#if CULI_WATCHDOG
+__device__ CULI_COLD bool watchdog_fired(Ctx C, uint32_t form, uint64_t steps, uint32_t sp, uint32_t d, uint32_t root) {
+  const EvalArgs& A = *C.A;
+  if (gtime() - *(volatile unsigned long long*)&A.sctl->t0 < (unsigned long long)CULI_WATCHDOG * 1000000ull) return false;
+  if (atomicAdd(&A.sctl->wd[0], 1u) == 0) {
+    uint32_t* w = A.sctl->wd;
+    w[1] = form; w[2] = (uint32_t)steps; w[3] = sp; w[4] = d; w[5] = root; w[6] = 0;
+    w[7] = *(volatile uint32_t*)A.finished;
+  }
+  return true;
+}
+#endif
+
 // In-use bits of the SPLIT_GPW group slots of each warp of the block (the block has 4 warps); cleared by
-// the kernel prologue, set by try_split, cleared by the last owner lane that joins the group.
+// the kernel prologue, set by try_split (atomic test-and-set), cleared by the last owner lane that joins.
 __shared__ uint32_t culi_split_busy[4];
 
-// Called by the lanes of a warp at a poll point (their top continuation already flushed to memory).  If an
-// idle warp is waiting (a token in A.hungry) and the warp has a free group slot, each lane looks for the
-// outermost KF_ARGS frame whose next argument is an unevaluated list, copies that frame's environment to
-// the heap (promote) and publishes the argument as task `lane` of the group; the frame becomes KF_JOIN and
-// its V-stack header records the group.  The owner later joins (RET KF_JOIN): it takes the group back if
-// no thief claimed it.
-// The lanes that call this together are those of __activemask(): in a diverged warp several lane groups
-// can be here at once, each with its own leader.  The slot is therefore claimed with an atomic
-// test-and-set of its busy bit (a plain read-then-set let two lane groups share one slot: the second
-// overwrote mask / remaining of the first, whose owners then waited for tasks no thief ran).
+__device__ __forceinline__ uint32_t my_slot() { return blockIdx.x * blockDim.x + threadIdx.x; }
+
+// Called by a lane at a poll point (its top continuation already flushed to memory).  If an idle warp waits
+// for work (head > tail), each polling lane looks for the outermost KF_ARGS frame whose next argument is an
+// unevaluated list and copies that frame's environment to the heap (promote).  Then the lanes that poll
+// together (__activemask(): typically a converged warp of same-shaped forms) publish their arguments as one
+// group: the first lane takes a free group slot of the warp, each lane with an argument writes task `lane`
+// and turns its frame into KF_JOIN (the V-stack header records the group), and the group goes into the
+// queue with one ticket.  Each owner lane later joins (RET KF_JOIN); the first to find the group unclaimed
+// takes the whole group back.
+// (Warp intrinsics only as __activemask -> ballot/shuffle over that mask with no other collective in
+// between, results restricted to the mask: a lane group of the same warp inside its own call can execute
+// the same instruction converged with ours.  DESIGN.md §5.5.)
 __device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t fuel, uint32_t form) {
   const EvalArgs& A = *C.A;
-  unsigned mask = __activemask();
-  int lane = threadIdx.x & 31;
-  int leader = __ffs(mask) - 1;
-  uint32_t* busy = &culi_split_busy[threadIdx.x >> 5];
   SplitCtl* Q = A.sctl;
-  int j = -1;
-  if (lane == leader && *(volatile int*)&Q->hungry > 0 &&
-      *(volatile unsigned long long*)&Q->tail - *(volatile unsigned long long*)&Q->head < A.gqcap / 2) {
-    for (;;) {
-      uint32_t freeb = ~*(volatile uint32_t*)busy & ((1u << SPLIT_GPW) - 1u);
-      if (!freeb) break;
-      uint32_t bit = freeb & (0u - freeb);
-      if (atomicOr(busy, bit) & bit) continue;                  // another lane group took it: retry
-      if (atomicSub(&Q->hungry, 1) > 0) {
-        j = __ffs(bit) - 1;
-      } else {
-        atomicAdd(&Q->hungry, 1);
-        atomicAnd(busy, ~bit);
-      }
-      break;
-    }
-  }
-  j = __shfl_sync(mask, j, leader);
-  if (j < 0) return;
+  uint32_t* busy = &culi_split_busy[threadIdx.x >> 5];
+  bool have = false;
   uint32_t lvl = 0xffffffffu, henv = 0;
   uint4 fr = make_uint4(0, 0, 0, 0);
-  for (uint32_t i = 0; i < sp; ++i) {
-    uint4 f = *KS(C, i);
-    if (kkind(f.w) == KF_ARGS && f.x != 0 && (ntag(C, car_of(C, f.x)) & KIND_MASK) == K_CONS) {
-      lvl = i;
-      fr = f;
-      break;
+  unsigned long long tail = ld_relaxed64(&Q->tail), head = ld_relaxed64(&Q->head);
+  if (head > tail && (~*(volatile uint32_t*)busy & ((1u << SPLIT_GPW) - 1u))) {
+    for (uint32_t i = 0; i < sp; ++i) {
+      uint4 f = *KS(C, i);
+      if (kkind(f.w) == KF_ARGS && f.x != 0 && (ntag(C, car_of(C, f.x)) & KIND_MASK) == K_CONS) {
+        lvl = i;
+        fr = f;
+        break;
+      }
     }
+    have = lvl != 0xffffffffu && promote(C, fr.y, &henv);
   }
-  bool have = lvl != 0xffffffffu && promote(C, fr.y, &henv);
-  unsigned part = __ballot_sync(mask, have);
-  if (!part) {                                                  // nothing to split: return slot and token
-    if (lane == leader) {
-      atomicAnd(busy, ~(1u << j));
-      atomicAdd(&Q->hungry, 1);
-    }
-    return;
+  unsigned m = __activemask();
+  unsigned part = __ballot_sync(m, have) & m;
+  if (!part) return;
+  int lane = threadIdx.x & 31, leader = __ffs(part) - 1;
+  int j = -1;
+  if (lane == leader) {                                         // one atomic test-and-set of a free slot
+    // (no retry loop: a spinning leader between two collectives let the other lanes pass the shuffle
+    // without it on sm_100a, a deadlock; a lost race just skips this poll)
+    uint32_t freeb = ~*(volatile uint32_t*)busy & ((1u << SPLIT_GPW) - 1u);
+    uint32_t bit = freeb & (0u - freeb);
+    if (bit && !(atomicOr(busy, bit) & bit)) j = __ffs(bit) - 1;
   }
-  uint32_t g = (blockIdx.x * blockDim.x + threadIdx.x) / 32 * SPLIT_GPW + (uint32_t)j;
+  j = __shfl_sync(m, j, leader);
+  if (j < 0) return;                                            // (promoted frames stay valid copies)
+  uint32_t g = my_slot() / 32 * SPLIT_GPW + (uint32_t)j;
   SplitGroup* G = A.groups + g;
-  if (lane == leader) G->state = SPLIT_TAKEN;                   // not claimable while it is rewritten
   if (have) {
     SplitTask* T = &G->t[lane];
     T->expr = car_of(C, fr.x);
@@ -904,8 +943,9 @@ __device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t
     T->done = 0;
     KS(C, lvl)->w = (fr.w & ~(0xfu << 12)) | (KF_JOIN << 12);
     VS(C, fr.z)->z = g + 1;                                     // the call's header: the group
+    __threadfence();
   }
-  __syncwarp(mask);
+  __syncwarp(m);                                                // every task written (and fenced)
   if (lane == leader) {
     G->mask = part;
     G->remaining = __popc(part);
@@ -918,18 +958,17 @@ __device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t
     unsigned long long e = ((q & 0xffffffffull) << 32) | (g + 1);
     asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(&A.gqueue[q & (A.gqcap - 1)]), "l"(e) : "memory");
   }
-  __syncwarp(mask);
 }
 
-// the owner lane is done with group G (joined): the last one frees the warp's slot
-__device__ __forceinline__ void split_release(const EvalArgs& A, uint32_t g) {
+// the owner lane is done with group g: the last one frees the warp's slot
+__device__ __forceinline__ void group_release(const EvalArgs& A, uint32_t g) {
   if (atomicSub(&A.groups[g].remaining, 1u) == 1u)
     atomicAnd(&culi_split_busy[threadIdx.x >> 5], ~(1u << (g % SPLIT_GPW)));
 }
 
-// Owner side of a join whose group a thief claimed: wait for this lane's task (bounded).  false = the
-// wait gave up; the owner then evaluates the argument itself and leaves the slot busy for the rest of the
-// launch, so a late thief can never write into a reused group.
+// Owner side of a join whose group a thief claimed: wait for this lane's task (bounded).  false = the wait
+// gave up; the owner then evaluates the argument itself and does not release the group, so its slot stays
+// busy for the rest of the launch and a late thief can never write into a reused group.
 __device__ CULI_COLD bool join_wait(const EvalArgs& A, SplitTask* T, uint32_t g, uint32_t form) {
   unsigned long long t0 = gtime();
   for (uint32_t spin = 1;; ++spin) {
@@ -942,19 +981,17 @@ __device__ CULI_COLD bool join_wait(const EvalArgs& A, SplitTask* T, uint32_t g,
   }
 }
 
-// A lane leaves its evaluation with an error while KF_JOIN frames are on its stack: hand their groups
-// back (still open: take it back, return the token, release the slot) so a warp whose forms fail does not
-// lose its slots; a group already claimed stays busy until the launch ends (its thief still writes it).
+// A lane leaves its evaluation with an error while KF_JOIN frames are on its stack: hand their groups back
+// (still open: take the group back and release this lane's share); a claimed group stays busy until the
+// launch ends (its thief still writes it).
 __device__ CULI_COLD void abandon_joins(Ctx C, uint32_t sp, uint4 ktop) {
   const EvalArgs& A = *C.A;
   for (uint32_t i = 0; i < sp; ++i) {
     uint4 f = i + 1 == sp ? ktop : *KS(C, i);
     if (kkind(f.w) != KF_JOIN) continue;
     uint32_t g = VS(C, f.z)->z - 1;
-    if (atomicCAS(&A.groups[g].state, SPLIT_OPEN, SPLIT_TAKEN) == SPLIT_OPEN) {
-      atomicAdd(&A.sctl->hungry, 1);
-      split_release(A, g);
-    }
+    uint32_t st = atomicCAS(&A.groups[g].state, SPLIT_OPEN, SPLIT_TAKEN);
+    if (st == SPLIT_OPEN || st == SPLIT_TAKEN) group_release(A, g);
   }
 }
 
@@ -1006,9 +1043,15 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32
 #define FAIL(e) do { err = (e); goto done; } while (0)
 // setq batches (R7): a frame moves to the heap as soon as it is made, so that no copy of it can go stale
 #define MUT_FRAME() do { uint32_t h_; if (__builtin_expect(!!(!promote(C, env, &h_)), 0)) FAIL(E_OOM); env = h_; } while (0)
+#if CULI_WATCHDOG
+#define WATCHDOG() do { if ((steps & 0x3fff) == 0 && watchdog_fired(C, form, steps, sp, d, root)) FAIL(E_OOM); } while (0)
+#else
+#define WATCHDOG() do { } while (0)
+#endif
 #define STEP(depth)                                     \
   do {                                                  \
     ++steps;                                            \
+    WATCHDOG();                                         \
     if (__builtin_expect(steps > fuel || (depth) > maxd, 0)) { \
       err = steps > fuel ? E_FUEL : E_DEPTH;            \
       goto done;                                        \
@@ -1368,17 +1411,17 @@ RET_POP:
       uint32_t g = hv.z - 1;
       SplitGroup* G = C.A->groups + g;
       uint32_t st = ld_acquire(&G->state);
-      if (st == SPLIT_OPEN) {                                   // unclaimed: take it back, evaluate here
+      if (st == SPLIT_OPEN) {                                   // unclaimed: take the group back
         st = atomicCAS(&G->state, SPLIT_OPEN, SPLIT_TAKEN);
-        if (st == SPLIT_OPEN) { atomicAdd(&C.A->sctl->hungry, 1); st = SPLIT_TAKEN; }
+        if (st == SPLIT_OPEN) st = SPLIT_TAKEN;
       }
-      if (st == SPLIT_TAKEN) { split_release(*C.A, g); goto ARGS; }
+      if (st == SPLIT_TAKEN) { group_release(*C.A, g); goto ARGS; }   // evaluate the argument here
       SplitTask* T = &G->t[threadIdx.x & 31];
       if (ld_acquire(&T->done) == 0 && !join_wait(*C.A, T, g, form)) goto ARGS;   // gave up: evaluate here
       uint64_t ts = T->rsteps;
       uint32_t te = T->rerr;
       V tv = mkv(T->rt, T->rw);
-      split_release(*C.A, g);
+      group_release(*C.A, g);
       // c.10: the sequential count at the end of this argument is steps + ts; fuel is checked first
       if (te == E_FUEL || steps + ts > fuel) { err = E_FUEL; steps = fuel + 1; goto done; }
       steps += ts;

@@ -11,7 +11,7 @@ import ctypes
 import os
 
 HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(HERE, "libculi.so")
+LIB_PATH = os.environ.get("CULI_LIB") or os.path.join(HERE, "libculi.so")   # CULI_LIB: A/B builds (tools/)
 
 ERR_NAMES = ["NONE", "TYPE", "ARITY", "DIV0", "SYNTAX", "ARG", "DEPTH", "FUEL", "DEFINE_IN_BATCH", "OOM"]
 TAG_NAMES = {0: "NIL", 1: "T", 2: "INT", 3: "FLOAT", 4: "STRING", 5: "SYMBOL", 6: "CONS", 7: "BUILTIN",
@@ -33,7 +33,7 @@ SYMBOLS = [
     "culi_result_int", "culi_result_float", "culi_print", "culi_results_totals", "culi_results_free",
     "culi_env_export", "culi_env_import", "culi_results_serialize", "culi_results_merge",
     "culi_status_string", "culi_error_name", "culi_last_timing", "culi_records_device",
-    "culi_last_stats", "culi_last_splits", "culi_last_waits", "culi_last_reruns", "culi_image_pin", "culi_results_wire_bytes",
+    "culi_last_stats", "culi_last_splits", "culi_last_split_claims", "culi_last_waits", "culi_last_reruns", "culi_image_pin", "culi_results_wire_bytes",
     "culi_define_text", "culi_eval_text", "culi_upload_text", "culi_last_read", "culi_collect",
     "culi_heap_usage", "culi_arena_bytes", "culi_eval_batch_async", "culi_sync", "culi_complete",
     "culi_results_export", "culi_results_import",
@@ -97,6 +97,7 @@ def load(path: str = LIB_PATH) -> ctypes.CDLL:
         "culi_records_device": (I, [P, P, SZ, pp(SZ)]),
         "culi_last_stats": (I, [P, pp(U32), pp(U32), pp(U32)]),
         "culi_last_splits": (I, [P, pp(U32)]),
+        "culi_last_split_claims": (I, [P, pp(U32)]),
         "culi_last_waits": (I, [P, pp(U32), pp(U32)]),
         "culi_last_reruns": (I, [P, pp(U32), pp(U32)]),
         "culi_image_pin": (I, [P, pp(U64)]),
@@ -115,6 +116,8 @@ def load(path: str = LIB_PATH) -> ctypes.CDLL:
         "culi_results_import": (I, [P, pp(P), pp(SZ), I, pp(pp(U32)), pp(P)]),
     }
     for name, (res, args) in sig.items():
+        if os.environ.get("CULI_LIB") and not hasattr(L, name):   # an older A/B build: skip newer calls
+            continue
         fn = getattr(L, name)
         fn.restype = res
         fn.argtypes = args
@@ -283,7 +286,10 @@ class Context:
             self._p = None
 
     def __del__(self):
-        self.close()
+        try:
+            self.close()
+        except Exception:  # noqa: BLE001 - interpreter shutdown (module globals already torn down)
+            pass
 
     def read(self, text: str | bytes) -> Image:
         b = text.encode() if isinstance(text, str) else text
@@ -412,6 +418,12 @@ class Context:
         """Split groups published by the last batch (argument splitting)."""
         g = ctypes.c_uint32()
         _check(load().culi_last_splits(self._p, ctypes.byref(g)), "culi_last_splits")
+        return g.value
+
+    def last_split_claims(self) -> int:
+        """Split tasks of the last batch that an idle lane claimed (the rest were taken back)."""
+        g = ctypes.c_uint32()
+        _check(load().culi_last_split_claims(self._p, ctypes.byref(g)), "culi_last_split_claims")
         return g.value
 
     def last_waits(self) -> tuple[int, list[int]]:
