@@ -270,20 +270,29 @@ def culi_arm(args):
     img = ctx.read(shard_text)
     t_read = time.perf_counter() - t0
     h = ctx.upload(img)
-    nrec = ctx.records_device(None)
-    rec = torch.empty(max(nrec, 8), dtype=torch.uint8, device=dev)
-    gathered = torch.empty(world * rec.numel(), dtype=torch.uint8, device=dev) if world > 1 else None
     flush = torch.empty(L2_FLUSH_BYTES, dtype=torch.uint8, device=dev)
+    # N > 1: the step ends with the device-resident result gather: every rank packs records
+    # + list payload + names into a fixed-size device buffer (culi_results_export, no host sync) and one
+    # NCCL all_gather moves the padded buffers; rank 0 can merge them on its GPU (culi_results_import, the
+    # e2e path below).  The capacity is the largest exact size over the ranks (+25 %), from one eval.
+    xcap, xbuf, gathered = 0, None, None
+    if world > 1:
+        from paper_conf_cluster_subdbn18_b200 import dist as D
+        ctx.eval_uploaded(h)
+        xcap = D.export_capacity(ctx)
+        xbuf = torch.empty(xcap, dtype=torch.uint8, device=dev)
+        gathered = torch.empty(world * xcap, dtype=torch.uint8, device=dev)
 
     def step():
         ctx.eval_uploaded(h)
         if world > 1:
-            ctx.records_device(rec.data_ptr(), rec.numel())
+            ctx.results_export(xbuf.data_ptr(), xcap)
             if cdev.type == "cuda":
-                dist.all_gather_into_tensor(gathered, rec)
+                dist.all_gather_into_tensor(gathered, xbuf)
             else:
-                g = torch.empty(world * rec.numel(), dtype=torch.uint8)
-                dist.all_gather_into_tensor(g, rec.cpu())
+                torch.cuda.synchronize()
+                g = torch.empty(world * xcap, dtype=torch.uint8)
+                dist.all_gather_into_tensor(g, xbuf.cpu())
                 gathered.copy_(g)
 
     for _ in range(args.warmup):
@@ -354,10 +363,8 @@ def culi_arm(args):
                 dist.barrier()
             a.record(stream)
             r = run()
-            nbytes = r.wire_bytes()
-            if world > 1:
-                from paper_conf_cluster_subdbn18_b200 import dist as D
-                D.gather_results(r, wl.nforms)
+            if r is not None:
+                nbytes = r.wire_bytes()
             b.record(stream)
             torch.cuda.synchronize()
             ms.append(a.elapsed_time(b))
@@ -369,11 +376,25 @@ def culi_arm(args):
             t = float(tt.item())
         return units_all * len(ms) / t, 1e3 * t / len(ms), nbytes
 
+    def e2e_text():
+        if world == 1:
+            return ctx.eval_text(text_host)
+        # N > 1: device read + eval of this rank's shard, device-resident gather, merge on rank 0's GPU,
+        # one D2H of the whole batch's results there (no Python bytes on the path)
+        hh, _nf = ctx.upload_text(text_host)
+        ctx.eval_uploaded(hh)
+        ctx.complete(hh)
+        merged = D.gather_results_device(ctx, xcap, dst=0)
+        ctx.release(hh)
+        return merged
+
     ctx.eval_text(text_host)                         # warm the reader's buffers
-    e2e_value, e2e_ms_step, d2h = e2e_loop(lambda: ctx.eval_text(text_host))
+    e2e_value, e2e_ms_step, d2h = e2e_loop(e2e_text)
     # the same through a host-read image (culi_read outside the timed region, culi_eval_batch inside)
     img_h2d = img.pin()
-    img_value, img_ms_step, _ = e2e_loop(lambda: ctx.eval_batch(img))
+    img_value, img_ms_step = None, None
+    if world == 1:
+        img_value, img_ms_step, _ = e2e_loop(lambda: ctx.eval_batch(img))
 
     # ---- device reader alone (§8(f)2): text resident in HBM -> node image in the heap
     text_dev = text_host.to(dev)
@@ -458,8 +479,10 @@ def culi_arm(args):
         "roofline": roof,
         "cpu_baseline": cpu,
         "e2e": {"value": e2e_value, "unit": "forms/s", "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
-                "ms_per_step": e2e_ms_step, "path": "culi_eval_text: pinned host text -> device read -> eval -> "
-                                                    "host results"},
+                "ms_per_step": e2e_ms_step,
+                "path": ("culi_eval_text: pinned host text -> device read -> eval -> host results" if world == 1
+                         else "per rank: pinned host text -> device read -> eval -> culi_results_export -> NCCL "
+                              "all_gather; rank 0: culi_results_import (device merge) -> host results")},
         "e2e_image": {"value": img_value, "unit": "forms/s", "h2d_bytes_per_step": img_h2d,
                       "ms_per_step": img_ms_step, "path": "culi_eval_batch on a host-read image"},
         "reader": reader,

@@ -840,13 +840,25 @@ int culi_eval_uploaded(culi_ctx* c, uint32_t handle) {
       if (g) cudaGraphDestroy(g);
       return rc ? rc : CULI_E_CUDA;
     }
+    // the exact number of kernels one step launches: the kernel nodes of the captured graph (the library
+    // sort picks its kernels by size, so counting launch calls would only estimate it)
+    size_t nn = 0;
+    uint32_t kn = 0;
+    if (cudaGraphGetNodes(g, nullptr, &nn) == cudaSuccess && nn) {
+      std::vector<cudaGraphNode_t> nodes(nn);
+      if (cudaGraphGetNodes(g, nodes.data(), &nn) == cudaSuccess)
+        for (size_t q = 0; q < nn; ++q) {
+          cudaGraphNodeType ty;
+          if (cudaGraphNodeGetType(nodes[q], &ty) == cudaSuccess && ty == cudaGraphNodeTypeKernel) ++kn;
+        }
+    }
     e = cudaGraphInstantiate(&c->graph_exec, g, 0);
     cudaGraphDestroy(g);
     if (e != cudaSuccess) {
       c->graph_exec = nullptr;
       return CULI_E_CUDA;
     }
-    c->graph_kernels = c->last_kernels;
+    c->graph_kernels = kn ? kn : c->last_kernels;
   }
   CK(cudaGraphLaunch(c->graph_exec, c->stream));
   c->last_kernels = c->graph_kernels;

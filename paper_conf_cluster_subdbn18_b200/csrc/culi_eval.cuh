@@ -221,7 +221,7 @@ cudaError_t launch_dispatch(cudaStream_t s, const DevHeap& H, const uint32_t* ro
                             uint32_t* keys, uint32_t* keys_alt, uint32_t* perm, uint32_t* perm_alt,
                             void* temp, size_t temp_bytes, uint32_t** perm_out, int sms);
 size_t dispatch_temp_bytes(uint32_t nforms);
-uint32_t dispatch_launches(uint32_t nforms);   // kernels launch_dispatch issues
+uint32_t dispatch_launches(uint32_t nforms);   // kernels launch_dispatch issues (an estimate: the graph path counts them)
 // Batches of at most this many forms in which no closure can exist (no lambda / defun) are evaluated in
 // input order: with <= 128 warps (fewer than the 148 SMs) the eval time is the slowest warp's either way,
 // and the binning permutation scatters the warps' node loads.  Measured on C1 (1,024 forms): dispatch

@@ -114,8 +114,40 @@ def sweep(paths, peak_gbs=6547.5):
     return "\n".join(out)
 
 
+def eval_profiles(paths, outdir):
+    """profiles/eval_inst_<wl>.json from a sweep capture: warp instructions and DRAM bytes of one launch of
+    each eval-phase kernel (culi_eval*, culi_fanout_kernel), summed — the numbers bench.py's roofline uses."""
+    for path in paths:
+        wl = path.rsplit("_", 1)[-1].split(".")[0]
+        rows = list(csv.reader(open(path, errors="replace")))
+        hi = next(i for i, r in enumerate(rows) if "Metric Name" in r)
+        h = rows[hi]
+        ii, ki, mi, ui, vi = (h.index(x) for x in ("ID", "Kernel Name", "Metric Name", "Metric Unit", "Metric Value"))
+        per = {}
+        for r in rows[hi + 1:]:
+            if len(r) > vi:
+                per.setdefault((r[ki].split("(")[0], r[ii]), {})[r[mi]] = num(r[vi]) * UNIT.get(r[ui], 1.0)
+        seen, inst, dram, t, kern = set(), 0.0, 0.0, 0.0, []
+        for (k, lid), m in sorted(per.items(), key=lambda kv: int(kv[0][1])):
+            if k in seen or not ("culi_eval" in k or "culi_fanout_kernel" in k):
+                continue
+            seen.add(k)
+            kern.append(k.replace("void ", ""))
+            inst += m.get("smsp__inst_executed.sum", 0)
+            dram += m.get("dram__bytes_read.sum", 0) + m.get("dram__bytes_write.sum", 0)
+            t += m.get("gpu__time_duration.sum", 0)
+        out = {"source": path, "kernels": kern, "warp_inst_per_launch": inst, "dram_bytes": dram,
+               "kernel_seconds_under_ncu": t}
+        with open("%s/eval_inst_%s.json" % (outdir, wl.lower()), "w") as f:
+            json.dump(out, f)
+        print(wl, json.dumps(out))
+
+
 def main():
     mode, path = sys.argv[1], sys.argv[2]
+    if mode == "profiles":
+        eval_profiles(sys.argv[3:], path)
+        return
     if mode == "launches":
         print(launches(path))
         return

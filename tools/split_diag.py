@@ -25,12 +25,12 @@ t0 = time.time()
 for k in range(reps):
     ctx.eval_uploaded(h)
     ms, kern, _ = ctx.last_timing()
-    evs.append(ms[1])
+    evs.append(ms[1]); disp = ms[0]
 r = ctx.fetch_results(h)
 tot, nerr = r.totals()
 sp = ctx.last_splits()
 w = ctx.last_waits() if hasattr(L, "culi_last_waits") else None
 cl = ctx.last_split_claims() if hasattr(L, "culi_last_split_claims") else None
-print("%s flags=%d lib=%s eval ms %s steps %d err %d splits %d claimed %s waits %s wall %.1fs" % (
-    wlname, flags, os.path.basename(os.environ.get("CULI_LIB", "libculi.so")), " ".join("%.2f" % e for e in evs),
+print("%s flags=%d lib=%s dispatch %.3f eval ms %s steps %d err %d splits %d claimed %s waits %s wall %.1fs" % (
+    wlname, flags, os.path.basename(os.environ.get("CULI_LIB", "libculi.so")), disp, " ".join("%.2f" % e for e in evs),
     tot, nerr, sp, cl, w, time.time() - t0), flush=True)
