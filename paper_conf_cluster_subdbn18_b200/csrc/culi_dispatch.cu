@@ -2,9 +2,10 @@
 //
 // The paper notes that divergent branches of a warp are serialised (§III-D.d).  Forms are
 // independent, so their evaluation order is free: we give each form a 64-bit key
-//   (36-bit structure prefix << 28) | (12-bit shape hash << 16) | (0xffff - cost hint)
-// where the structure prefix is the form's first six pre-order tokens (list open / close, number kinds,
-// the reserved operator or a user-symbol bucket; 6 bits each, most significant first, so forms that share
+//   (30-bit structure prefix << 26) | (10-bit shape hash << 16) | (0xffff - cost hint)
+// where the structure prefix is the form's first five pre-order tokens (list open, number kinds, a
+// user-symbol bucket before the reserved operators — user functions are the heavy forms, so they start
+// first; 6 bits each, most significant first, so forms that share
 // a beginning sort next to each other even when they differ later), the shape hash covers the form's
 // first 48 nodes (kinds, symbols, structure; not number values) so identical shapes are contiguous inside
 // a prefix, and the cost hint is the first argument when it is an integer literal (e.g. n of (fib n)), so
@@ -47,16 +48,16 @@ __device__ uint32_t shape_hash(const uint8_t* __restrict__ tag, const uint64_t* 
   return h;
 }
 
-// Pre-order token stream of a form, most significant first: 6 bits per token, the first six tokens.
+// Pre-order token stream of a form, most significant first: 6 bits per token, the first five tokens.
 __device__ uint64_t structure_prefix(const uint8_t* __restrict__ tag, const uint64_t* __restrict__ word, uint32_t x) {
   uint32_t st[8];
   int sp = 0, n = 0;
   uint64_t key = 0;
   auto emit = [&](uint32_t code) {
-    if (n < 6) key |= (uint64_t)(code & 63u) << (6 * (5 - n));
+    if (n < 5) key |= (uint64_t)(code & 63u) << (6 * (4 - n));
     ++n;
   };
-  for (int visited = 0; visited < 24 && n < 6; ++visited) {
+  for (int visited = 0; visited < 24 && n < 5; ++visited) {
     uint32_t t = tag[x] & KIND_MASK;
     if (t == K_CONS) {
       uint64_t w = word[x];
@@ -69,7 +70,7 @@ __device__ uint64_t structure_prefix(const uint8_t* __restrict__ tag, const uint
     uint32_t code = t == K_INT ? 3 : t == K_FLOAT ? 4 : t == K_STR ? 5 : t == K_NIL ? 6 : t == K_T ? 7 : 2;
     if (t == K_SYM) {
       uint32_t sid = (uint32_t)word[x];
-      code = sid < N_RESERVED ? 8 + sid : 48 + (sid & 15u);
+      code = sid < N_RESERVED ? 24 + sid : 8 + (sid & 15u);   // user functions first: heaviest work early
     }
     emit(code);
     if (sp == 0) break;
@@ -102,15 +103,15 @@ __global__ void culi_classify_kernel(const uint8_t* __restrict__ tag, const uint
       }
       shape = shape_hash(tag, word, r);
     }
-    // 64 bits (8 radix passes): structure prefix 36 | shape hash 12 | inverted hint 16
-    keys[f] = (prefix << 28) | ((unsigned long long)((shape ^ (shape >> 12) ^ (shape >> 24)) & 0xfffu) << 16) |
+    // 56 bits (7 radix passes): structure prefix 30 | shape hash 10 | inverted hint 16
+    keys[f] = (prefix << 26) | ((unsigned long long)((shape ^ (shape >> 10) ^ (shape >> 20)) & 0x3ffu) << 16) |
               (0xffffu - hint);
     perm[f] = f;
   }
 }
 
-// classify + CUB histogram + exclusive sum + 8 one-sweep passes (64 key bits)
-uint32_t dispatch_launches(uint32_t) { return 11u; }
+// classify + CUB histogram + exclusive sum + 7 one-sweep passes (56 key bits)
+uint32_t dispatch_launches(uint32_t) { return 10u; }
 
 size_t dispatch_temp_bytes(uint32_t nforms) {
   size_t bytes = 0;
@@ -133,7 +134,7 @@ cudaError_t launch_dispatch(cudaStream_t s, const DevHeap& H, const uint32_t* ro
   cudaError_t e = cudaGetLastError();
   if (e != cudaSuccess) return e;
   size_t tb = temp_bytes;
-  e = cub::DeviceRadixSort::SortPairs(temp, tb, k0, k1, perm, perm_alt, (int)nforms, 0, 64, s);
+  e = cub::DeviceRadixSort::SortPairs(temp, tb, k0, k1, perm, perm_alt, (int)nforms, 0, 56, s);
   *perm_out = perm_alt;
   return e;
 }
