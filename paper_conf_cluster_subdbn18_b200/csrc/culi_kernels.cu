@@ -118,7 +118,7 @@ __device__ __noinline__ uint32_t claim_group(const EvalArgs& A) {
   const unsigned long long* qe = &A.gqueue[h & (A.gqcap - 1)];
   uint32_t ns = 64;
   for (uint32_t spin = 0;; ++spin) {
-    unsigned long long e = ld_acquire64(qe);
+    unsigned long long e = ld_relaxed64(qe);             // (relaxed: an acquire poll invalidates L1)
     if ((uint32_t)(e >> 32) == (uint32_t)h && (uint32_t)e != 0) {   // (0: never written)
       uint32_t g = (uint32_t)e - 1;
       if (atomicCAS(&A.groups[g].state, SPLIT_OPEN, SPLIT_CLAIMED) != SPLIT_OPEN) return 0xfffffffeu;
@@ -268,8 +268,7 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
       T->rw = o.w;
       T->rsteps = o.steps;
       T->rerr = o.err;
-      __threadfence();
-      st_release(&T->done, 1u);
+      st_release(&T->done, 1u);                         // (the release orders the result writes)
     } else {
       write_result(A, f, o);
       if (NEST || SPLIT) atomicAdd(A.finished, 1u);

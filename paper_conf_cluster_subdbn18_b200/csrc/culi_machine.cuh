@@ -943,15 +943,15 @@ __device__ CULI_COLD void try_split(Ctx C, uint32_t sp, uint64_t steps, uint64_t
     T->done = 0;
     KS(C, lvl)->w = (fr.w & ~(0xfu << 12)) | (KF_JOIN << 12);
     VS(C, fr.z)->z = g + 1;                                     // the call's header: the group
-    __threadfence();
   }
-  __syncwarp(m);                                                // every task written (and fenced)
+  // every task written: bar.warp.sync orders the lanes' writes before the leader's release below (no
+  // fence.sc: it would invalidate the SM's L1)
+  __syncwarp(m);
   if (lane == leader) {
     G->mask = part;
     G->remaining = __popc(part);
     G->form = form;
     G->claimer = 0xffffffffu;
-    __threadfence();
     st_release(&G->state, SPLIT_OPEN);
     unsigned long long q = atomicAdd(&Q->tail, 1ull);
     atomicAdd(&Q->published, 1u);
@@ -969,11 +969,24 @@ __device__ __forceinline__ void group_release(const EvalArgs& A, uint32_t g) {
 // Owner side of a join whose group a thief claimed: wait for this lane's task (bounded).  false = the wait
 // gave up; the owner then evaluates the argument itself and does not release the group, so its slot stays
 // busy for the rest of the launch and a late thief can never write into a reused group.
+// The poll is a relaxed load: an acquire (ld.acquire / fence.sc) invalidates the SM's whole L1 on sm_100a
+// (CCTL.IVALL), and waiting owners polling every 200 ns did so 490 M times per C2 launch, evicting the
+// stacks and code of every busy warp on the SM (ncu).  One acquire once the flag is seen.
+__device__ __forceinline__ uint32_t ld_relaxed(const uint32_t* p) {
+  uint32_t v;
+  asm volatile("ld.relaxed.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  return v;
+}
 __device__ CULI_COLD bool join_wait(const EvalArgs& A, SplitTask* T, uint32_t g, uint32_t form) {
   unsigned long long t0 = gtime();
+  uint32_t ns = 128;
   for (uint32_t spin = 1;; ++spin) {
-    if (ld_acquire(&T->done) != 0) return true;
-    __nanosleep(200);
+    if (ld_relaxed(&T->done) != 0) {
+      ld_acquire(&T->done);
+      return true;
+    }
+    __nanosleep(ns);
+    ns = ns < 1024 ? ns * 2 : ns;
     if ((spin & 63) == 0 && gtime() - t0 > A.wait_ns) {
       wait_gave_up(A, WAIT_JOIN, g, form);
       return false;
