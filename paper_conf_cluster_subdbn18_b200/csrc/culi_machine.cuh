@@ -986,8 +986,8 @@ __device__ CULI_COLD bool join_wait(const EvalArgs& A, SplitTask* T, uint32_t g,
       return true;
     }
     __nanosleep(ns);
-    ns = ns < 1024 ? ns * 2 : ns;
-    if ((spin & 63) == 0 && gtime() - t0 > A.wait_ns) {
+    ns = ns < A.split_sleep ? ns * 2 : ns;                      // (polling warps cost issue slots and I$)
+    if ((spin & 15) == 0 && gtime() - t0 > A.wait_ns) {
       wait_gave_up(A, WAIT_JOIN, g, form);
       return false;
     }
