@@ -88,9 +88,11 @@ struct Arena {
 };
 
 // ---- reserved names: special forms (c.5) then builtins (c.6) -------------------------------------
-enum Special { S_QUOTE, S_IF, S_DEFINE, S_DEFUN, S_DEFMACRO, S_LAMBDA, S_LET, S_PROGN, S_SETQ, N_SPECIAL };
+enum Special { S_QUOTE, S_IF, S_DEFINE, S_DEFUN, S_DEFMACRO, S_LAMBDA, S_LET, S_PROGN, S_SETQ,
+               S_QUASIQUOTE, S_UNQUOTE, S_UNQUOTE_SPLICING, N_SPECIAL };
 static const char* kSpecialNames[N_SPECIAL] = {"quote", "if", "define", "defun", "defmacro",
-                                               "lambda", "let", "progn", "setq"};
+                                               "lambda", "let", "progn", "setq",
+                                               "quasiquote", "unquote", "unquote-splicing"};
 enum Builtin {
   B_ADD, B_SUB, B_MUL, B_DIV, B_REM, B_MOD, B_SQRT, B_FLOAT, B_TRUNC,
   B_NUM_EQ, B_LT, B_GT, B_LE, B_GE, B_EQ, B_EQUAL, B_NULL, B_NOT,
@@ -285,10 +287,11 @@ struct Reader {
     if (p >= src.size()) throw ReadError{p};
     char c = src[p];
     if (c == ')') throw ReadError{p};
-    if (c == '\'') {                                    // 'x == (quote x)
-      ++p;
+    if (c == '\'' || c == '`' || c == ',') {            // 'x == (quote x); DESIGN R8: `x == (quasiquote x),
+      ++p;                                              // ,x == (unquote x) (no ,@ shorthand)
       Val d = datum();
-      return mk_cons(A, mk_sym(S.intern("quote")), mk_cons(A, d, mk_nil()));
+      const char* name = c == '\'' ? "quote" : c == '`' ? "quasiquote" : "unquote";
+      return mk_cons(A, mk_sym(S.intern(name)), mk_cons(A, d, mk_nil()));
     }
     if (c == '(') {                                     // L416-421
       size_t open = p;
@@ -411,6 +414,48 @@ struct Interp {
     Val v; v.tag = t; v.clo = &A.closures.back(); return v;
   }
 
+  // ---- quasiquote (reading R8) ------------------------------------------------
+  // qq(t, L): the template t at nesting level L.  An atom is itself (not evaluated).  (unquote e) at
+  // level 1 is eval(e) at depth+1 of the quasiquote form; at a deeper level it is rebuilt as
+  // (unquote qq(e, L-1)); (quasiquote e) inside is rebuilt as (quasiquote qq(e, L+1)).  Any other list is
+  // rebuilt element by element, left to right; an element (unquote-splicing e) at level 1 evaluates e,
+  // which must be a proper list (else TYPE), and its elements are copied in.  Every list of the template
+  // is a fresh contiguous copy.  (unquote ...) / (unquote-splicing ...) / (quasiquote ...) with other than
+  // one argument, (unquote-splicing e) not in an element position at level 1, and an improper template
+  // list are SYNTAX errors, raised when the walk reaches them.  The walk itself takes no steps.
+  bool is_op_list(Val t, int op) {
+    return t.tag == CONS && t.cell->car.tag == SYMBOL && t.cell->car.sym == (uint32_t)op;
+  }
+  Val qq_arg(Val t) {                                   // the single argument of (op x), else SYNTAX
+    if (!is_proper_list(t)) fail(E_SYNTAX);
+    std::vector<Val> xs = list_elems(t);
+    if (xs.size() != 2) fail(E_SYNTAX);
+    return xs[1];
+  }
+  Val qq(Val t, int level, const Frame* env, uint32_t depth) {
+    if (t.tag != CONS) return t;
+    if (!is_proper_list(t)) fail(E_SYNTAX);
+    if (is_op_list(t, S_UNQUOTE) && level == 1) return eval(qq_arg(t), env, depth + 1);
+    if (is_op_list(t, S_UNQUOTE_SPLICING) && level == 1) fail(E_SYNTAX);   // not in an element position
+    int rest_level = level;
+    if (is_op_list(t, S_QUASIQUOTE)) { qq_arg(t); rest_level = level + 1; }
+    else if (is_op_list(t, S_UNQUOTE) || is_op_list(t, S_UNQUOTE_SPLICING)) { qq_arg(t); rest_level = level - 1; }
+    std::vector<Val> out;
+    std::vector<Val> xs = list_elems(t);
+    for (size_t k = 0; k < xs.size(); ++k) {
+      int L = k == 0 ? level : rest_level;
+      Val e = xs[k];
+      if (L == 1 && is_op_list(e, S_UNQUOTE_SPLICING)) {
+        Val v = eval(qq_arg(e), env, depth + 1);
+        if (!is_proper_list(v)) fail(E_TYPE);
+        for (Val y : list_elems(v)) out.push_back(y);
+        continue;
+      }
+      out.push_back(qq(e, L, env, depth));
+    }
+    return make_list(A, out, mk_nil());
+  }
+
   // ---- special forms (c.5): syntax checked before anything is evaluated; sub-evals at depth+1 ----
   Val apply_special(int op, Val rest, const Frame* env, uint32_t depth) {
     std::vector<Val> a = list_elems(rest);
@@ -467,6 +512,12 @@ struct Interp {
         for (Val x : a) r = eval(x, env, depth + 1);
         return r;
       }
+      case S_QUASIQUOTE:
+        if (n != 1) fail(E_SYNTAX);
+        return qq(a[0], 1, env, depth);
+      case S_UNQUOTE:
+      case S_UNQUOTE_SPLICING:
+        fail(E_SYNTAX);                                      // only meaningful inside a quasiquote template
       case S_SETQ: {
         // "setq updates the nearest existing symbol that matches" — a local variable or,
         // failing that, the global one.  DESIGN.md R7: the value is evaluated first; during a batch the

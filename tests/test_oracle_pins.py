@@ -522,3 +522,68 @@ def test_bruteforce_arith_trees_exhaustive(sess):
     res = sess.eval("\n".join(t for t, _, _ in trees))
     for (text, val, ops), r in zip(trees, res):
         assert (int(r.printed), r.steps) == (wrap64(val), 3 * ops + 1), text
+
+
+# ---- quasiquote (reading R8) --------------------------------------------------
+@pytest.mark.parametrize("row", load_tsv("quasiquote_pins.tsv"), ids=lambda r: r[0][:40])
+def test_quasiquote_pins(oracle_mod, row):
+    s = oracle_mod.Session()
+    r = s.eval1(row[0])
+    assert (r.printed, r.steps) == (row[1], int(row[2])), row
+
+
+def test_quasiquote_macro(oracle_mod):
+    """A macro written with a quasiquote template expands to the same code as its list-built twin: same
+    value; steps differ only by the construction cost of the expansion (R8: the walk is free, each unquote
+    one step for a parameter symbol, vs. list + head + one step per list argument)."""
+    s = oracle_mod.Session()
+    s.define("(defmacro my-if (c a b) `(if ,c ,a ,b))\n(defmacro my-if2 (c a b) (list 'if c a b))")
+    r1 = s.eval1("(my-if (< 1 2) 'yes 'no)")
+    assert (r1.printed, r1.steps) == ("yes", 15)        # 2 call + 5 template (2 + c a b) + 8 expansion
+    r2 = s.eval1("(my-if2 (< 1 2) 'yes 'no)")
+    assert (r2.printed, r2.steps) == ("yes", 17)        # 2 call + 7 (list 'if c a b), as c.12b's when, + 8
+
+
+def _qq_equiv(t):
+    """Python model of R8 for flat templates: items are ('lit', x) | ('uq', expr, value) | ('spl', expr, list)."""
+    out, text, steps = [], [], 2
+    for it in t:
+        if it[0] == "lit":
+            out.append(it[1]); text.append(str(it[1]))
+        elif it[0] == "uq":
+            out.append(it[2]); text.append(",(+ %d %d)" % it[1]); steps += 4
+        else:
+            out.extend(it[2]); text.append("(unquote-splicing (list%s))" % "".join(" %d" % v for v in it[2]))
+            steps += 2 + len(it[2])
+    return "`(" + " ".join(text) + ")", ("(" + " ".join(map(str, out)) + ")") if out else "nil", steps
+
+
+def test_quasiquote_bruteforce(oracle_mod):
+    """Random flat templates against a Python model of R8 (values and step counts)."""
+    rnd = random.Random(8)
+    s = oracle_mod.Session()
+    cases = []
+    for _ in range(300):
+        t = []
+        for _ in range(rnd.randint(0, 6)):
+            k = rnd.randint(0, 2)
+            if k == 0:
+                t.append(("lit", rnd.randint(-9, 9)))
+            elif k == 1:
+                a, b = rnd.randint(-9, 9), rnd.randint(-9, 9)
+                t.append(("uq", (a, b), a + b))
+            else:
+                t.append(("spl", None, [rnd.randint(-9, 9) for _ in range(rnd.randint(0, 3))]))
+        cases.append(_qq_equiv(t))
+    res = s.eval("\n".join(c[0] for c in cases))
+    for (text, printed, steps), r in zip(cases, res):
+        assert (r.printed, r.steps) == (printed, steps), text
+
+
+def test_quasiquote_reader(oracle_mod):
+    s = oracle_mod.Session()
+    assert s.read_print("`(a ,b)\n'`x\n,,y\na`b\nc,d") == [
+        "(quasiquote (a (unquote b)))", "(quote (quasiquote x))", "(unquote (unquote y))", "a`b", "c,d"]
+    for bad in ["`", "(a ,)", ",", "`)"]:
+        with pytest.raises(oracle_mod.OracleError):
+            s.read_print(bad)
