@@ -48,6 +48,7 @@ __device__ uint32_t shape_hash(const uint8_t* __restrict__ tag, const uint64_t* 
   return h;
 }
 
+static_assert(16 + N_RESERVED <= 64, "reserved-operator token codes fit in 6 bits");
 // Pre-order token stream of a form, most significant first: 6 bits per token, the first five tokens.
 __device__ uint64_t structure_prefix(const uint8_t* __restrict__ tag, const uint64_t* __restrict__ word, uint32_t x) {
   uint32_t st[8];
@@ -70,7 +71,7 @@ __device__ uint64_t structure_prefix(const uint8_t* __restrict__ tag, const uint
     uint32_t code = t == K_INT ? 3 : t == K_FLOAT ? 4 : t == K_STR ? 5 : t == K_NIL ? 6 : t == K_T ? 7 : 2;
     if (t == K_SYM) {
       uint32_t sid = (uint32_t)word[x];
-      code = sid < N_RESERVED ? 24 + sid : 8 + (sid & 15u);   // user functions first: heaviest work early
+      code = sid < N_RESERVED ? 16 + sid : 8 + (sid & 7u);    // user functions first: heaviest work early
     }
     emit(code);
     if (sp == 0) break;

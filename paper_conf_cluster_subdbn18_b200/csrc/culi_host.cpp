@@ -78,7 +78,8 @@ void pinned_pool_free(void* p, size_t bytes) {
 }
 
 const char* const kSpecialName[N_SPECIALS] = {"quote", "if", "define", "defun", "defmacro", "lambda",
-                                              "let", "progn", "setq"};
+                                              "let", "progn", "setq", "quasiquote", "unquote",
+                                              "unquote-splicing"};
 const char* const kBuiltinName[N_BUILTINS] = {
     "+", "-", "*", "/", "rem", "mod", "sqrt", "float", "trunc",
     "=", "<", ">", "<=", ">=", "eq", "equal", "null", "not",
@@ -144,9 +145,10 @@ static bool classify_float(const char* s, size_t n) {
 
 namespace {
 struct Open {
-  bool quote;                  // a pending ' prefix (completes after one datum)
-  size_t offset;               // byte offset of '(' or '\''
+  bool quote;                  // a pending prefix (' ` ,) that completes after one datum
+  size_t offset;               // byte offset of '(' or the prefix
   std::vector<uint32_t> elems; // elements of an open list
+  uint32_t prefix_sym = SP_QUOTE;   // quote / quasiquote / unquote (reading R8)
 };
 
 struct Builder {
@@ -197,7 +199,8 @@ struct Builder {
     if ((ltag(h) & KIND_MASK) != K_SYM || lword(h) >= N_SPECIALS) return false;
     size_t n = xs.size() - 1;
     switch (lword(h)) {
-      case SP_QUOTE: return n == 1;
+      case SP_QUOTE:
+      case SP_QUASIQUOTE: return n == 1;
       case SP_IF: return n == 2 || n == 3;
       case SP_PROGN: return true;
       case SP_LAMBDA: return n >= 1 && params_ok(xs[1]);
@@ -228,7 +231,6 @@ int read_image(SymTable& st, const char* text, size_t len, Image& img, size_t* e
     if (err_offset) *err_offset = off;
     return (int)CULI_E_PARSE;
   };
-  const uint32_t quote_id = SP_QUOTE;
 
   // deliver a finished datum to the innermost open construct
   auto deliver = [&](uint32_t d) {
@@ -236,8 +238,9 @@ int read_image(SymTable& st, const char* text, size_t len, Image& img, size_t* e
       if (stack.empty()) { img.roots.push_back(d); return; }
       Open& top = stack.back();
       if (!top.quote) { top.elems.push_back(d); return; }
-      stack.pop_back();                              // 'x == (quote x)
-      std::vector<uint32_t> q{B.symbol(quote_id), d};
+      uint32_t sym = top.prefix_sym;
+      stack.pop_back();                              // 'x == (quote x), `x, ,x (R8)
+      std::vector<uint32_t> q{B.symbol(sym), d};
       d = B.spine(q);
     }
   };
@@ -259,8 +262,9 @@ int read_image(SymTable& st, const char* text, size_t len, Image& img, size_t* e
       stack.pop_back();
       ++p;
       deliver(B.spine(xs));
-    } else if (c == '\'') {
-      stack.push_back(Open{true, p, {}});
+    } else if (c == '\'' || c == '`' || c == ',') {
+      stack.push_back(Open{true, p, {}, c == '\'' ? (uint32_t)SP_QUOTE : c == '`' ? (uint32_t)SP_QUASIQUOTE
+                                                                            : (uint32_t)SP_UNQUOTE});
       ++p;
     } else if (c == '"') {
       const void* q = std::memchr(text + p + 1, '"', len - p - 1);

@@ -34,7 +34,7 @@ enum ErrCode : uint8_t {
 
 // Reserved symbols (SURVEY c.5 "reserved names"): ids [0, N_RESERVED) in this order.
 enum SpecialOp : uint8_t { SP_QUOTE, SP_IF, SP_DEFINE, SP_DEFUN, SP_DEFMACRO, SP_LAMBDA, SP_LET,
-                           SP_PROGN, SP_SETQ, N_SPECIALS };
+                           SP_PROGN, SP_SETQ, SP_QUASIQUOTE, SP_UNQUOTE, SP_UNQUOTE_SPLICING, N_SPECIALS };
 enum BuiltinOp : uint8_t {
   BI_ADD, BI_SUB, BI_MUL, BI_DIV, BI_REM, BI_MOD, BI_SQRT, BI_FLOAT, BI_TRUNC,
   BI_NUMEQ, BI_LT, BI_GT, BI_LE, BI_GE, BI_EQ, BI_EQUAL, BI_NULL, BI_NOT,

@@ -712,6 +712,7 @@ __device__ CULI_COLD bool special_syntax_ok(Ctx C, uint32_t op, uint32_t cur) {
     case SP_SETQ: return n == 2 && bindable_node(C, car_of(C, cur));
     case SP_DEFUN: case SP_DEFMACRO:
       return n >= 2 && bindable_node(C, car_of(C, cur)) && valid_params(C, car_of(C, cdr_of(C, cur)));
+    case SP_QUASIQUOTE: return n == 1;
     case SP_LET: {
       if (n < 1) return false;
       uint32_t bl = car_of(C, cur);
@@ -794,8 +795,27 @@ __device__ __forceinline__ int try_leaf(const Ctx& C, uint32_t xt, uint64_t xw, 
   return 1;
 }
 
+// ---- quasiquote (reading R8) ----------------------------------------------------
+// The quasiquote operator a template list starts with (its head node), else 0xff.
+__device__ __forceinline__ uint32_t qq_op(const Ctx& C, uint64_t listword) {
+  uint32_t ht;
+  uint64_t hw;
+  ldnode(C, lo32(listword), ht, hw);
+  if ((ht & KIND_MASK) != K_SYM) return 0xffu;
+  return (hw == SP_QUASIQUOTE || hw == SP_UNQUOTE || hw == SP_UNQUOTE_SPLICING) ? (uint32_t)hw : 0xffu;
+}
+// The single argument of a proper (op x) whose cell word is `listword`; false: not exactly one argument.
+__device__ __forceinline__ bool qq_arg(const Ctx& C, uint64_t listword, uint32_t* arg) {
+  uint32_t rest = hi32(listword);
+  if (rest == 0) return false;
+  uint64_t rw = nword(C, rest);
+  if (hi32(rw) != 0) return false;
+  *arg = lo32(rw);
+  return true;
+}
+
 // ---- the machine ---------------------------------------------------------------------------------------
-enum KKind : uint32_t { KF_HEAD = 1, KF_ARGS, KF_BODY, KF_IF, KF_LET, KF_DEFINE, KF_MACRO, KF_PAR, KF_DATA,
+enum KKind : uint32_t { KF_HEAD = 1, KF_ARGS, KF_BODY, KF_IF, KF_LET, KF_DEFINE, KF_MACRO, KF_PAR, KF_DATA, KF_QQ,
                        KF_JOIN, KF_SETQ };   // KF_JOIN: a KF_ARGS frame whose next argument was split off
 
 // ---- argument splitting ----------------------------------------------------------------
@@ -1044,7 +1064,7 @@ __device__ __forceinline__ FormOut eval_form(const Ctx& C, uint32_t root, uint32
   const bool fanout = FANOUT && !APPLY && C.A->fanout;
   V v = mkv(K_NIL, 0), a0 = mkv(K_NIL, 0), a1 = mkv(K_NIL, 0);
   uint32_t x = root, t = 0, env = env0, d = d0, cur = 0, base = 0, cnt = 0, sp = 0, vtop = 0;
-  uint32_t a = 0, at = 0, nxt = 0, kd = 0, hop = 0;
+  uint32_t a = 0, at = 0, nxt = 0, kd = 0, hop = 0, qlev = 0;
   uint64_t w = 0, aw = 0, w0 = 0;
   uint64_t steps = 0;
   uint8_t err = 0;
@@ -1268,6 +1288,13 @@ HEAD:
         d = d + 1;
         goto EVAL_NODE;
       }
+      case SP_QUASIQUOTE:                                       // R8: walk the template (cold code below)
+        x = car_of(C, cur);
+        qlev = 1;
+        goto QQ_NODE;
+      case SP_UNQUOTE:
+      case SP_UNQUOTE_SPLICING:
+        FAIL(E_SYNTAX);                                         // only meaningful inside a template
       default: {                                                // defun / defmacro
         w0 = nword(C, cur);
         uint32_t s = (uint32_t)nword(C, lo32(w0));
@@ -1457,6 +1484,7 @@ RET_POP:
     case KF_MACRO: goto RET_MACRO;
     case KF_PAR: goto RET_PAR;
     case KF_DATA: goto RET_DATA;
+    case KF_QQ: goto RET_QQ;
     default:
       FAIL(E_SYNTAX);
   }
@@ -1711,6 +1739,98 @@ DATA_LOOP: {
   vtop = base;
   v = mkv(K_CONS, s);
   goto RET;
+}
+
+  // ======================================================== quasiquote template walk (R8)
+  // QQ_NODE: template node x at level qlev; its value returns to the top continuation.  A template list is
+  // rebuilt on the V-stack (header at base: element count when a KF_QQ frame is pushed; elements above)
+  // and then copied into a fresh contiguous spine.  d stays the quasiquote form's depth; unquoted
+  // expressions are evaluated at d + 1.  The walk itself takes no steps.
+QQ_NODE: {
+    uint32_t tt;
+    uint64_t tw;
+    ldnode(C, x, tt, tw);
+    if ((tt & KIND_MASK) != K_CONS) { v = unbox_loaded(x, tt, tw); goto RET; }
+    if (__builtin_expect(!!(!(tt & TAG_PROPER)), 0)) FAIL(E_SYNTAX);
+    uint32_t op = qq_op(C, tw), arg = 0;
+    if (op == SP_UNQUOTE && qlev == 1) {
+      if (!qq_arg(C, tw, &arg)) FAIL(E_SYNTAX);
+      x = arg; d = d + 1;
+      goto EVAL_NODE;                                           // (tail: the value returns to our caller)
+    }
+    if (op == SP_UNQUOTE_SPLICING && qlev == 1) FAIL(E_SYNTAX);   // not in an element position
+    hop = qlev;                                                 // level of the elements after the head
+    if (op != 0xffu) {
+      if (!qq_arg(C, tw, &arg)) FAIL(E_SYNTAX);
+      hop = op == SP_QUASIQUOTE ? qlev + 1 : qlev - 1;
+    }
+    if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
+    base = vtop;
+    vtop = base + 1;
+    cur = x;
+    goto QQ_LIST;
+}
+QQ_LIST:                                                        // element `cur` next, at level qlev
+  while (cur != 0) {
+    w0 = nword(C, cur);
+    a = lo32(w0);
+    nxt = hi32(w0);
+    ldnode(C, a, at, aw);
+    if ((at & KIND_MASK) != K_CONS) {                           // an atom: itself
+      if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
+      *VS(C, vtop) = vpack(unbox_loaded(a, at, aw), 0);
+      ++vtop;
+      cur = nxt;
+      qlev = hop;
+      continue;
+    }
+    VS(C, base)->x = vtop - base - 1;                           // elements so far
+    if (qlev == 1 && qq_op(C, aw) == SP_UNQUOTE_SPLICING) {     // evaluate, then splice
+      uint32_t arg;
+      if (!(at & TAG_PROPER) || !qq_arg(C, aw, &arg)) FAIL(E_SYNTAX);
+      KPUSH(KF_QQ, nxt, env, base, d, hop | 0x100u);
+      x = arg; d = d + 1;
+      goto EVAL_NODE;
+    }
+    KPUSH(KF_QQ, nxt, env, base, d, hop);                       // a sub-template
+    x = a;
+    goto QQ_NODE;
+  }
+  {
+    uint32_t n = vtop - base - 1, s;
+    if (n == 0) {
+      v = mkv(K_NIL, 0);
+    } else {
+      if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &s)), 0)) FAIL(E_OOM);
+      for (uint32_t i = 0; i < n; ++i) {
+        uint32_t ca = box_into(H, vunpack(*VS(C, base + 1 + i)), s + n + i);
+        H.tag[s + i] = K_CONS | TAG_PROPER;
+        H.word[s + i] = pack2(ca, i + 1 < n ? s + i + 1 : 0);
+      }
+      v = mkv(K_CONS, s);
+    }
+    vtop = base;
+    goto RET;
+  }
+RET_QQ: {                                                       // an element's value (or a list to splice)
+    base = k.z;
+    cur = k.x; env = k.y; d = kd;
+    hop = kcount(k.w) & 0xffu;
+    qlev = hop;
+    vtop = base + 1 + VS(C, base)->x;
+    if (kcount(k.w) & 0x100u) {
+      if (__builtin_expect(!!(!proper_value(C, v)), 0)) FAIL(E_TYPE);
+      for (uint32_t c = v.t == K_NIL ? 0 : (uint32_t)v.w; c != 0; c = cdr_of(C, c)) {
+        if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
+        *VS(C, vtop) = vpack(unbox(C, car_of(C, c)), 0);
+        ++vtop;
+      }
+    } else {
+      if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
+      *VS(C, vtop) = vpack(v, 0);
+      ++vtop;
+    }
+    goto QQ_LIST;
 }
 
   // ======================================================== ||| : start element i (frame in ktop)

@@ -535,3 +535,44 @@ def test_defun_definitions(culi, oracle_mod):
     assert ctx.eval_batch("(h 3)").printed() == ["81"]
     ctx.define("(defun sq (x) (+ x x))")
     assert ctx.eval_batch("(h 3)").printed() == ["12"]
+
+
+def test_quasiquote(culi, oracle_mod):
+    """Quasiquote (reading R8): the hand-derived pins, random templates with unquote,
+    unquote-splicing and nesting, and macros written with templates — host reader and device reader."""
+    rows = _tsv("quasiquote_pins.tsv")
+    rnd = random.Random(21)
+
+    def tmpl(d):
+        k = rnd.randint(0, 6 if d < 3 else 2)
+        if k == 0:
+            return str(rnd.randint(-9, 9))
+        if k == 1:
+            return rnd.choice(["a", "b", "nil", "T", '"s"', "2.5"])
+        if k == 2:
+            return ",(+ %d x)" % rnd.randint(-5, 5)
+        if k == 3:
+            return "(unquote-splicing (list %d x))" % rnd.randint(0, 3)
+        if k == 4:
+            return "`(q %s)" % tmpl(d + 1)
+        if k == 5:
+            return "(unquote-splicing %s)" % rnd.choice(["nil", "5", "'(1 2)", "(cons 1 2)"])
+        return "(%s)" % " ".join(tmpl(d + 1) for _ in range(rnd.randint(0, 4)))
+
+    forms = [r[0] for r in rows] + ["(let ((x %d)) `%s)" % (rnd.randint(-3, 3), tmpl(0)) for _ in range(600)]
+    defs = "\n".join([
+        "(defmacro my-if (c a b) `(if ,c ,a ,b))",
+        "(defmacro swap (a b) `(list ,b ,a))",
+        "(defmacro my-let1 (v e body) `((lambda (,v) ,body) ,e))",
+        "(defmacro build (n) `(list (unquote-splicing (list n n)) ,n))",
+        "(define k 7)"])
+    forms += ["(my-if (< %d 0) 'neg 'nonneg)" % v for v in range(-3, 3)]
+    forms += ["(swap 1 2)", "(my-let1 y (+ 1 2) (* y y))", "`(k ,k)", "(build 4)"]
+    text = "\n".join(forms)
+    gp, gs, _ = assert_parity(culi, oracle_mod, defs, text)
+    for r, p, st in zip(rows, gp, gs):
+        assert (p, st) == (r[1], int(r[2])), r
+    ctx = culi.Context(**SMALL)
+    ctx.define_text(defs)
+    r = ctx.eval_text(text)
+    assert (r.printed(), r.steps()) == (gp, gs)

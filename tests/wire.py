@@ -12,6 +12,7 @@ import struct
 
 MAGIC = 0x31534552494C5543
 RESERVED = ["quote", "if", "define", "defun", "defmacro", "lambda", "let", "progn", "setq",
+            "quasiquote", "unquote", "unquote-splicing",
             "+", "-", "*", "/", "rem", "mod", "sqrt", "float", "trunc",
             "=", "<", ">", "<=", ">=", "eq", "equal", "null", "not",
             "atom", "consp", "numberp", "symbolp", "cons", "car", "cdr", "list",
