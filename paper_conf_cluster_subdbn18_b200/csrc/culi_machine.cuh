@@ -814,6 +814,38 @@ __device__ __forceinline__ bool qq_arg(const Ctx& C, uint64_t listword, uint32_t
   return true;
 }
 
+// try_leaf out of line (CULI_LEAF_CALL=1): one copy of the leaf evaluator (and of the symbol lookups it
+// inlines) instead of four — the machine is instruction-fetch bound, at the price of a call.
+#ifndef CULI_LEAF_CALL
+#define CULI_LEAF_CALL 0
+#endif
+struct LeafOut {
+  V v;
+  uint64_t steps;
+  int kind;
+  uint8_t err;
+};
+__device__ __noinline__ LeafOut try_leaf_call(Ctx C, uint32_t xt, uint64_t xw, uint32_t dx, uint32_t env,
+                                              uint64_t steps, uint64_t fuel, uint32_t maxd) {
+  LeafOut o;
+  o.steps = steps;
+  o.err = 0;
+  o.v = mkv(K_NIL, 0);
+  o.kind = try_leaf(C, xt, xw, dx, env, o.steps, fuel, maxd, &o.v, &o.err);
+  return o;
+}
+#if CULI_LEAF_CALL
+#define TRY_LEAF(res, outv)                                                               \
+  do {                                                                                    \
+    LeafOut lo_ = try_leaf_call(C, at, aw, d + 1, env, steps, fuel, maxd);                \
+    res = lo_.kind;                                                                       \
+    steps = lo_.steps;                                                                    \
+    if (res == 1) outv = lo_.v; else if (res == 2) err = lo_.err;                         \
+  } while (0)
+#else
+#define TRY_LEAF(res, outv) res = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &outv, &err)
+#endif
+
 // ---- the machine ---------------------------------------------------------------------------------------
 enum KKind : uint32_t { KF_HEAD = 1, KF_ARGS, KF_BODY, KF_IF, KF_LET, KF_DEFINE, KF_MACRO, KF_PAR, KF_DATA, KF_QQ,
                        KF_JOIN, KF_SETQ };   // KF_JOIN: a KF_ARGS frame whose next argument was split off
@@ -1195,7 +1227,7 @@ HEAD:
       int leaf = 0;
       V av;
       if ((at & KIND_MASK) == K_CONS) {
-        leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &av, &err);
+        TRY_LEAF(leaf, av);
         if (__builtin_expect(leaf == 2, 0)) goto done;
       } else {
         av = ATOMVAL(a, at, aw);
@@ -1234,6 +1266,7 @@ HEAD:
       if (__builtin_expect(!!(!C.A->define_mode), 0)) FAIL(E_DEFINE_IN_BATCH);
     }
     if (__builtin_expect(!!(!(t & TAG_VALID) && !special_syntax_ok(C, op, cur)), 0)) FAIL(E_SYNTAX);
+    if (__builtin_expect(op >= SP_QUASIQUOTE, 0)) goto QQ_SPECIAL;   // R8 (cold code below)
     switch (op) {
       case SP_IF: {
         w0 = nword(C, cur);
@@ -1242,7 +1275,8 @@ HEAD:
         ldnode(C, a, at, aw);
         STEP(d + 1);
         if ((at & KIND_MASK) == K_CONS) {
-          int leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &v, &err);
+          int leaf;
+          TRY_LEAF(leaf, v);
           if (__builtin_expect(leaf == 2, 0)) goto done;
           if (leaf == 0) {
             KPUSH(KF_IF, c1, env, vtop, d, 0);
@@ -1288,13 +1322,6 @@ HEAD:
         d = d + 1;
         goto EVAL_NODE;
       }
-      case SP_QUASIQUOTE:                                       // R8: walk the template (cold code below)
-        x = car_of(C, cur);
-        qlev = 1;
-        goto QQ_NODE;
-      case SP_UNQUOTE:
-      case SP_UNQUOTE_SPLICING:
-        FAIL(E_SYNTAX);                                         // only meaningful inside a template
       default: {                                                // defun / defmacro
         w0 = nword(C, cur);
         uint32_t s = (uint32_t)nword(C, lo32(w0));
@@ -1326,7 +1353,8 @@ ARGS:
     STEP(d + 1);
     V av;
     if ((at & KIND_MASK) == K_CONS) {
-      int leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &av, &err);
+      int leaf;
+      TRY_LEAF(leaf, av);
       if (__builtin_expect(leaf == 2, 0)) goto done;
       if (leaf == 0) {
         vtop = base + 1 + cnt;
@@ -1689,7 +1717,8 @@ LET_LOOP:
     STEP(d + 1);
     V lv;
     if ((at & KIND_MASK) == K_CONS) {
-      int leaf = try_leaf(C, at, aw, d + 1, env, steps, fuel, maxd, &lv, &err);
+      int leaf;
+      TRY_LEAF(leaf, lv);
       if (__builtin_expect(leaf == 2, 0)) goto done;
       if (leaf == 0) {
         vtop = base + 1 + cnt;
@@ -1746,6 +1775,11 @@ DATA_LOOP: {
   // rebuilt on the V-stack (header at base: element count when a KF_QQ frame is pushed; elements above)
   // and then copied into a fresh contiguous spine.  d stays the quasiquote form's depth; unquoted
   // expressions are evaluated at d + 1.  The walk itself takes no steps.
+QQ_SPECIAL:                                                     // (quasiquote t); unquote forms: SYNTAX
+  if (v.w != SP_QUASIQUOTE) FAIL(E_SYNTAX);                     // only meaningful inside a template
+  x = car_of(C, cur);
+  qlev = 1;
+  // fallthrough
 QQ_NODE: {
     uint32_t tt;
     uint64_t tw;
