@@ -183,6 +183,7 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
     sgword[i] = A.H.gword[i];
     sgtag[i] = A.H.gtag[i];
   }
+  alloc_init();
   if (SPLIT && threadIdx.x < 4) {
     culi_split_busy[threadIdx.x] = 0;
     culi_warp_idle[threadIdx.x] = 0;
@@ -296,6 +297,7 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_vote_kernel
     sgword[i] = A.H.gword[i];
     sgtag[i] = A.H.gtag[i];
   }
+  alloc_init();
   __syncthreads();
   uint32_t slot = blockIdx.x * blockDim.x + threadIdx.x;
   Ctx C = make_ctx(A, slot);
@@ -345,6 +347,7 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_vote_kernel
 // global frame; stops at the first error.  No staging: this kernel writes globals.
 __global__ void culi_define_kernel(const __grid_constant__ EvalArgs A) {
   if (blockIdx.x != 0 || threadIdx.x != 0) return;
+  alloc_init();
   Ctx C = make_ctx(A, 0);
   for (uint32_t f = 0; f < A.nforms; ++f) {
     FormOut o = eval_form<false, false>(C, A.roots[f], f, 0, 0, A.fuel);
@@ -462,6 +465,7 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_fanout_kernel(co
     sgword[i] = A.H.gword[i];
     sgtag[i] = A.H.gtag[i];
   }
+  alloc_init();
   __syncthreads();
   uint32_t slot = blockIdx.x * blockDim.x + threadIdx.x;
   uint32_t nthreads = gridDim.x * blockDim.x;

@@ -125,8 +125,28 @@ __device__ __forceinline__ uint32_t car_of(const Ctx& C, uint32_t c) { return lo
 __device__ __forceinline__ uint32_t cdr_of(const Ctx& C, uint32_t c) { return hi32(nword(C, c)); }
 
 // Warp-aggregated bump allocation (north_star; "the sequentially next free node"):
-// lanes asking for the same size in the same instruction share one atomicAdd (__match_any_sync) and
-// receive adjacent ranges, so their node stores coalesce.
+// lanes asking for the same size in the same instruction share one allocation (__match_any_sync) and
+// receive adjacent ranges, so their node stores coalesce.  Small requests come from a per-warp chunk in
+// shared memory (one shared atomic; the global bump pointer is touched once per ALLOC_CHUNK nodes), so
+// allocation-heavy batches (C4's macro expansions) do not serialise on one global counter.  The chunk
+// word packs next | end << 32 (heap indices are < 2^31); a request that overflows the chunk takes a fresh
+// one from the global pointer and installs it with one exchange — no retry loop, so nothing spins
+// between the two collectives.  Every kernel that allocates zeroes culi_alloc first.
+constexpr uint32_t ALLOC_CHUNK = 512;
+__shared__ unsigned long long culi_alloc[4];
+__device__ __forceinline__ void alloc_init() {
+  if ((threadIdx.x & 31) == 0 && threadIdx.x < 128) culi_alloc[threadIdx.x >> 5] = 0;
+}
+__device__ __forceinline__ unsigned long long alloc_range(const DevHeap& H, unsigned long long need) {
+  if (need > ALLOC_CHUNK / 4) return atomicAdd(H.top, need);
+  unsigned long long* s = &culi_alloc[threadIdx.x >> 5];
+  unsigned long long old = atomicAdd(s, need);
+  unsigned long long next = old & 0xffffffffull, end = old >> 32;
+  if (next + need <= end) return next;
+  unsigned long long b = atomicAdd(H.top, (unsigned long long)ALLOC_CHUNK);
+  if (b + ALLOC_CHUNK <= H.cap) atomicExch(s, ((b + ALLOC_CHUNK) << 32) | (b + need));
+  return b;
+}
 __device__ __forceinline__ bool heap_alloc(const DevHeap& H, uint32_t n, uint32_t* out) {
   unsigned mask = __activemask();
   // (& mask: a lane group of another call converged onto this instruction must not leak into the result,
@@ -136,7 +156,7 @@ __device__ __forceinline__ bool heap_alloc(const DevHeap& H, uint32_t n, uint32_
   int leader = __ffs(peers) - 1;
   unsigned rank = __popc(peers & ((1u << lane) - 1u));
   unsigned long long base = 0;
-  if (lane == leader) base = atomicAdd(H.top, (unsigned long long)n * (unsigned)__popc(peers));
+  if (lane == leader) base = alloc_range(H, (unsigned long long)n * (unsigned)__popc(peers));
   base = __shfl_sync(peers, base, leader);
   unsigned long long mine = base + (unsigned long long)rank * n;
   if (mine + n > H.cap) return false;
