@@ -35,7 +35,7 @@ def build(verbose: bool = False, force: bool = False, ptxas_v: bool = False, def
     deps = [os.path.join(CSRC, f) for f in os.listdir(CSRC)] + [os.path.join(ROOT, "include", "culi.h")]
     if not force and not _stale(LIB, deps):
         return LIB
-    objs = []
+    objs, cmds = [], []
     for src in SOURCES:
         obj = os.path.join(CSRC, src + ".o")
         cmd = [NVCC, *ARCH, *FLAGS, "-c", os.path.join(CSRC, src), "-o", obj]
@@ -43,8 +43,9 @@ def build(verbose: bool = False, force: bool = False, ptxas_v: bool = False, def
             cmd += ["-Xptxas", "-v"]
         if verbose:
             print(" ".join(cmd), file=sys.stderr)
-        subprocess.check_call(cmd)
+        cmds.append(cmd)
         objs.append(obj)
+    _compile_all(cmds)
     cmd = [NVCC, *ARCH, "-shared", "-o", LIB, *objs, "-lcudart"]
     subprocess.check_call(cmd)
     for o in objs:
@@ -52,17 +53,26 @@ def build(verbose: bool = False, force: bool = False, ptxas_v: bool = False, def
     return LIB
 
 
+def _compile_all(cmds: list[list[str]]) -> None:
+    """Translation units compile in parallel (one nvcc per unit); any failure raises."""
+    from concurrent.futures import ThreadPoolExecutor
+    with ThreadPoolExecutor(max_workers=max(1, min(len(cmds), os.cpu_count() or 1))) as ex:
+        for f in [ex.submit(subprocess.check_call, c) for c in cmds]:
+            f.result()
+
+
 def _build_variant(defines: list[str], out: str, verbose: bool) -> str:
     import tempfile
     tmp = tempfile.mkdtemp()
-    objs = []
+    objs, cmds = [], []
     for src in SOURCES:
         obj = os.path.join(tmp, src + ".o")
         cmd = [NVCC, *ARCH, *FLAGS, *["-D" + d for d in defines], "-c", os.path.join(CSRC, src), "-o", obj]
         if verbose:
             print(" ".join(cmd), file=sys.stderr)
-        subprocess.check_call(cmd)
+        cmds.append(cmd)
         objs.append(obj)
+    _compile_all(cmds)
     subprocess.check_call([NVCC, *ARCH, "-shared", "-o", out, *objs, "-lcudart"])
     return out
 

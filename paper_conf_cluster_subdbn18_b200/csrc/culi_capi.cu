@@ -268,6 +268,36 @@ static bool image_mentions_par(const Image& img, bool skip_root_heads = false) {
     if ((img.tag[k] & KIND_MASK) == K_CONS && !root[k] && (uint32_t)img.word[k] == par) return true;
   return false;
 }
+// Is there a wide list (a data list or (list ...) with >= WIDE_MIN elements after its head) below the top
+// level that is not the operand of a quote?  Its evaluation may suspend (nested mode, NEST_EVAL).  Reader
+// spines are contiguous (c.14): cell k continues a list iff cell k-1 is a cons whose cdr is k.
+static bool image_has_wide_nested(const Image& img) {
+  size_t N = img.tag.size();
+  std::vector<char> skip(N, 0);
+  for (uint32_t r : img.roots)
+    if (r >= IMG_FIRST) skip[r - IMG_FIRST] = 1;
+  auto is_cons = [&](size_t k) { return (img.tag[k] & KIND_MASK) == K_CONS; };
+  for (size_t k = 0; k < N; ++k) {                    // (quote x): x is not evaluated
+    if (!is_cons(k)) continue;
+    uint32_t h = (uint32_t)img.word[k], c2 = (uint32_t)(img.word[k] >> 32);
+    if (h < IMG_FIRST || (img.tag[h - IMG_FIRST] & KIND_MASK) != K_SYM || img.word[h - IMG_FIRST] != SP_QUOTE) continue;
+    if (c2 < IMG_FIRST || !is_cons(c2 - IMG_FIRST)) continue;
+    uint32_t x = (uint32_t)img.word[c2 - IMG_FIRST];
+    if (x >= IMG_FIRST) skip[x - IMG_FIRST] = 1;
+  }
+  size_t start = 0, run = 0;
+  for (size_t k = 0; k < N; ++k) {
+    if (!is_cons(k)) { run = 0; continue; }
+    if (run && (uint32_t)(img.word[k - 1] >> 32) == IMG_FIRST + k) {
+      ++run;
+    } else {
+      start = k;
+      run = 1;
+    }
+    if (run == WIDE_MIN + 1 && !skip[start]) return true;
+  }
+  return false;
+}
 static bool image_mentions_setq(const Image& img) {
   for (size_t k = 0; k < img.tag.size(); ++k)
     if ((img.tag[k] & KIND_MASK) == K_SYM && img.word[k] == SP_SETQ) return true;
@@ -430,7 +460,7 @@ extern "C" int culi_define(culi_ctx* c, const culi_image* defs, uint32_t* failed
   int rc = upload_image(c, img, str_base);
   if (rc) return rc;
   c->strings += img.strings;
-  c->persist_has_par = c->persist_has_par || image_mentions_par(img);
+  c->persist_has_par = c->persist_has_par || image_mentions_par(img) || image_has_wide_nested(img);
   c->persist_has_closure = c->persist_has_closure || image_mentions_closure(img);
   c->define_mut = c->persist_has_setq || image_mentions_setq(img);
   c->persist_has_setq = c->define_mut;
@@ -445,7 +475,7 @@ extern "C" int culi_define_text(culi_ctx* c, const char* text, size_t len, int t
   int rc = device_read(c, text, len, text_on_device != 0, &ro, err_offset);
   if (rc) return rc;
   c->strings += ro.strings;
-  c->persist_has_par = c->persist_has_par || ro.par_root_head || ro.par_nested;
+  c->persist_has_par = c->persist_has_par || ro.par_root_head || ro.par_nested || ro.wide_nested;
   c->persist_has_closure = c->persist_has_closure || ro.closure;
   c->define_mut = c->persist_has_setq || ro.setq;
   c->persist_has_setq = c->define_mut;
@@ -577,8 +607,9 @@ static int prepare_batch(culi_ctx* c, const Image& img) {
     CK(c->wide.ensure(nf));
     CK(cudaMemcpyAsync(c->wide.p, wide.data(), nf * 4, cudaMemcpyHostToDevice, c->stream));
   }
-  return finish_prepare(c, nf, img.tag.size(), img.strings, image_mentions_par(img, false),
-                        image_mentions_par(img, true), par_head, has_wide, image_mentions_setq(img),
+  bool wide_nested = image_has_wide_nested(img);      // (counts as a nested ||| for the launch mode)
+  return finish_prepare(c, nf, img.tag.size(), img.strings, image_mentions_par(img, false) || wide_nested,
+                        image_mentions_par(img, true) || wide_nested, par_head, has_wide, image_mentions_setq(img),
                         image_mentions_closure(img));
 }
 
@@ -587,8 +618,9 @@ static int prepare_text(culi_ctx* c, const char* text, size_t len, bool on_devic
   ReadOut ro;
   int rc = device_read(c, text, len, on_device, &ro, err_offset);
   if (rc) return rc;
-  return finish_prepare(c, ro.nforms, ro.nodes, std::move(ro.strings), ro.par_root_head || ro.par_nested,
-                        ro.par_nested, ro.par_root_head, ro.wide, ro.setq, ro.closure);
+  return finish_prepare(c, ro.nforms, ro.nodes, std::move(ro.strings),
+                        ro.par_root_head || ro.par_nested || ro.wide_nested, ro.par_nested || ro.wide_nested,
+                        ro.par_root_head, ro.wide, ro.setq, ro.closure);
 }
 
 // ||| forms the fan-out could not decide (an element error, fuel overflow, a short or non-contiguous

@@ -128,7 +128,14 @@ constexpr uint8_t E_SUSPEND = 0xfc;
 // Warp voting (north_star "ballot for branch voting"): a lane group that diverged yields
 // at a return; the kernel re-forms groups by (stack height, continuation kind) and resumes the deepest.
 constexpr uint8_t E_YIELD = 0xfb;
-struct NestDesc {
+// NEST_WIDE: a wide list — a data list or (list a1..an) with at least WIDE_MIN elements to evaluate —
+// reached below the top level suspends the same way (kind NEST_EVAL): element i is the expression in
+// cell heads[0] + i, evaluated in the heap environment env at depth+1; its value goes to spine cell
+// off + i of the ncells-cell result spine (cell 0 of a data list holds the head value already).
+enum NestKind : uint32_t { NEST_APPLY = 0, NEST_EVAL = 1 };
+// The claim counter and the completion counters sit in lines of their own: every idle thread of the grid
+// polls `ready`/`next` while the element threads update `done`/`total`.
+struct alignas(128) NestDesc {
   uint32_t form, n, m, spine;
   uint32_t ftag, depth;
   uint64_t fword;
@@ -136,8 +143,11 @@ struct NestDesc {
   uint64_t top;
   uint32_t heads[FANOUT_MAXM];
   uint32_t sp, vtop;
-  unsigned long long total;
-  uint32_t next, done, bad, ready;            // ready: fields published, elements claimable
+  uint32_t kind, env, off, ncells;            // NEST_EVAL only (kind NEST_APPLY: 0)
+  uint32_t ready;                             // fields published, elements claimable
+  alignas(128) uint32_t next;                 // elements claimed
+  alignas(128) unsigned long long total;      // sum of element steps
+  uint32_t done, bad;
 };
 
 // Argument splitting.  When idle warps wait for work, the lanes of a busy warp that poll

@@ -52,15 +52,58 @@ __device__ __forceinline__ Ctx make_ctx(const EvalArgs& A, uint32_t slot) {
 // Runs on the thread's secondary stacks (C2).  Element i: f applied to (l1[i] .. lm[i]) at the depth of the
 // ||| call, with the fuel left when the owner suspended.  A failed contiguity check or an element error
 // marks the descriptor bad (the owner's form is then re-evaluated sequentially, exactly).
+#if CULI_NEST_TRACE
+// debug: [0] first claim, [1] last element done, [2] owner resumed, [3] owner suspended (min/max globaltimer)
+__device__ unsigned long long culi_nest_trace[8];
+extern "C" int culi_debug_nest_trace(unsigned long long* out) {
+  return cudaMemcpyFromSymbol(out, culi_nest_trace, sizeof(culi_nest_trace)) == cudaSuccess ? 0 : 1;
+}
+extern "C" int culi_debug_nest_trace_reset() {
+  unsigned long long z[8] = {~0ull, 0, 0, ~0ull, 0, 0, 0, 0};
+  return cudaMemcpyToSymbol(culi_nest_trace, z, sizeof(z)) == cudaSuccess ? 0 : 1;
+}
+#define NTRACE_MIN(k) atomicMin(&culi_nest_trace[k], gtime())
+#define NTRACE_MAX(k) atomicMax(&culi_nest_trace[k], gtime())
+#define NTRACE_ADD(k, v) atomicAdd(&culi_nest_trace[k], (unsigned long long)(v))
+#else
+#define NTRACE_MIN(k) do { } while (0)
+#define NTRACE_MAX(k) do { } while (0)
+#define NTRACE_ADD(k, v) do { } while (0)
+#endif
 __device__ __forceinline__ bool nest_run_one(const EvalArgs& A, const Ctx& C2, NestDesc* D) {
   if (*(volatile uint32_t*)&D->ready == 0) return false;
   uint32_t n = D->n;
   if (*(volatile uint32_t*)&D->next >= n) return false;
-  uint32_t i = atomicAdd(&D->next, 1u);
+  uint32_t i = fetch_add_grouped(&D->next);           // (one atomic per warp and descriptor)
   if (i >= n) return false;
+  NTRACE_MIN(0);
+  NTRACE_ADD(4, 1);
   const DevHeap& H = A.H;
   uint32_t m = D->m, spine = D->spine;
   bool ok = true;
+  if (D->kind == NEST_EVAL) {                           // wide list: evaluate element expression i
+    uint32_t c = D->heads[0] + i, nc = D->ncells, cell = D->off + i;
+    uint32_t tc = H.tag[c];
+    uint64_t wc = H.word[c];
+    if ((uint64_t)c >= D->top || (tc & KIND_MASK) != K_CONS || (i + 1 < n && hi32(wc) != c + 1)) {
+      atomicOr(&D->bad, 1u);
+    } else {
+      FormOut o = eval_form<false, false>(C2, lo32(wc), D->form, 0, 0, A.fuel - D->steps0, D->depth + 1,
+                                          false, Resume{}, D->env);
+      if (o.err) {
+        atomicOr(&D->bad, 2u);
+      } else {
+        uint32_t ca = box_into(H, mkv(o.t, o.w), spine + nc + cell);
+        H.tag[spine + cell] = K_CONS | TAG_PROPER;
+        H.word[spine + cell] = pack2(ca, cell + 1 < nc ? spine + cell + 1 : 0);
+        atomicAdd(&D->total, (unsigned long long)o.steps);
+      }
+    }
+    __threadfence();
+    atomicAdd(&D->done, 1u);
+    NTRACE_MAX(1);
+    return true;
+  }
   *VS(C2, 0) = vpack(mkv(D->ftag, D->fword), 0);
   for (uint32_t j = 0; j < m; ++j) {
     uint32_t c = D->heads[j] + i;
@@ -243,6 +286,7 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
       o = eval_form<FANOUT, false, NEST, SPLIT>(C, root, f, 0, 0, fuel, d, resume, R, env);
       if (!NEST || o.err != E_SUSPEND) break;
       NestDesc* D = A.ndesc + o.aux;                    // suspended on a nested |||: help until done
+      NTRACE_MIN(3);
       unsigned long long t0 = 0;
       while (*(volatile uint32_t*)&D->done < D->n) {
         if (nest_help_any(A, C2, D)) { t0 = 0; continue; }
@@ -258,6 +302,7 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
         o.err = E_PENDING;
         break;
       }
+      NTRACE_MAX(2);
       R.sp = D->sp;
       R.vtop = D->vtop;
       R.steps = s;
@@ -276,8 +321,12 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
     }
   }
   if (NEST) {                                           // no forms left: help until every form is done
-    while (*(volatile uint32_t*)A.finished < A.nforms)
-      if (!nest_help_any(A, C2, nullptr)) __nanosleep(256);
+    uint32_t ns = 128;                                  // (back off while there is nothing to claim: the
+    while (*(volatile uint32_t*)A.finished < A.nforms) {  //  whole grid polls the same descriptors)
+      if (nest_help_any(A, C2, nullptr)) { ns = 128; continue; }
+      __nanosleep(ns);
+      ns = ns * 2 > 2048 ? 2048 : ns * 2;
+    }
   }
 }
 

@@ -124,6 +124,35 @@ __device__ __forceinline__ V unbox(const Ctx& C, uint32_t n) {
 __device__ __forceinline__ uint32_t car_of(const Ctx& C, uint32_t c) { return lo32(nword(C, c)); }
 __device__ __forceinline__ uint32_t cdr_of(const Ctx& C, uint32_t c) { return hi32(nword(C, c)); }
 
+// Length of the cdr chain from c (the count loop of a data list / list).  Reader spines are contiguous
+// (c.14), so the next 16 cells are loaded before their links are checked (branch-free, so all loads are in
+// flight together: one L2 round trip per 16 cells instead of one per cell); a link that leaves the run
+// restarts the scan there, so exactly the same chain is walked.  Out of line: its registers stay out of
+// the eval loop's allocation.
+__device__ CULI_COLD uint32_t chain_length(Ctx C, uint32_t c) {
+  uint32_t n = 0;
+  const uint64_t cap = C.A->H.cap;
+  const uint64_t* word = C.A->H.word;
+  while (c != 0) {
+    if ((c & 1u) || (uint64_t)c + 16 > cap) { ++n; c = cdr_of(C, c); continue; }
+    // 16 cells per round trip: 8 aligned 16-byte loads, links checked afterwards (all loads in flight)
+    uint32_t q[16];
+#pragma unroll
+    for (int k = 0; k < 8; ++k) {
+      uint4 v = *reinterpret_cast<const uint4*>(word + c + 2 * k);
+      q[2 * k] = v.y;
+      q[2 * k + 1] = v.w;
+    }
+    uint32_t brk = 0, nx = c + 16;
+#pragma unroll
+    for (int k = 15; k >= 0; --k)
+      if (q[k] != c + k + 1) { brk |= 1u << k; nx = q[k]; }       // the lowest break wins
+    n += brk ? __ffs(brk) : 16;
+    c = nx;
+  }
+  return n;
+}
+
 // Warp-aggregated bump allocation (north_star; "the sequentially next free node"):
 // lanes asking for the same size in the same instruction share one allocation (__match_any_sync) and
 // receive adjacent ranges, so their node stores coalesce.  Small requests come from a per-warp chunk in
@@ -920,6 +949,20 @@ __device__ __forceinline__ uint32_t fetch_add_lanes32(uint32_t* p) {
   return base + rank;
 }
 
+// fetch_add_lanes32 for lanes that may address different counters: the lanes executing it together are
+// grouped by address (__match_any_sync, restricted to the caller's mask), one atomic per group.
+__device__ __forceinline__ uint32_t fetch_add_grouped(uint32_t* p) {
+  unsigned mask = __activemask();
+  unsigned peers = __match_any_sync(mask, (unsigned long long)p) & mask;
+  int lane = threadIdx.x & 31;
+  int leader = __ffs(peers) - 1;
+  unsigned rank = __popc(peers & ((1u << lane) - 1u));
+  uint32_t base = 0;
+  if (lane == leader) base = atomicAdd(p, (uint32_t)__popc(peers));
+  base = __shfl_sync(peers, base, leader);
+  return base + rank;
+}
+
 // A bounded wait gave up: count it and keep the first occurrence's state for diagnosis.
 // Every wait on another lane is bounded by EvalArgs.wait_ns, so a protocol bug shows up as a counter and a
 // status (culi_last_waits), never as a frozen GPU.
@@ -1624,7 +1667,13 @@ MACRO_CALL: {
 DATA_START: {
     bool data = v.t != K_BUILTIN;
     uint32_t n = data ? 1 : 0;
-    for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
+    if (NEST) {                                                 // (batches with wide lists run NEST)
+      uint32_t c = cur;
+      for (uint32_t k = 0; k < 16 && c != 0; ++k, ++n) c = cdr_of(C, c); // short lists inline;
+      if (c != 0) n += chain_length(C, c);                              // long ones 16 cells per load round
+    } else {
+      for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
+    }
     if (n == 0) { v = mkv(K_NIL, 0); goto RET; }
     uint32_t s;
     if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &s)), 0)) FAIL(E_OOM);
@@ -1632,6 +1681,44 @@ DATA_START: {
       uint32_t ca = box_into(H, v, s + n);
       H.tag[s] = K_CONS | TAG_PROPER;
       H.word[s] = pack2(ca, n > 1 ? s + 1 : 0);
+    }
+    if (NEST && !APPLY && C.A->nest && n - (data ? 1 : 0) >= WIDE_MIN) {
+      // a wide list below the top level (K12 "per warp for wide forms", §8(f)1): suspend; any thread
+      // evaluates element i in a heap copy of env (frames are immutable, c.3) into spine cell off + i,
+      // then we resume at RET with the spine (steps: the sum over the elements, as in DATA_LOOP)
+      uint32_t henv;
+      if (__builtin_expect(!!(!promote(C, env, &henv)), 0)) FAIL(E_OOM);
+      uint32_t slot = atomicAdd(C.A->nnest, 1u);
+      if (slot < C.A->maxnest) {
+        NestDesc* D = C.A->ndesc + slot;
+        D->form = form;
+        D->n = n - (data ? 1 : 0);
+        D->m = 0;
+        D->spine = s;
+        D->ftag = 0;
+        D->depth = d;
+        D->fword = 0;
+        D->steps0 = steps;
+        D->top = atomicAdd(H.top, 0ull);
+        D->heads[0] = cur;
+        D->sp = sp;
+        D->vtop = vtop;
+        D->kind = NEST_EVAL;
+        D->env = henv;
+        D->off = data ? 1 : 0;
+        D->ncells = n;
+        D->total = 0;
+        D->bad = 0;
+        D->done = 0;
+        D->next = 0;
+        __threadfence();
+        atomicExch(&D->ready, 1u);                              // publish: elements may be claimed
+        if (kdirty) *KS(C, sp - 1) = ktop;                      // the resume reloads the top frame
+        v = mkv(K_CONS, s);
+        aux = slot;
+        err = E_SUSPEND;
+        goto done;
+      }
     }
     if (__builtin_expect(!!(vtop >= vcap), 0)) FAIL(E_OOM);
     base = vtop;
@@ -1699,6 +1786,7 @@ PAR_APPLY: {
           for (uint32_t j = 0; j < cnt - 2; ++j) D->heads[j] = (uint32_t)arg(C, base, 2 + j).w;
           D->sp = sp;
           D->vtop = base;
+          D->kind = NEST_APPLY;
           D->total = 0;
           D->bad = 0;
           D->done = 0;

@@ -42,12 +42,15 @@ constexpr uint32_t RF_PAR_NESTED = 2;            // ||| is the car of some other
 constexpr uint32_t RF_WIDE = 4;                  // some top-level form has >= WIDE_MIN arguments
 constexpr uint32_t RF_SETQ = 8;                  // the setq symbol occurs (R7)
 constexpr uint32_t RF_CLOSURE = 16;              // lambda or defun occurs: closures may exist
+constexpr uint32_t RF_WIDE_NESTED = 32;          // a list below the top level, not a quote's operand, has
+                                                 // >= WIDE_MIN elements after its head (NEST_EVAL)
 
 struct ReadOut {
   uint32_t nforms = 0;
   uint32_t nodes = 0;
   std::string strings;           // the batch's string bytes (host mirror, for printing)
   bool par_root_head = false, par_nested = false, wide = false, setq = false, closure = false;
+  bool wide_nested = false;
 };
 
 // Parse `len` bytes (host or device pointer) into the heap at ctx->mark, the form table into ctx->roots

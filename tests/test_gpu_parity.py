@@ -403,6 +403,64 @@ def test_nested_par_limits(culi, oracle_mod):
                       oracle_kw=dict(fuel=fuel, max_depth=depth))
 
 
+WIDE_DEFS = "\n".join([W.FIB_DEF, W.FACT_DEF,
+    "(define wsq (lambda (k) (list %s)))" % " ".join("(* k %d)" % i for i in range(70)),
+    "(define wdat (lambda (a b) (5 %s)))" % " ".join(("a", "b", "(+ a b)", "(fib a)", "'q", "2.5")[i % 6]
+                                                     for i in range(90)),
+    "(define wbad (lambda (a) (list %s)))" % " ".join(("(car a)" if i in (40, 60) else str(i)) for i in range(80)),
+    "(define wq (lambda () '(%s)))" % " ".join(str(i) for i in range(100))])
+
+
+def _wide(n, elem="5"):
+    return "(%s)" % " ".join([elem] * n)
+
+
+def test_wide_lists_below_top_level(culi, oracle_mod):
+    """Wide data lists and (list a1..an) below the top level (>= WIDE_MIN elements): the
+    evaluation suspends and any thread evaluates the elements (NEST_EVAL) — in a function body (stack
+    environment, promoted to the heap), as a ||| argument (the paper-shaped C0), nested in each other, with
+    element errors (exact sequential fallback: the first error in order) and under fuel/depth limits."""
+    forms = ["(||| 100 fib %s)" % _wide(100), "(||| 64 fib %s)" % _wide(64), "(||| 63 fib %s)" % _wide(63),
+             "(length (wsq 3))", "(wsq 7)", "(wdat 6 7)", "(car (cdr (wdat 10 2)))",
+             "(wbad '(1 2))", "(wbad 5)", "(wq)", "(length (list %s))" % " ".join("(fib %d)" % (i % 15) for i in range(200)),
+             "(list 1 %s 2)" % _wide(80, "(+ 1 2)"), "(+ 1 (length %s))" % _wide(300, "(fact 5)"),
+             "(||| 3 + (1 2 3) (list %s))" % " ".join(str(i) for i in range(65)),
+             "(let ((x 4)) (list %s))" % " ".join("(* x %d)" % i for i in range(66)),
+             "(%s)" % " ".join(["(fib 10)"] * 65), "(1 %s)" % " ".join(["(undefined-f 1)"] * 70)] * 2
+    text = "\n".join(forms)
+    assert_parity(culi, oracle_mod, WIDE_DEFS, text)
+    ctx = culi.Context(**SMALL)
+    ctx.define(WIDE_DEFS)
+    r = ctx.eval_batch(text)
+    fan, fb = ctx.last_stats()
+    assert ctx.last_nested >= 2 * 10 and fb >= 2, (fan, fb, ctx.last_nested)
+    ctx2 = culi.Context(**SMALL, flags=culi.CULI_F_NO_NESTED)
+    ctx2.define(WIDE_DEFS)
+    r2 = ctx2.eval_batch(text)
+    assert r.printed() == r2.printed() and r.steps() == r2.steps()
+    # the same through the device reader (its RF_WIDE_NESTED flag selects the launch mode)
+    ctx3 = culi.Context(**SMALL)
+    ctx3.define_text(WIDE_DEFS)
+    r3 = ctx3.eval_text(text)
+    ctx3.last_stats()
+    assert r3.printed() == r.printed() and r3.steps() == r.steps() and ctx3.last_nested >= 2 * 10
+    for fuel, depth in ((3000, 1024), (1 << 40, 4), (1 << 40, 3)):
+        assert_parity(culi, oracle_mod, WIDE_DEFS, text, ctx_kw=dict(fuel=fuel, max_depth=depth),
+                      oracle_kw=dict(fuel=fuel, max_depth=depth))
+
+
+def test_c0_paper_shape_full(culi, oracle_mod):
+    """C0 at its bench size ((||| 4096 fib (5 5 ... 5))): the data list is evaluated by the
+    whole grid, the elements fan out; value and steps equal the oracle's."""
+    wl = W.c0(4096)
+    assert_parity(culi, oracle_mod, wl.defs, wl.forms)
+    ctx = culi.Context(**SMALL)
+    ctx.define(wl.defs)
+    ctx.eval_batch(wl.forms)
+    ctx.last_stats()
+    assert ctx.last_nested == 1
+
+
 @pytest.mark.parametrize("n", [1, 2, 4095, 4096, 4097])
 def test_small_batch_dispatch_boundary(culi, oracle_mod, n):
     """Batches of <= 4096 forms run in input order, larger ones through the binning permutation
