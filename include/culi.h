@@ -63,8 +63,8 @@ typedef struct {
   int device;              /* CUDA device ordinal                                                       */
   void* stream;            /* cudaStream_t (e.g. torch.cuda.current_stream().cuda_stream); NULL = the
                               legacy default stream.  Borrowed: must outlive the ctx.                    */
-  uint64_t heap_nodes;     /* node capacity of the SoA heap (tag u8 + word u64 per node); 0 = default
-                              (64 Mi nodes = 576 MB).  The paper's node array was fixed at compile time
+  uint64_t heap_nodes;     /* node capacity of the heap (16-byte nodes: word u64 + tag u8, loaded with one
+                              16-byte access); 0 = default (64 Mi nodes = 1 GiB).  The paper's node array was fixed at compile time
                               (L361-365); here it is sized at init.                                     */
   uint32_t max_depth;      /* canonical eval-nesting limit (c.10); 0 = default 1024; at most 4095         */
   uint64_t fuel;           /* canonical step limit per top-level form (c.10); 0 = default 2^40            */
@@ -77,7 +77,7 @@ typedef struct {
   uint64_t heap_bytes;     /* size of heap_base; at least culi_arena_bytes(opts) (CULI_E_ARG otherwise)   */
 } culi_opts;
 
-/* Bytes of device memory a ctx with these opts places in heap_base (heap tag + word arrays, the global
+/* Bytes of device memory a ctx with these opts places in heap_base (the heap's node array, the global
  * frame, the string area, K- and V-stacks; SURVEY §8(d) "heap and stack budget").  The remaining session
  * state (counters, descriptors, result buffers) stays library-allocated. */
 int culi_arena_bytes(const culi_opts* opts, uint64_t* bytes);
@@ -85,7 +85,8 @@ int culi_arena_bytes(const culi_opts* opts, uint64_t* bytes);
 #define CULI_F_NO_BINNING 1u   /* evaluate forms in input order (no classify+sort dispatch, §8(a)5)     */
 #define CULI_F_NO_FANOUT  2u   /* evaluate top-level ||| forms in one thread (no fan-out, §8(a)6)        */
 #define CULI_F_NO_STAGING 4u   /* do not stage the global frame / hot code in shared memory (§8(a)4)     */
-#define CULI_F_NO_VOTING  8u   /* reserved (no effect in this version)                                   */
+#define CULI_F_NO_VOTING  8u   /* batches that neither split nor nest: plain kernel instead of the warp-voting
+                                  one (lanes regroup by stack height + continuation at returns) */
 #define CULI_F_NO_NESTED 16u   /* run nested (non-top-level) ||| forms inside one thread (§8(f)1 off)     */
 #define CULI_F_NO_SPLIT  32u   /* no argument splitting: each form is evaluated by one thread only        */
 #define CULI_F_NO_GC     64u   /* do not compact the persistent heap segment after culi_define (§8(f)3)  */

@@ -32,17 +32,17 @@ static void drop_graph(culi_ctx* c) {
   c->graph_exec = nullptr;
 }
 
-// Caller-owned arena (culi_opts.heap_base): heap tag + word, global frame, string area, K- and V-stacks,
-// each 256-byte aligned, in this order.
+// Caller-owned arena (culi_opts.heap_base): heap nodes (16 B each), global frame tag + word, string area,
+// K- and V-stacks, each 256-byte aligned, in this order.
 struct ArenaLayout {
-  size_t off[7];
+  size_t off[6];
   size_t total;
 };
 static ArenaLayout arena_layout(uint64_t heap_nodes, uint64_t str_cap, size_t nslots, size_t kcap, size_t vcap) {
-  size_t sz[7] = {heap_nodes, heap_nodes * 8, GCAP, (size_t)GCAP * 8, str_cap, nslots * kcap * 16, nslots * vcap * 16};
+  size_t sz[6] = {heap_nodes * sizeof(Node), GCAP, (size_t)GCAP * 8, str_cap, nslots * kcap * 16, nslots * vcap * 16};
   ArenaLayout L{};
   size_t o = 0;
-  for (int k = 0; k < 7; ++k) {
+  for (int k = 0; k < 6; ++k) {
     L.off[k] = o;
     o = (o + sz[k] + 255) & ~(size_t)255;
   }
@@ -129,16 +129,18 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
     if (o.heap_bytes < L.total || ((uintptr_t)o.heap_base & 255)) { delete c; return CULI_E_ARG; }
     char* b = (char*)o.heap_base;
     c->arena_owned = false;
-    c->H.tag = (uint8_t*)(b + L.off[0]);
-    c->H.word = (uint64_t*)(b + L.off[1]);
-    c->H.gtag = (uint8_t*)(b + L.off[2]);
-    c->H.gword = (uint64_t*)(b + L.off[3]);
-    c->H.strs = (const char*)(b + L.off[4]);
-    c->kst = (uint4*)(b + L.off[5]);
-    c->vst = (uint4*)(b + L.off[6]);
+    c->H.tag = TagArr{(Node*)(b + L.off[0])};
+    c->H.word = WordArr{c->H.tag.p};
+    c->H.gtag = (uint8_t*)(b + L.off[1]);
+    c->H.gword = (uint64_t*)(b + L.off[2]);
+    c->H.strs = (const char*)(b + L.off[3]);
+    c->kst = (uint4*)(b + L.off[4]);
+    c->vst = (uint4*)(b + L.off[5]);
   } else {
-    ok &= cudaMalloc(&c->H.tag, o.heap_nodes) == cudaSuccess;
-    ok &= cudaMalloc(&c->H.word, o.heap_nodes * 8) == cudaSuccess;
+    Node* nodes = nullptr;
+    ok &= cudaMalloc(&nodes, o.heap_nodes * sizeof(Node)) == cudaSuccess;
+    c->H.tag = TagArr{nodes};
+    c->H.word = WordArr{nodes};
     ok &= cudaMalloc(&c->H.gtag, GCAP) == cudaSuccess;
     ok &= cudaMalloc(&c->H.gword, (size_t)GCAP * 8) == cudaSuccess;
     ok &= cudaMalloc((void**)&c->H.strs, c->str_cap) == cudaSuccess;
@@ -162,10 +164,8 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   c->H.cap = o.heap_nodes;
   c->H.gcap = GCAP;
   // nil and T nodes; every symbol unbound; builtins are resolved by id (reserved names)
-  uint8_t t01[2] = {K_NIL, K_T};
-  uint64_t w01[2] = {0, 0};
-  bool ok2 = cudaMemcpyAsync(c->H.tag, t01, 2, cudaMemcpyHostToDevice, c->stream) == cudaSuccess &&
-             cudaMemcpyAsync(c->H.word, w01, 16, cudaMemcpyHostToDevice, c->stream) == cudaSuccess &&
+  static const Node n01[2] = {Node{0, K_NIL, {}}, Node{0, K_T, {}}};
+  bool ok2 = cudaMemcpyAsync(c->H.tag.p, n01, sizeof(n01), cudaMemcpyHostToDevice, c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->H.gtag, K_UNBOUND, GCAP, c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->flags, 0, 8 * sizeof(int), c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->groups, 0xff, (size_t)c->nslots / 32 * SPLIT_GPW * sizeof(SplitGroup), c->stream) == cudaSuccess &&
@@ -185,8 +185,7 @@ void culi_shutdown(culi_ctx* c) {
     c->pending = nullptr;
   }
   if (c->arena_owned) {
-    cudaFree(c->H.tag);
-    cudaFree(c->H.word);
+    cudaFree(c->H.tag.p);
     cudaFree(c->H.gtag);
     cudaFree(c->H.gword);
     cudaFree((void*)c->H.strs);
@@ -387,15 +386,18 @@ static int upload_image(culi_ctx* c, const Image& img, uint32_t str_base) {
   if ((uint64_t)str_base + img.strings.size() > c->str_cap) return CULI_E_HEAP_FULL;
   uint32_t nr = (uint32_t)img.roots.size();
   CK(c->roots.ensure(std::max<uint32_t>(nr, 1)));
+  size_t tw = (n + 7) / 8;                           // staging: word[] at [0, n), tag[] after it
   if (n) {
-    CK(cudaMemcpyAsync(c->H.tag + c->mark, img.tag.data(), n, cudaMemcpyHostToDevice, c->stream));
-    CK(cudaMemcpyAsync(c->H.word + c->mark, img.word.data(), n * 8, cudaMemcpyHostToDevice, c->stream));
+    CK(c->stage.ensure(n + tw));
+    CK(cudaMemcpyAsync(c->stage.p, img.word.data(), n * 8, cudaMemcpyHostToDevice, c->stream));
+    CK(cudaMemcpyAsync(c->stage.p + n, img.tag.data(), n, cudaMemcpyHostToDevice, c->stream));
   }
   if (!img.strings.empty())
     CK(cudaMemcpyAsync((char*)c->H.strs + str_base, img.strings.data(), img.strings.size(),
                        cudaMemcpyHostToDevice, c->stream));
   if (nr) CK(cudaMemcpyAsync(c->roots.p, img.roots.data(), nr * 4, cudaMemcpyHostToDevice, c->stream));
-  CK(launch_relocate(c->stream, c->H.tag, c->H.word, c->mark, n, str_base, c->roots.p, nr, c->sms));
+  CK(launch_relocate(c->stream, (const uint8_t*)(c->stage.p + n), c->stage.p, c->H.tag.p, c->mark, n, str_base,
+                     c->roots.p, nr, c->sms));
   return CULI_OK;
 }
 

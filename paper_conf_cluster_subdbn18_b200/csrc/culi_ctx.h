@@ -124,6 +124,7 @@ struct culi_ctx {
   int* flags = nullptr;             // [0] oom [1] define fail idx+1 [2] define err [3] payload ovf [4] export ovf
   DevBuf<uint32_t> roots, keys, keys_alt, perm, perm_alt;
   DevBuf<uint8_t> rtag, rerr, dtemp;
+  DevBuf<uint64_t> stage;             // host image (SoA tag + word) before the relocate kernel interleaves it
   DevBuf<uint64_t> rsteps, rword;
   DevBuf<uint4> payload;
   // ||| fan-out state

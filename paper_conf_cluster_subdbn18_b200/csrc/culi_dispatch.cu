@@ -23,7 +23,7 @@ namespace culi {
 // Shape of a form: FNV-1a over a pre-order walk of its first 48 nodes — node kinds, symbol ids, list
 // structure; numbers contribute only their kind (their values are in the hint).  Forms with equal shape
 // expand macros and take calls in the same order, so a warp of them stays converged longer (C4).
-__device__ uint32_t shape_hash(const uint8_t* __restrict__ tag, const uint64_t* __restrict__ word, uint32_t x) {
+__device__ uint32_t shape_hash(TagArr tag, WordArr word, uint32_t x) {
   uint32_t st[12];
   int sp = 0;
   uint32_t h = 2166136261u;
@@ -50,7 +50,7 @@ __device__ uint32_t shape_hash(const uint8_t* __restrict__ tag, const uint64_t* 
 
 static_assert(16 + N_RESERVED <= 64, "reserved-operator token codes fit in 6 bits");
 // Pre-order token stream of a form, most significant first: 6 bits per token, the first five tokens.
-__device__ uint64_t structure_prefix(const uint8_t* __restrict__ tag, const uint64_t* __restrict__ word, uint32_t x) {
+__device__ uint64_t structure_prefix(TagArr tag, WordArr word, uint32_t x) {
   uint32_t st[8];
   int sp = 0, n = 0;
   uint64_t key = 0;
@@ -80,7 +80,7 @@ __device__ uint64_t structure_prefix(const uint8_t* __restrict__ tag, const uint
   return key;
 }
 
-__global__ void culi_classify_kernel(const uint8_t* __restrict__ tag, const uint64_t* __restrict__ word,
+__global__ void culi_classify_kernel(TagArr tag, WordArr word,
                                      const uint32_t* __restrict__ roots, uint32_t nforms,
                                      unsigned long long* __restrict__ keys, uint32_t* __restrict__ perm) {
   uint32_t stride = gridDim.x * blockDim.x;

@@ -37,11 +37,10 @@ struct EnvHeader {
 inline uint64_t align8(uint64_t x) { return (x + 7) & ~7ull; }
 
 struct EnvLayout {
-  uint64_t o_tag, o_word, o_gtag, o_gword, o_str, o_names, total;
+  uint64_t o_node, o_gtag, o_gword, o_str, o_names, total;
   EnvLayout(const EnvHeader& h) {
-    o_tag = sizeof(EnvHeader);
-    o_word = align8(o_tag + h.mark);
-    o_gtag = o_word + 8 * h.mark;
+    o_node = (sizeof(EnvHeader) + 15) & ~15ull;     // the persistent segment's 16-byte nodes, verbatim
+    o_gtag = o_node + sizeof(Node) * h.mark;
     o_gword = align8(o_gtag + h.nsyms);
     o_str = o_gword + 8 * h.nsyms;
     o_names = o_str + h.nstr;
@@ -90,8 +89,7 @@ int culi_env_export(culi_ctx* c, void* dev_buf, size_t cap, size_t* bytes) {
   if (!dev_buf || cap < L.total) return dev_buf ? CULI_E_ARG : CULI_OK;
   char* d = (char*)dev_buf;
   CK(cudaMemcpyAsync(d, &h, sizeof h, cudaMemcpyHostToDevice, c->stream));
-  CK(cudaMemcpyAsync(d + L.o_tag, c->H.tag, h.mark, cudaMemcpyDeviceToDevice, c->stream));
-  CK(cudaMemcpyAsync(d + L.o_word, c->H.word, 8 * h.mark, cudaMemcpyDeviceToDevice, c->stream));
+  CK(cudaMemcpyAsync(d + L.o_node, c->H.tag.p, sizeof(Node) * h.mark, cudaMemcpyDeviceToDevice, c->stream));
   CK(cudaMemcpyAsync(d + L.o_gtag, c->H.gtag, h.nsyms, cudaMemcpyDeviceToDevice, c->stream));
   CK(cudaMemcpyAsync(d + L.o_gword, c->H.gword, 8 * h.nsyms, cudaMemcpyDeviceToDevice, c->stream));
   if (h.nstr) CK(cudaMemcpyAsync(d + L.o_str, c->H.strs, h.nstr, cudaMemcpyDeviceToDevice, c->stream));
@@ -115,8 +113,7 @@ int culi_env_import(culi_ctx* c, const void* dev_buf, size_t nbytes) {
   std::string names(h.names_bytes, '\0');
   if (h.names_bytes)
     CK(cudaMemcpyAsync(&names[0], d + L.o_names, h.names_bytes, cudaMemcpyDeviceToHost, c->stream));
-  CK(cudaMemcpyAsync(c->H.tag, d + L.o_tag, h.mark, cudaMemcpyDeviceToDevice, c->stream));
-  CK(cudaMemcpyAsync(c->H.word, d + L.o_word, 8 * h.mark, cudaMemcpyDeviceToDevice, c->stream));
+  CK(cudaMemcpyAsync(c->H.tag.p, d + L.o_node, sizeof(Node) * h.mark, cudaMemcpyDeviceToDevice, c->stream));
   CK(cudaMemcpyAsync(c->H.gtag, d + L.o_gtag, h.nsyms, cudaMemcpyDeviceToDevice, c->stream));
   CK(cudaMemcpyAsync(c->H.gword, d + L.o_gword, 8 * h.nsyms, cudaMemcpyDeviceToDevice, c->stream));
   if (h.nstr) CK(cudaMemcpyAsync((char*)c->H.strs, d + L.o_str, h.nstr, cudaMemcpyDeviceToDevice, c->stream));

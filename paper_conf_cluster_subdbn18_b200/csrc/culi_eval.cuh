@@ -1,4 +1,4 @@
-// culi_eval.cuh — device side of libculi.so: SoA heap access, warp-aggregated bump allocator,
+// culi_eval.cuh — device side of libculi.so: heap access (16-byte nodes), warp-aggregated bump allocator,
 // environment lookup, and the explicit-stack (non-recursive) eval/apply machine.  sm_100a only.
 //
 // The paper's evaluator is a recursive tree walk using CUDA device recursion (§III-B.c,
@@ -33,8 +33,8 @@ constexpr uint32_t STACK_ENV = 0x80000000u;   // env reference into the thread's
 #endif
 
 struct DevHeap {
-  uint8_t* tag;
-  uint64_t* word;
+  TagArr tag;                  // views of the node array (struct Node, culi_internal.h): tag.p == word.p
+  WordArr word;
   unsigned long long* top;     // bump pointer (node index)
   uint64_t cap;                // node capacity
   uint8_t* gtag;               // global frame: direct-indexed by symbol id (identity hash)
@@ -200,8 +200,8 @@ constexpr uint32_t WAIT_JOIN = 1, WAIT_QUEUE = 2, WAIT_NEST = 3;
 #endif
 
 struct ExportArgs {
-  const uint8_t* tag;
-  const uint64_t* word;
+  TagArr tag;
+  WordArr word;
   uint8_t* rtag;
   uint64_t* rword;
   uint32_t nforms;
@@ -216,8 +216,8 @@ struct ExportArgs {
 };
 
 // host-side launchers (culi_kernels.cu, culi_dispatch.cu)
-cudaError_t launch_relocate(cudaStream_t s, uint8_t* tag, uint64_t* word, uint64_t base, uint64_t n,
-                            uint32_t str_base, uint32_t* roots, uint32_t nroots, int sms);
+cudaError_t launch_relocate(cudaStream_t s, const uint8_t* stag, const uint64_t* sword, Node* nodes, uint64_t base,
+                            uint64_t n, uint32_t str_base, uint32_t* roots, uint32_t nroots, int sms);
 cudaError_t launch_eval(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
 cudaError_t launch_define(cudaStream_t s, const EvalArgs& A);
 cudaError_t launch_export(cudaStream_t s, const ExportArgs& X, uint32_t blocks);

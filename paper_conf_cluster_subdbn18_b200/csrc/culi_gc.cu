@@ -29,8 +29,8 @@ constexpr uint32_t REFS = (1u << K_STR) | (1u << K_CONS) | (1u << K_CLOSURE) | (
 constexpr uint32_t STRUCT = (1u << K_CONS) | (1u << K_CLOSURE) | (1u << K_MACRO) | (1u << K_FRAME);
 
 struct Args {
-  const uint8_t* tag;
-  const uint64_t* word;
+  TagArr tag;                   // views of the heap's node array
+  WordArr word;
   uint64_t mark;
   uint32_t* role;               // per node of [0, mark)
   const uint32_t* in;           // frontier of this round
@@ -117,8 +117,8 @@ __device__ __forceinline__ uint32_t fwd(const uint32_t* pos, uint32_t y) {
 }
 
 // live node i -> scratch[pos[i]], references remapped
-__global__ void copy_kernel(const uint8_t* tag, const uint64_t* word, const uint32_t* role, const uint32_t* pos,
-                            uint64_t mark, uint8_t* stag, uint64_t* sword) {
+__global__ void copy_kernel(TagArr tag, WordArr word, const uint32_t* role, const uint32_t* pos,
+                            uint64_t mark, TagArr stag, WordArr sword) {
   for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < mark; i += (uint64_t)gridDim.x * blockDim.x) {
     uint32_t r = role[i];
     if (i < IMG_FIRST || r == R_DEAD) continue;
@@ -208,10 +208,8 @@ int collect_persistent(culi_ctx* c, uint64_t* live_out, uint64_t* freed_out) {
   if (mark + live > c->H.cap) return CULI_OK;           // no scratch room: keep the segment as it is
   copy_kernel<<<blocks, 256, 0, st>>>(c->H.tag, c->H.word, S.role.p, S.pos.p, mark, c->H.tag + mark, c->H.word + mark);
   GK(cudaGetLastError());
-  if (live) {
-    GK(cudaMemcpyAsync(c->H.tag + IMG_FIRST, c->H.tag + mark, live, cudaMemcpyDeviceToDevice, st));
-    GK(cudaMemcpyAsync(c->H.word + IMG_FIRST, c->H.word + mark, (size_t)live * 8, cudaMemcpyDeviceToDevice, st));
-  }
+  if (live)
+    GK(cudaMemcpyAsync(c->H.tag.p + IMG_FIRST, c->H.tag.p + mark, (size_t)live * sizeof(Node), cudaMemcpyDeviceToDevice, st));
   globals_kernel<<<blocks, 256, 0, st>>>(c->H.gtag, c->H.gword, nsyms, S.pos.p);
   GK(cudaGetLastError());
   GK(cudaStreamSynchronize(st));

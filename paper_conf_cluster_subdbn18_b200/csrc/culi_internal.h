@@ -1,10 +1,10 @@
 // culi_internal.h — internal layout shared by the host reader/printer and the device kernels of
 // libculi.so.  (Product code: never included by oracle/.)
 //
-// Heap: structure-of-arrays node pool in HBM (§III-A.c "nodes are stored in a large
-// array ... the sequentially next free node"; node = value + links, L288-293 §III-A.a Fig.1):
-//   tag[i]  : uint8   kind (low 4 bits) | CULI_TAG_PROPER (cons whose cdr chain ends in nil)
-//   word[i] : uint64  payload — INT int64 / FLOAT f64 bits / SYM id / STR off|len<<32 /
+// Heap: node pool in HBM (§III-A.c "nodes are stored in a large array ... the sequentially
+// next free node"; node = value + links, L288-293 §III-A.a Fig.1), 16 bytes per node (struct Node):
+//   tag     : uint8   kind (low 4 bits) | CULI_TAG_PROPER (cons whose cdr chain ends in nil)
+//   word    : uint64  payload — INT int64 / FLOAT f64 bits / SYM id / STR off|len<<32 /
 //                     CONS car|cdr<<32 (node indices) / BUILTIN,SPECIAL op /
 //                     CLOSURE,MACRO code|env<<32 (code = cons (params . body), env = heap frame or 0) /
 //                     FRAME parent|n<<32 / BIND sym|valnode<<32
@@ -53,5 +53,26 @@ constexpr uint32_t IMG_FIRST = 2;
 #define CULI_HD inline
 #endif
 CULI_HD uint64_t pack2(uint32_t lo, uint32_t hi) { return (uint64_t)lo | ((uint64_t)hi << 32); }
+
+// Device heap node: payload and tag co-located in 16 bytes, so the device reads a node with one aligned
+// 16-byte load (north_star "coalesced, vectorised node loads"; culi_machine.cuh ldnode).  TagArr / WordArr
+// view the node array as the tag[] / word[] arrays the kernels index (node i's fields, 16 bytes apart).
+// Host images stay structure-of-arrays (9 B/node on the wire); the relocate kernel interleaves them.
+struct alignas(16) Node {
+  uint64_t word;
+  uint8_t tag;
+  uint8_t pad[7];
+};
+static_assert(sizeof(Node) == 16, "one 16-byte access per node");
+struct TagArr {
+  Node* p;
+  CULI_HD uint8_t& operator[](uint64_t i) const { return p[i].tag; }
+  CULI_HD TagArr operator+(uint64_t o) const { return TagArr{p + o}; }
+};
+struct WordArr {
+  Node* p;
+  CULI_HD uint64_t& operator[](uint64_t i) const { return p[i].word; }
+  CULI_HD WordArr operator+(uint64_t o) const { return WordArr{p + o}; }
+};
 
 }  // namespace culi

@@ -8,23 +8,25 @@
 
 namespace culi {
 
-// Relocate an uploaded image in place: image-local indices -> heap indices.
-__global__ void culi_relocate_kernel(uint8_t* tag, uint64_t* word, uint64_t base, uint64_t n,
+// Relocate an uploaded image into the heap: image-local indices -> heap indices, and
+// interleave the image's tag[] / word[] arrays (staged in HBM) into 16-byte nodes (one store per node).
+__global__ void culi_relocate_kernel(const uint8_t* __restrict__ stag, const uint64_t* __restrict__ sword,
+                                     Node* nodes, uint64_t base, uint64_t n,
                                      uint32_t str_base, uint32_t* roots, uint32_t nroots) {
   uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
   for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
     uint64_t g = base + i;
-    uint32_t t = tag[g] & KIND_MASK;
+    uint32_t tg = stag[i], t = tg & KIND_MASK;
+    uint64_t w = sword[i];
     if (t == K_CONS) {
-      uint64_t w = word[g];
       uint32_t a = lo32(w), b = hi32(w);
       a = a < IMG_FIRST ? a : (uint32_t)(base + a - IMG_FIRST);
       b = b < IMG_FIRST ? b : (uint32_t)(base + b - IMG_FIRST);
-      word[g] = pack2(a, b);
+      w = pack2(a, b);
     } else if (t == K_STR) {
-      uint64_t w = word[g];
-      word[g] = pack2(lo32(w) + str_base, hi32(w));
+      w = pack2(lo32(w) + str_base, hi32(w));
     }
+    *reinterpret_cast<uint4*>(nodes + g) = make_uint4(lo32(w), hi32(w), tg, 0);
   }
   for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < nroots; i += stride) {
     uint32_t r = roots[i];
@@ -666,13 +668,13 @@ __global__ void culi_flat_commit_kernel(const __grid_constant__ EvalArgs A) {
 }
 
 // ---- host launchers ----------------------------------------------------------------------------------
-cudaError_t launch_relocate(cudaStream_t s, uint8_t* tag, uint64_t* word, uint64_t base, uint64_t n,
-                            uint32_t str_base, uint32_t* roots, uint32_t nroots, int sms) {
+cudaError_t launch_relocate(cudaStream_t s, const uint8_t* stag, const uint64_t* sword, Node* nodes, uint64_t base,
+                            uint64_t n, uint32_t str_base, uint32_t* roots, uint32_t nroots, int sms) {
   uint64_t work = n > nroots ? n : nroots;
   uint64_t blocks = (work + 255) / 256;
   if (blocks > (uint64_t)sms * 16) blocks = (uint64_t)sms * 16;
   if (blocks == 0) blocks = 1;
-  culi_relocate_kernel<<<(unsigned)blocks, 256, 0, s>>>(tag, word, base, n, str_base, roots, nroots);
+  culi_relocate_kernel<<<(unsigned)blocks, 256, 0, s>>>(stag, sword, nodes, base, n, str_base, roots, nroots);
   return cudaGetLastError();
 }
 

@@ -76,7 +76,7 @@ __device__ __forceinline__ const uint8_t* sm_gtag(const Ctx& C) {
   return reinterpret_cast<const uint8_t*>(sm_gword(C) + C.A->gst);
 }
 
-// ---- heap access (SoA: tag u8[], word u64[]) ------------------------------------------
+// ---- heap access (16-byte nodes {word, tag}, culi_internal.h) ------------------------------
 // CULI_STAGE_CODE=1 serves the persistent code segment from shared memory.  Measured on C2 (round 1):
 // the range check makes every node load execute both paths predicated (~25 % of all instructions),
 // which costs more than the L1 hits it replaces, so it is off by default; the global frame (one lookup
@@ -94,8 +94,9 @@ __device__ __forceinline__ void ldnode(const Ctx& C, uint32_t n, uint32_t& t, ui
     return;
   }
 #endif
-  t = C.A->H.tag[n];
-  w = C.A->H.word[n];
+  const uint4 q = *reinterpret_cast<const uint4*>(C.A->H.tag.p + n);   // one 16-byte load per node
+  t = q.z & 0xffu;
+  w = ((uint64_t)q.y << 32) | q.x;
 }
 __device__ __forceinline__ uint64_t nword(const Ctx& C, uint32_t n) {
 #if CULI_STAGE_CODE
@@ -132,17 +133,13 @@ __device__ __forceinline__ uint32_t cdr_of(const Ctx& C, uint32_t c) { return hi
 __device__ CULI_COLD uint32_t chain_length(Ctx C, uint32_t c) {
   uint32_t n = 0;
   const uint64_t cap = C.A->H.cap;
-  const uint64_t* word = C.A->H.word;
+  const Node* nodes = C.A->H.tag.p;
   while (c != 0) {
-    if ((c & 1u) || (uint64_t)c + 16 > cap) { ++n; c = cdr_of(C, c); continue; }
-    // 16 cells per round trip: 8 aligned 16-byte loads, links checked afterwards (all loads in flight)
+    if ((uint64_t)c + 16 > cap) { ++n; c = cdr_of(C, c); continue; }
+    // 16 cells per round trip: the cdr halves of 16 nodes, links checked afterwards (all loads in flight)
     uint32_t q[16];
 #pragma unroll
-    for (int k = 0; k < 8; ++k) {
-      uint4 v = *reinterpret_cast<const uint4*>(word + c + 2 * k);
-      q[2 * k] = v.y;
-      q[2 * k + 1] = v.w;
-    }
+    for (int k = 0; k < 16; ++k) q[k] = reinterpret_cast<const uint32_t*>(nodes + c + k)[1];
     uint32_t brk = 0, nx = c + 16;
 #pragma unroll
     for (int k = 15; k >= 0; --k)

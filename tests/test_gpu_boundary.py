@@ -63,8 +63,9 @@ def test_caller_owned_arena(culi, oracle_mod):
     ctx.define(wl.defs)
     r = ctx.eval_batch(wl.forms)
     assert not compare(r.printed(), r.steps(), _oracle(oracle_mod, wl.defs, wl.forms))
-    # the heap really lives in the caller's tensor: nil/T nodes at its start are tags 0 and 1
-    assert arena[:2].tolist() == [0, 1]
+    # the heap really lives in the caller's tensor: the nil / T nodes at its start (16-byte nodes
+    # {word u64, tag u8, pad}) carry tags 0 and 1
+    assert arena[8].item() == 0 and arena[24].item() == 1 and arena[:8].tolist() == [0] * 8
     small = torch.empty(need - 4096, dtype=torch.uint8, device="cuda")
     with pytest.raises(culi.CuliError) as ei:
         culi.Context(arena=small, **kw)
