@@ -82,7 +82,36 @@ class ClockSampler:
         self._stop = threading.Event()
         self._t = None
 
+    def _nvml_handle(self):
+        """NVML handle of the CUDA device (by PCI bus id, so CUDA_VISIBLE_DEVICES remapping is respected)."""
+        import pynvml
+        import torch
+        pynvml.nvmlInit()
+        try:
+            p = torch.cuda.get_device_properties(self.device)
+            bus = "%08x:%02x:%02x.0" % (p.pci_domain_id, p.pci_bus_id, p.pci_device_id)
+            return pynvml, pynvml.nvmlDeviceGetHandleByPciBusId(bus.encode())
+        except Exception:  # noqa: BLE001
+            return pynvml, pynvml.nvmlDeviceGetHandleByIndex(self.device)
+
     def _run(self):
+        # NVML every 5 ms (a 10-step C2 run gets ~130 samples); nvidia-smi every 0.2 s if NVML is missing
+        try:
+            nv, h = self._nvml_handle()
+            bits = (0x8, 0x40, 0x20, 0x4)     # hw_slowdown, hw_thermal, sw_thermal, sw_power_cap
+            mx = nv.nvmlDeviceGetMaxClockInfo(h, nv.NVML_CLOCK_SM)
+            get_r = getattr(nv, "nvmlDeviceGetCurrentClocksEventReasons", None) or \
+                nv.nvmlDeviceGetCurrentClocksThrottleReasons
+            self.source = "nvml 5 ms"
+            while not self._stop.is_set():
+                sm = nv.nvmlDeviceGetClockInfo(h, nv.NVML_CLOCK_SM)
+                r = get_r(h)
+                self.samples.append([str(sm), str(mx)] + ["Active" if r & b else "Not Active" for b in bits])
+                self._stop.wait(0.005)
+            return
+        except Exception:  # noqa: BLE001
+            pass
+        self.source = "nvidia-smi 0.2 s"
         while not self._stop.is_set():
             try:
                 out = subprocess.run(["nvidia-smi", "-i", str(self.device), "--query-gpu=" + self.Q,
@@ -112,7 +141,7 @@ class ClockSampler:
         reasons = sorted({names[k] for s in self.samples for k in range(4)
                           if len(s) > 2 + k and s[2 + k].lower() == "active"})
         return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
-                "reasons": reasons, "samples": len(self.samples)}
+                "reasons": reasons, "samples": len(self.samples), "source": getattr(self, "source", None)}
 
 
 def host_cpu_info():
