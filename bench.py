@@ -94,23 +94,23 @@ class ClockSampler:
         except Exception:  # noqa: BLE001
             return pynvml, pynvml.nvmlDeviceGetHandleByIndex(self.device)
 
+    def _nvml_sample(self):
+        nv, h, mx, get_r = self._nv
+        bits = (0x8, 0x40, 0x20, 0x4)         # hw_slowdown, hw_thermal, sw_thermal, sw_power_cap
+        sm = nv.nvmlDeviceGetClockInfo(h, nv.NVML_CLOCK_SM)
+        r = get_r(h)
+        self.samples.append([str(sm), str(mx)] + ["Active" if r & b else "Not Active" for b in bits])
+
     def _run(self):
-        # NVML every 5 ms (a 10-step C2 run gets ~130 samples); nvidia-smi every 0.2 s if NVML is missing
-        try:
-            nv, h = self._nvml_handle()
-            bits = (0x8, 0x40, 0x20, 0x4)     # hw_slowdown, hw_thermal, sw_thermal, sw_power_cap
-            mx = nv.nvmlDeviceGetMaxClockInfo(h, nv.NVML_CLOCK_SM)
-            get_r = getattr(nv, "nvmlDeviceGetCurrentClocksEventReasons", None) or \
-                nv.nvmlDeviceGetCurrentClocksThrottleReasons
-            self.source = "nvml 5 ms"
-            while not self._stop.is_set():
-                sm = nv.nvmlDeviceGetClockInfo(h, nv.NVML_CLOCK_SM)
-                r = get_r(h)
-                self.samples.append([str(sm), str(mx)] + ["Active" if r & b else "Not Active" for b in bits])
-                self._stop.wait(0.005)
+        # NVML every 5 ms (a 10-step C2 run gets ~130 samples; __enter__ / __exit__ add one sample each, so a
+        # timed region shorter than the period still has two); nvidia-smi every 0.2 s if NVML is missing
+        if self._nv:
+            while not self._stop.wait(0.005):
+                try:
+                    self._nvml_sample()
+                except Exception:  # noqa: BLE001
+                    pass
             return
-        except Exception:  # noqa: BLE001
-            pass
         self.source = "nvidia-smi 0.2 s"
         while not self._stop.is_set():
             try:
@@ -124,6 +124,16 @@ class ClockSampler:
             self._stop.wait(0.2)
 
     def __enter__(self):
+        self._nv = None
+        try:
+            nv, h = self._nvml_handle()
+            get_r = getattr(nv, "nvmlDeviceGetCurrentClocksEventReasons", None) or \
+                nv.nvmlDeviceGetCurrentClocksThrottleReasons
+            self._nv = (nv, h, nv.nvmlDeviceGetMaxClockInfo(h, nv.NVML_CLOCK_SM), get_r)
+            self.source = "nvml 5 ms"
+            self._nvml_sample()
+        except Exception:  # noqa: BLE001
+            self._nv = None
         self._t = threading.Thread(target=self._run, daemon=True)
         self._t.start()
         return self
@@ -131,6 +141,11 @@ class ClockSampler:
     def __exit__(self, *a):
         self._stop.set()
         self._t.join(timeout=10)
+        if self._nv:
+            try:
+                self._nvml_sample()
+            except Exception:  # noqa: BLE001
+                pass
 
     def summary(self):
         if not self.samples:
