@@ -261,6 +261,9 @@ def culi_arm(args):
     from paper_conf_cluster_subdbn18_b200 import build as B
 
     world = int(os.environ.get("WORLD_SIZE", "1"))
+    # CULI_FORCE_DIST=1: take the N > 1 path (process group, NCCL environment broadcast, device-resident
+    # result gather) even with one rank — exercises the collectives on a single GPU
+    dist_on = world > 1 or os.environ.get("CULI_FORCE_DIST") == "1"
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
     if world != args.gpus:
@@ -270,7 +273,7 @@ def culi_arm(args):
         local = 0
     backend = os.environ.get("CULI_DIST_BACKEND", "nccl")
     torch.cuda.set_device(local)
-    if world > 1:
+    if dist_on:
         if backend == "nccl":
             dist.init_process_group("nccl", device_id=torch.device("cuda", local))
         else:
@@ -296,7 +299,7 @@ def culi_arm(args):
 
     # ---- define on rank 0, broadcast the environment over NCCL (a3 + a10)
     t_env = None
-    if world == 1:
+    if not dist_on:
         if wl.defs:
             ctx.define(wl.defs)
     else:
@@ -320,7 +323,7 @@ def culi_arm(args):
     # NCCL all_gather moves the padded buffers; rank 0 can merge them on its GPU (culi_results_import, the
     # e2e path below).  The capacity is the largest exact size over the ranks (+25 %), from one eval.
     xcap, xbuf, gathered = 0, None, None
-    if world > 1:
+    if dist_on:
         from paper_conf_cluster_subdbn18_b200 import dist as D
         ctx.eval_uploaded(h)
         xcap = D.export_capacity(ctx)
@@ -329,7 +332,7 @@ def culi_arm(args):
 
     def step():
         ctx.eval_uploaded(h)
-        if world > 1:
+        if dist_on:
             ctx.results_export(xbuf.data_ptr(), xcap)
             if cdev.type == "cuda":
                 dist.all_gather_into_tensor(gathered, xbuf)
@@ -356,7 +359,7 @@ def culi_arm(args):
     ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
           for _ in range(args.steps)]
     eval_ms, disp_ms, exp_ms = [], [], []
-    if world > 1:
+    if dist_on:
         dist.barrier()
     torch.cuda.synchronize()
     with ClockSampler(local) as clk:
@@ -370,7 +373,7 @@ def culi_arm(args):
             eval_ms.append(ms3[1])
             exp_ms.append(ms3[2])
         torch.cuda.synchronize()
-    if world > 1:
+    if dist_on:
         dist.barrier()
     chk = ctx.fetch_results(h)                  # the timed steps' own results: same totals, no re-runs
     assert chk.totals() == (total_steps, n_err) and ctx.last_reruns() == (0, 0), ctx.last_reruns()
@@ -380,7 +383,7 @@ def culi_arm(args):
     step_ms = [a.elapsed_time(b) for a, b in ev]
     t_rank = sum(step_ms) / 1e3
     t_max = t_rank
-    if world > 1:
+    if dist_on:
         tt = torch.tensor([t_rank], dtype=torch.float64, device=cdev)
         dist.all_reduce(tt, op=dist.ReduceOp.MAX)
         t_max = float(tt.item())
@@ -403,7 +406,7 @@ def culi_arm(args):
         ms, nbytes = [], 0
         for k in range(args.e2e_steps):
             a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-            if world > 1:
+            if dist_on:
                 dist.barrier()
             a.record(stream)
             r = run()
@@ -414,14 +417,14 @@ def culi_arm(args):
             ms.append(a.elapsed_time(b))
             del r
         t = sum(ms) / 1e3
-        if world > 1:
+        if dist_on:
             tt = torch.tensor([t], dtype=torch.float64, device=cdev)
             dist.all_reduce(tt, op=dist.ReduceOp.MAX)
             t = float(tt.item())
         return units_all * len(ms) / t, 1e3 * t / len(ms), nbytes
 
     def e2e_text():
-        if world == 1:
+        if not dist_on:
             return ctx.eval_text(text_host)
         # N > 1: device read + eval of this rank's shard, device-resident gather, merge on rank 0's GPU,
         # one D2H of the whole batch's results there (no Python bytes on the path)
@@ -437,7 +440,7 @@ def culi_arm(args):
     # the same through a host-read image (culi_read outside the timed region, culi_eval_batch inside)
     img_h2d = img.pin()
     img_value, img_ms_step = None, None
-    if world == 1:
+    if not dist_on:
         img_value, img_ms_step, _ = e2e_loop(lambda: ctx.eval_batch(img))
 
     # ---- device reader alone (§8(f)2): text resident in HBM -> node image in the heap
@@ -459,7 +462,7 @@ def culi_arm(args):
               "timing": "CUDA events around the whole read incl. its 3 host sync points (culi_last_read)"}
 
     if rank != 0:
-        if world > 1:
+        if dist_on:
             dist.barrier()
             dist.destroy_process_group()
         return
@@ -524,7 +527,7 @@ def culi_arm(args):
         "cpu_baseline": cpu,
         "e2e": {"value": e2e_value, "unit": "forms/s", "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
                 "ms_per_step": e2e_ms_step,
-                "path": ("culi_eval_text: pinned host text -> device read -> eval -> host results" if world == 1
+                "path": ("culi_eval_text: pinned host text -> device read -> eval -> host results" if not dist_on
                          else "per rank: pinned host text -> device read -> eval -> culi_results_export -> NCCL "
                               "all_gather; rank 0: culi_results_import (device merge) -> host results")},
         "e2e_image": {"value": img_value, "unit": "forms/s", "h2d_bytes_per_step": img_h2d,
@@ -533,7 +536,7 @@ def culi_arm(args):
         "clocks": clocks,
     }
     print(json.dumps(line), flush=True)
-    if world > 1:
+    if dist_on:
         dist.barrier()
         dist.destroy_process_group()
 

@@ -86,3 +86,24 @@ def test_two_ranks_broadcast_shard_gather(oracle_mod):
         bad = compare(printed, steps, o, forms.splitlines())
         assert not bad, "\n".join(bad)
         assert (dprinted, dsteps) == (printed, steps)
+
+
+@pytest.mark.timeout(600)
+def test_bench_nccl_path_single_rank():
+    """bench.py's N > 1 path with the NCCL backend for real (one rank: the box has one GPU; CULI_FORCE_DIST):
+    process group over NCCL, environment broadcast, device-resident export + all_gather_into_tensor in the
+    timed step, the e2e gather + device merge on rank 0; the line must carry the distributed e2e path."""
+    import json
+    import subprocess
+    import sys
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    env = dict(os.environ, CULI_FORCE_DIST="1")
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", "--nproc-per-node", "1",
+           "--master-addr", "127.0.0.1", "--master-port", str(_free_port()), os.path.join(root, "bench.py"),
+           "--gpus", "1", "--workload", "C2", "--steps", "2", "--warmup", "3", "--e2e-steps", "1",
+           "--no-cpu-baseline"]
+    out = subprocess.run(cmd, capture_output=True, text=True, env=env, cwd=root, timeout=540)
+    assert out.returncode == 0, out.stderr[-3000:]
+    line = json.loads([x for x in out.stdout.splitlines() if x.startswith("{")][-1])
+    assert line["value"] > 0 and line["waits_gave_up"] == 0
+    assert "all_gather" in line["e2e"]["path"] and line["env_broadcast_ms"]["bytes"] > 0
