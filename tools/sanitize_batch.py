@@ -46,4 +46,14 @@ for _ in range(3):
 print(c4.fetch_results(h).totals())
 c4.release(h)
 c4.close()
+# nested ||| and wide lists below the top level (NEST_EVAL), incl. an element error
+c5 = culi.Context(slots=148 * 128, heap_nodes=1 << 22, vstack_entries=1024)
+c5.define(W.FIB_DEF + "\n(define pfib (lambda (xs) (||| (length xs) fib xs)))\n" +
+          "(define wl (lambda (k) (list %s)))" % " ".join("(* k %d)" % i for i in range(70)))
+wide = " ".join(["5"] * 300)
+r = c5.eval_batch("\n".join(["(||| 300 fib (%s))" % wide, "(length (wl 3))", "(pfib '(%s))" % wide,
+                              "(car (list %s))" % " ".join(["(fib 6)"] * 100),
+                              "(1 %s)" % " ".join(["(car 5)"] * 80)]))
+print(r.printed()[1], r.totals(), c5.last_stats())
+c5.close()
 print("done")
