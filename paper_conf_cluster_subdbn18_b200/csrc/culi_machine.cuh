@@ -158,13 +158,20 @@ __device__ CULI_COLD uint32_t chain_length(Ctx C, uint32_t c) {
 // word packs next | end << 32 (heap indices are < 2^31); a request that overflows the chunk takes a fresh
 // one from the global pointer and installs it with one exchange — no retry loop, so nothing spins
 // between the two collectives.  Every kernel that allocates zeroes culi_alloc first.
-constexpr uint32_t ALLOC_CHUNK = 512;
+#ifndef CULI_ALLOC_CHUNK
+#define CULI_ALLOC_CHUNK 512
+#endif
+constexpr uint32_t ALLOC_CHUNK = CULI_ALLOC_CHUNK;   // 0: every request goes to the global pointer
 __shared__ unsigned long long culi_alloc[4];
 __device__ __forceinline__ void alloc_init() {
   if ((threadIdx.x & 31) == 0 && threadIdx.x < 128) culi_alloc[threadIdx.x >> 5] = 0;
 }
+// CHUNK = false (the warp-voting kernel's own sites): every request goes to the global pointer.  Measured
+// on C4 (262,144 macro forms whose diverged lanes allocate one at a time): without the chunk code the
+// voting kernel is smaller and faster, while C2 / C5 gain from the chunks (tools/ab.sh).
+template <bool CHUNK = true>
 __device__ __forceinline__ unsigned long long alloc_range(const DevHeap& H, unsigned long long need) {
-  if (need > ALLOC_CHUNK / 4) return atomicAdd(H.top, need);
+  if (!CHUNK || need > ALLOC_CHUNK / 4) return atomicAdd(H.top, need);
   unsigned long long* s = &culi_alloc[threadIdx.x >> 5];
   unsigned long long old = atomicAdd(s, need);
   unsigned long long next = old & 0xffffffffull, end = old >> 32;
@@ -173,6 +180,7 @@ __device__ __forceinline__ unsigned long long alloc_range(const DevHeap& H, unsi
   if (b + ALLOC_CHUNK <= H.cap) atomicExch(s, ((b + ALLOC_CHUNK) << 32) | (b + need));
   return b;
 }
+template <bool CHUNK = true>
 __device__ __forceinline__ bool heap_alloc(const DevHeap& H, uint32_t n, uint32_t* out) {
   unsigned mask = __activemask();
   // (& mask: a lane group of another call converged onto this instruction must not leak into the result,
@@ -182,7 +190,7 @@ __device__ __forceinline__ bool heap_alloc(const DevHeap& H, uint32_t n, uint32_
   int leader = __ffs(peers) - 1;
   unsigned rank = __popc(peers & ((1u << lane) - 1u));
   unsigned long long base = 0;
-  if (lane == leader) base = alloc_range(H, (unsigned long long)n * (unsigned)__popc(peers));
+  if (lane == leader) base = alloc_range<CHUNK>(H, (unsigned long long)n * (unsigned)__popc(peers));
   base = __shfl_sync(peers, base, leader);
   unsigned long long mine = base + (unsigned long long)rank * n;
   if (mine + n > H.cap) return false;
@@ -563,6 +571,7 @@ __device__ CULI_COLD uint8_t equal_values(Ctx C, uint32_t vtop, V a, V b, bool* 
 }
 
 // general builtin application over vs[base+1 .. base+cnt] (any arity)
+template <bool CHUNK = true>
 __device__ CULI_COLD uint8_t apply_builtin(Ctx C, uint32_t op, uint32_t base, uint32_t cnt,
                                               uint32_t vtop, V* out) {
   const DevHeap& H = C.A->H;
@@ -614,7 +623,7 @@ __device__ CULI_COLD uint8_t apply_builtin(Ctx C, uint32_t op, uint32_t base, ui
     case BI_CONS: {
       V a = arg(C, base, 0), b = arg(C, base, 1);
       uint32_t c;
-      if (!heap_alloc(H, 3, &c)) return E_OOM;
+      if (!heap_alloc<CHUNK>(H, 3, &c)) return E_OOM;
       uint32_t ca = box_into(H, a, c + 1), cd = box_into(H, b, c + 2);
       H.tag[c] = (uint8_t)(K_CONS | (proper_value(C, b) ? TAG_PROPER : 0));
       H.word[c] = pack2(ca, cd);
@@ -624,7 +633,7 @@ __device__ CULI_COLD uint8_t apply_builtin(Ctx C, uint32_t op, uint32_t base, ui
     case BI_LIST: {
       if (cnt == 0) { *out = mkv(K_NIL, 0); return 0; }
       uint32_t c;
-      if (!heap_alloc(H, 2 * cnt, &c)) return E_OOM;
+      if (!heap_alloc<CHUNK>(H, 2 * cnt, &c)) return E_OOM;
       for (uint32_t i = 0; i < cnt; ++i) {
         uint32_t ca = box_into(H, arg(C, base, i), c + cnt + i);
         H.tag[c + i] = K_CONS | TAG_PROPER;
@@ -652,7 +661,7 @@ __device__ CULI_COLD uint8_t apply_builtin(Ctx C, uint32_t op, uint32_t base, ui
       V last = arg(C, base, cnt - 1);
       if (total == 0) { *out = last; return 0; }
       uint32_t c;
-      if (!heap_alloc(H, total + 1, &c)) return E_OOM;
+      if (!heap_alloc<CHUNK>(H, total + 1, &c)) return E_OOM;
       uint32_t tail = box_into(H, last, c + total);
       uint8_t tg = (uint8_t)(K_CONS | (proper_value(C, last) ? TAG_PROPER : 0));
       uint32_t k = 0;
@@ -676,7 +685,7 @@ __device__ CULI_COLD uint8_t apply_builtin(Ctx C, uint32_t op, uint32_t base, ui
       uint32_t n = 0;
       for (uint32_t x = (uint32_t)a.w; x != 0; x = cdr_of(C, x)) ++n;
       uint32_t c;
-      if (!heap_alloc(H, n, &c)) return E_OOM;
+      if (!heap_alloc<CHUNK>(H, n, &c)) return E_OOM;
       uint32_t k = 0;
       for (uint32_t x = (uint32_t)a.w; x != 0; ++k) {
         uint64_t w = nword(C, x);
@@ -1248,7 +1257,7 @@ HEAD:
       if (slot < C.A->maxdesc) {
         uint32_t nargs = C.A->wide[form];
         uint32_t ncells = kind == FAN_DATA ? nargs + 1 : nargs, spine;
-        if (__builtin_expect(!!(!heap_alloc(H, kind == FAN_FOLD ? nargs : 2 * ncells, &spine)), 0)) FAIL(E_OOM);
+        if (__builtin_expect(!!(!heap_alloc<!VOTE>(H, kind == FAN_FOLD ? nargs : 2 * ncells, &spine)), 0)) FAIL(E_OOM);
         if (kind == FAN_DATA) {                                   // cell 0 holds the head value
           uint32_t ca = box_into(H, v, spine + ncells);
           H.tag[spine] = K_CONS | TAG_PROPER;
@@ -1469,7 +1478,7 @@ APPLY: {                                                        // apply vs[base
   if (__builtin_expect(!!(h.t != K_BUILTIN), 0)) FAIL(E_SYNTAX);
   if ((uint32_t)h.w == BI_PAR) goto PAR_APPLY;                 // (||| n f l1 ... lm), c.7 (below RET)
   {
-    uint8_t e = apply_builtin(C, (uint32_t)h.w, base, cnt, vtop, &v);
+    uint8_t e = apply_builtin<!VOTE>(C, (uint32_t)h.w, base, cnt, vtop, &v);
     if (__builtin_expect(!!(e), 0)) FAIL(e);
   }
   vtop = base;
@@ -1673,7 +1682,7 @@ DATA_START: {
     }
     if (n == 0) { v = mkv(K_NIL, 0); goto RET; }
     uint32_t s;
-    if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &s)), 0)) FAIL(E_OOM);
+    if (__builtin_expect(!!(!heap_alloc<!VOTE>(H, 2 * n, &s)), 0)) FAIL(E_OOM);
     if (data) {
       uint32_t ca = box_into(H, v, s + n);
       H.tag[s] = K_CONS | TAG_PROPER;
@@ -1737,7 +1746,7 @@ PAR_APPLY: {
       uint32_t slot = atomicAdd(C.A->npend, 1u);
       if (slot < C.A->maxdesc) {
         uint32_t spine;
-        if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
+        if (__builtin_expect(!!(!heap_alloc<!VOTE>(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
         FanDesc* D = C.A->desc + slot;
         V f = arg(C, base, 1);
         D->form = form;
@@ -1768,7 +1777,7 @@ PAR_APPLY: {
         uint32_t slot = atomicAdd(C.A->nnest, 1u);
         if (slot < C.A->maxnest) {
           uint32_t spine;
-          if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
+          if (__builtin_expect(!!(!heap_alloc<!VOTE>(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
           NestDesc* D = C.A->ndesc + slot;
           V f = arg(C, base, 1);
           D->form = form;
@@ -1802,7 +1811,7 @@ PAR_APPLY: {
     if (__builtin_expect(!!(e), 0)) FAIL(e);
     if (n == 0) { v = mkv(K_NIL, 0); vtop = base; goto RET; }
     uint32_t m = cnt - 2, spine;
-    if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
+    if (__builtin_expect(!!(!heap_alloc<!VOTE>(H, 2 * n, &spine)), 0)) FAIL(E_OOM);
     // state: vs[base] = {spine, n}, vs[base+1] = f, vs[base+2+j] = list cursor j
     V f = arg(C, base, 1);
     for (uint32_t j = 0; j < m; ++j) *VS(C, base + 2 + j) = *VS(C, base + 3 + j);
@@ -1940,7 +1949,7 @@ QQ_LIST:                                                        // element `cur`
     if (n == 0) {
       v = mkv(K_NIL, 0);
     } else {
-      if (__builtin_expect(!!(!heap_alloc(H, 2 * n, &s)), 0)) FAIL(E_OOM);
+      if (__builtin_expect(!!(!heap_alloc<!VOTE>(H, 2 * n, &s)), 0)) FAIL(E_OOM);
       for (uint32_t i = 0; i < n; ++i) {
         uint32_t ca = box_into(H, vunpack(*VS(C, base + 1 + i)), s + n + i);
         H.tag[s + i] = K_CONS | TAG_PROPER;
