@@ -587,3 +587,36 @@ def test_quasiquote_reader(oracle_mod):
     for bad in ["`", "(a ,)", ",", "`)"]:
         with pytest.raises(oracle_mod.OracleError):
             s.read_print(bad)
+
+
+# ---- float printing (SURVEY c.8 "shortest round trip"; reading R3) against Python's repr --------
+def _sig_digits(s: str) -> int:
+    m = s.lower().lstrip("-").split("e")[0].replace(".", "").lstrip("0").rstrip("0")
+    return max(len(m), 1)
+
+
+def test_float_printing_shortest_round_trip(sess):
+    """Every printed FLOAT reads back to the same double (bit-exact, Python float()) with as few significant
+    digits as Python's repr — an independent shortest-round-trip printer (David Gay / Ryu lineage) — and always
+    carries a '.' or an exponent (so it reads back as FLOAT, c.1); nan / ±inf print as nan / inf / -inf.
+    (std::to_chars picks plain notation when it is no longer than scientific; an integral value of 2^53 or
+    more then prints as its exact integer digits, which also round-trips.)"""
+    import struct
+    rnd = random.Random(11)
+    xs = [0.0, -0.0, 1.0, -2.5, 0.1, 1e16, 1e-5, 5e-324, 2.2250738585072014e-308, 1.7976931348623157e308,
+          123456789012345678.0, 9007199254740993.0, 0.30000000000000004, 1e22, 1e21, 1e-7]
+    xs += [rnd.uniform(-1e6, 1e6) for _ in range(300)]
+    xs += [struct.unpack("<d", struct.pack("<Q", rnd.getrandbits(64)))[0] for _ in range(600)]
+    xs = [x for x in xs if math.isfinite(x)]
+    forms = ["(* %r 1.0)" % x for x in xs]             # a computed float, not the literal's text
+    res = sess.eval("\n".join(forms))
+    for x, r in zip(xs, res):
+        p = r.printed
+        assert float(p) == x and (math.copysign(1, float(p)) == math.copysign(1, x)), (x, p)
+        assert "." in p or "e" in p.lower(), p
+        if "e" not in p.lower() and abs(x) >= 2.0 ** 53:
+            assert p == "%d.0" % int(x), (x, p)
+        else:
+            assert _sig_digits(p) == _sig_digits(repr(x)), (x, p, repr(x))
+    r = sess.eval("(/ 1.0 0.0)\n(/ -1.0 0.0)\n(- (/ 1.0 0.0) (/ 1.0 0.0))")
+    assert [x.printed for x in r] == ["inf", "-inf", "nan"]
