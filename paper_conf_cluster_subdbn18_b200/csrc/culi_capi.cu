@@ -272,18 +272,8 @@ static bool image_mentions_par(const Image& img, bool skip_root_heads = false) {
 // spines are contiguous (c.14): cell k continues a list iff cell k-1 is a cons whose cdr is k.
 static bool image_has_wide_nested(const Image& img) {
   size_t N = img.tag.size();
-  std::vector<char> skip(N, 0);
-  for (uint32_t r : img.roots)
-    if (r >= IMG_FIRST) skip[r - IMG_FIRST] = 1;
   auto is_cons = [&](size_t k) { return (img.tag[k] & KIND_MASK) == K_CONS; };
-  for (size_t k = 0; k < N; ++k) {                    // (quote x): x is not evaluated
-    if (!is_cons(k)) continue;
-    uint32_t h = (uint32_t)img.word[k], c2 = (uint32_t)(img.word[k] >> 32);
-    if (h < IMG_FIRST || (img.tag[h - IMG_FIRST] & KIND_MASK) != K_SYM || img.word[h - IMG_FIRST] != SP_QUOTE) continue;
-    if (c2 < IMG_FIRST || !is_cons(c2 - IMG_FIRST)) continue;
-    uint32_t x = (uint32_t)img.word[c2 - IMG_FIRST];
-    if (x >= IMG_FIRST) skip[x - IMG_FIRST] = 1;
-  }
+  std::vector<uint32_t> cand;                         // starts (image-local) of runs of >= WIDE_MIN + 1 cells
   size_t start = 0, run = 0;
   for (size_t k = 0; k < N; ++k) {
     if (!is_cons(k)) { run = 0; continue; }
@@ -293,8 +283,24 @@ static bool image_has_wide_nested(const Image& img) {
       start = k;
       run = 1;
     }
-    if (run == WIDE_MIN + 1 && !skip[start]) return true;
+    if (run == WIDE_MIN + 1) cand.push_back(IMG_FIRST + (uint32_t)start);
   }
+  if (cand.empty()) return false;                     // (the common case: one pass, nothing allocated)
+  std::vector<char> skip(cand.size(), 0);             // candidates that are top-level forms or quoted
+  auto mark = [&](uint32_t x) {
+    auto it = std::lower_bound(cand.begin(), cand.end(), x);
+    if (it != cand.end() && *it == x) skip[it - cand.begin()] = 1;
+  };
+  for (uint32_t r : img.roots) mark(r);
+  for (size_t k = 0; k < N; ++k) {                    // (quote x): x is not evaluated
+    if (!is_cons(k)) continue;
+    uint32_t h = (uint32_t)img.word[k], c2 = (uint32_t)(img.word[k] >> 32);
+    if (h < IMG_FIRST || (img.tag[h - IMG_FIRST] & KIND_MASK) != K_SYM || img.word[h - IMG_FIRST] != SP_QUOTE) continue;
+    if (c2 < IMG_FIRST || !is_cons(c2 - IMG_FIRST)) continue;
+    mark((uint32_t)img.word[c2 - IMG_FIRST]);
+  }
+  for (char s : skip)
+    if (!s) return true;
   return false;
 }
 static bool image_mentions_setq(const Image& img) {
