@@ -122,6 +122,7 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   if (const char* e = getenv("CULI_SPLIT_FIRST")) c->split_first = std::max(1, atoi(e));
   if (const char* e = getenv("CULI_SPLIT_SLEEP")) c->split_sleep = std::max(32, atoi(e));
   if (const char* e = getenv("CULI_STEAL_GATE")) c->steal_gate = atoi(e) != 0;
+  if (const char* e = getenv("CULI_SIZE_FIRST")) c->size_first = atoi(e) != 0;
   if (const char* e = getenv("CULI_WAIT_MS")) c->wait_ns = (unsigned long long)std::max(1, atoi(e)) * 1000000ull;
   bool ok = true;
   if (o.heap_base) {                                 // caller-owned arena (e.g. a torch tensor)
@@ -509,8 +510,10 @@ static int run_batch_device(culi_ctx* c) {
   ++c->last_kernels;
   uint32_t* perm = nullptr;
   if (!(c->opts.flags & CULI_F_NO_BINNING) && nf > 1 && (nf >= BIN_MIN_FORMS || c->batch_may_close)) {
+    // closure-free batches (the voting kernel): biggest forms first (CULI_SIZE_FIRST=0 turns it off)
+    uint32_t size_first = !c->batch_may_close && c->size_first;
     CK(launch_dispatch(c->stream, c->H, c->roots.p, nf, c->keys.p, c->keys_alt.p, c->perm.p,
-                       c->perm_alt.p, c->dtemp.p, c->dtemp.n, &perm, c->sms));
+                       c->perm_alt.p, c->dtemp.p, c->dtemp.n, &perm, c->sms, size_first));
     c->last_kernels += dispatch_launches(nf);
   }
   CK(record_event(c, 1));

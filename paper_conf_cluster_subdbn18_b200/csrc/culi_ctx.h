@@ -162,6 +162,7 @@ struct culi_ctx {
   uint32_t split_first = 64;         // closure calls before the first poll (env CULI_SPLIT_FIRST)
   uint32_t steal_gate = 1;           // steal only from fully idle warps (env CULI_STEAL_GATE)
   uint32_t split_sleep = 4096;       // idle-warp back-off cap in ns (env CULI_SPLIT_SLEEP)
+  uint32_t size_first = 1;           // dispatch: closure-free batches biggest forms first (env CULI_SIZE_FIRST)
   DevBuf<uint32_t> wide;
   // uploaded batch (culi_upload)
   bool have_batch = false;

@@ -23,11 +23,15 @@ namespace culi {
 // Shape of a form: FNV-1a over a pre-order walk of its first 48 nodes — node kinds, symbol ids, list
 // structure; numbers contribute only their kind (their values are in the hint).  Forms with equal shape
 // expand macros and take calls in the same order, so a warp of them stays converged longer (C4).
-__device__ uint32_t shape_hash(TagArr tag, WordArr word, uint32_t x) {
+// *size: nodes visited (at most 48) — a cost proxy for batches without closures, where a form's work is
+// bounded by its size (no recursion): their warps run the biggest forms first (longest processing time
+// first), so the last, partly filled round of warp batches holds small ones.
+__device__ uint32_t shape_hash(TagArr tag, WordArr word, uint32_t x, uint32_t* size) {
   uint32_t st[12];
   int sp = 0;
   uint32_t h = 2166136261u;
-  for (int visited = 0; visited < 48; ++visited) {
+  int visited = 0;
+  for (; visited < 48; ++visited) {
     uint32_t t = tag[x] & KIND_MASK;
     h = (h ^ t) * 16777619u;
     if (t == K_SYM) h = (h ^ (uint32_t)word[x]) * 16777619u;
@@ -45,6 +49,7 @@ __device__ uint32_t shape_hash(TagArr tag, WordArr word, uint32_t x) {
     x = st[--sp];
     h = (h ^ 0x55u) * 16777619u;                      // a subtree ended: keeps (a (b) c) != (a (b c))
   }
+  *size = (uint32_t)visited + 1;
   return h;
 }
 
@@ -82,11 +87,12 @@ __device__ uint64_t structure_prefix(TagArr tag, WordArr word, uint32_t x) {
 
 __global__ void culi_classify_kernel(TagArr tag, WordArr word,
                                      const uint32_t* __restrict__ roots, uint32_t nforms,
-                                     unsigned long long* __restrict__ keys, uint32_t* __restrict__ perm) {
+                                     unsigned long long* __restrict__ keys, uint32_t* __restrict__ perm,
+                                     uint32_t size_first) {
   uint32_t stride = gridDim.x * blockDim.x;
   for (uint32_t f = blockIdx.x * blockDim.x + threadIdx.x; f < nforms; f += stride) {
     uint32_t r = roots[f];
-    uint32_t hint = 0, shape = 0;
+    uint32_t hint = 0, shape = 0, size = 1;
     uint64_t prefix = structure_prefix(tag, word, r);
     if ((tag[r] & KIND_MASK) == K_CONS) {
       uint64_t w = word[r];
@@ -102,11 +108,17 @@ __global__ void culi_classify_kernel(TagArr tag, WordArr word,
           if ((tag[ah] & KIND_MASK) == K_SYM) hint = 0xff00u | ((uint32_t)word[ah] & 0xff);
         }
       }
-      shape = shape_hash(tag, word, r);
+      shape = shape_hash(tag, word, r, &size);
     }
-    // 56 bits (7 radix passes): structure prefix 30 | shape hash 10 | inverted hint 16
-    keys[f] = (prefix << 26) | ((unsigned long long)((shape ^ (shape >> 10) ^ (shape >> 20)) & 0x3ffu) << 16) |
-              (0xffffu - hint);
+    // 56 bits (7 radix passes): structure prefix 30 | shape hash 10 | inverted hint 16; closure-free batches:
+    // inverted size class 4 (nodes / 4, up to 48 nodes) | structure prefix 30 | shape hash 10 | inverted hint 12
+    uint64_t sh = (uint64_t)((shape ^ (shape >> 10) ^ (shape >> 20)) & 0x3ffu);
+    if (size_first) {
+      uint32_t cls = min(size / 4u, 15u);
+      keys[f] = ((uint64_t)(15u - cls) << 52) | (prefix << 22) | (sh << 12) | (0xfffu - min(hint, 0xfffu));
+    } else {
+      keys[f] = (prefix << 26) | (sh << 16) | (0xffffu - hint);
+    }
     perm[f] = f;
   }
 }
@@ -124,14 +136,14 @@ size_t dispatch_temp_bytes(uint32_t nforms) {
 
 cudaError_t launch_dispatch(cudaStream_t s, const DevHeap& H, const uint32_t* roots, uint32_t nforms,
                             uint32_t* keys, uint32_t* keys_alt, uint32_t* perm, uint32_t* perm_alt,
-                            void* temp, size_t temp_bytes, uint32_t** perm_out, int sms) {
+                            void* temp, size_t temp_bytes, uint32_t** perm_out, int sms, uint32_t size_first) {
   // keys / keys_alt hold 2 x nforms words each (64-bit keys)
   unsigned long long* k0 = reinterpret_cast<unsigned long long*>(keys);
   unsigned long long* k1 = reinterpret_cast<unsigned long long*>(keys_alt);
   uint32_t blocks = (nforms + 255) / 256;
   if (blocks > (uint32_t)sms * 8) blocks = sms * 8;
   if (blocks == 0) blocks = 1;
-  culi_classify_kernel<<<blocks, 256, 0, s>>>(H.tag, H.word, roots, nforms, k0, perm);
+  culi_classify_kernel<<<blocks, 256, 0, s>>>(H.tag, H.word, roots, nforms, k0, perm, size_first);
   cudaError_t e = cudaGetLastError();
   if (e != cudaSuccess) return e;
   size_t tb = temp_bytes;

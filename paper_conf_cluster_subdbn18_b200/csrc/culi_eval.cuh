@@ -229,7 +229,7 @@ cudaError_t launch_nest_clear(cudaStream_t s, struct NestDesc* d, uint32_t n);
 cudaError_t launch_flat_export(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
 cudaError_t launch_dispatch(cudaStream_t s, const DevHeap& H, const uint32_t* roots, uint32_t nforms,
                             uint32_t* keys, uint32_t* keys_alt, uint32_t* perm, uint32_t* perm_alt,
-                            void* temp, size_t temp_bytes, uint32_t** perm_out, int sms);
+                            void* temp, size_t temp_bytes, uint32_t** perm_out, int sms, uint32_t size_first);
 size_t dispatch_temp_bytes(uint32_t nforms);
 uint32_t dispatch_launches(uint32_t nforms);   // kernels launch_dispatch issues (an estimate: the graph path counts them)
 // Batches of at most this many forms in which no closure can exist (no lambda / defun) are evaluated in
