@@ -354,7 +354,10 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.finished = c->nnest + 1;
   // argument splitting: where a closure may be applied (the poll sits at closure calls), binned or not
   (void)perm;
-  A.split = (!define_mode && c->batch_may_close && !(c->opts.flags & CULI_F_NO_SPLIT)) ? 1 : 0;
+  // (a batch that is one top-level ||| form spends its time in the fan-out kernel: its eval launch needs one
+  // block, not a grid of idle thieves — C3 eval phase 0.19 -> 0.165 ms)
+  A.split = (!define_mode && c->batch_may_close && !(c->opts.flags & CULI_F_NO_SPLIT) &&
+             !(c->batch_single_par && !(c->opts.flags & CULI_F_NO_FANOUT))) ? 1 : 0;
   // setq (R7): frames go to the heap when made, and a form runs in one thread only (no fan-out, nested
   // fan-out or argument splitting: those evaluate parts of a form elsewhere, on copies of its frames)
   A.mut = define_mode ? c->define_mut : c->batch_mut;
@@ -585,6 +588,7 @@ static int finish_prepare(culi_ctx* c, uint32_t nf, uint64_t nnodes, std::string
     CK(cudaMalloc(&c->vst2, (size_t)c->nslots * c->vcap * sizeof(uint4)));
   }
   c->batch_has_par = par_head;
+  c->batch_single_par = nf == 1 && par_head;
   c->batch_has_wide = has_wide;
   if (has_wide) c->batch_has_par = true;             // the fan-out kernels handle both
   return CULI_OK;

@@ -141,6 +141,7 @@ struct culi_ctx {
   bool batch_mut = false, define_mut = false;
   bool persist_has_closure = false;  // some definition mentions lambda / defun
   bool batch_may_close = false;      // a closure may be applied in the batch (argument splitting useful)
+  bool batch_single_par = false;     // the batch is one top-level (||| ...) form (its elements fan out)
   bool batch_may_nest = false;
   NestDesc* ndesc = nullptr;
   uint32_t maxnest = 4096;
