@@ -522,6 +522,9 @@ static int run_batch_device(culi_ctx* c) {
   CK(record_event(c, 1));
   EvalArgs A = make_args(c, nf, perm, 0);
   A.fanout = A.fanout && c->batch_has_par;
+  // small unbinned batches (<= 128 warps, fewer than the SMs) are latency-bound: the voting kernel's
+  // regrouping costs more than the divergence it saves there (C1: 0.056 -> 0.049 ms eval)
+  if (nf < BIN_MIN_FORMS) A.voting = 0;
   if (A.nest) { CK(launch_nest_clear(c->stream, c->ndesc, c->maxnest)); ++c->last_kernels; }
   uint32_t blocks = c->nslots / 128;
   uint32_t need = (nf + 127) / 128;
