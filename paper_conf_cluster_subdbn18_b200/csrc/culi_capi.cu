@@ -123,6 +123,7 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   if (const char* e = getenv("CULI_SPLIT_SLEEP")) c->split_sleep = std::max(32, atoi(e));
   if (const char* e = getenv("CULI_STEAL_GATE")) c->steal_gate = atoi(e) != 0;
   if (const char* e = getenv("CULI_SIZE_FIRST")) c->size_first = atoi(e) != 0;
+  if (const char* e = getenv("CULI_THIN_LANES")) c->thin_lanes = std::min(32, std::max(0, atoi(e)));
   if (const char* e = getenv("CULI_WAIT_MS")) c->wait_ns = (unsigned long long)std::max(1, atoi(e)) * 1000000ull;
   bool ok = true;
   if (o.heap_base) {                                 // caller-owned arena (e.g. a torch tensor)
@@ -338,6 +339,7 @@ static EvalArgs make_args(culi_ctx* c, uint32_t nforms, const uint32_t* perm, in
   A.define_mode = define_mode;
   A.flags = c->flags;
   A.voting = (c->opts.flags & CULI_F_NO_VOTING) ? 0 : 1;
+  A.lanes = 32;
   A.fanout = (!define_mode && !(c->opts.flags & CULI_F_NO_FANOUT)) ? 1 : 0;
   A.desc = c->desc;
   A.npend = c->npend;
@@ -531,6 +533,16 @@ static int run_batch_device(culi_ctx* c) {
   // a batch that may suspend on nested ||| or split arguments keeps the whole grid: idle warps apply the
   // elements / evaluate split-off arguments
   if (need < blocks && !A.nest && !A.split) blocks = std::max<uint32_t>(need, 1);
+  // a small batch on the plain kernel is latency-bound and its lanes diverge (different forms): thin warps
+  // — `lanes` forms per warp, about one warp per scheduler of the GPU — serialise fewer paths per warp
+  A.lanes = 32;
+  if (!A.nest && !A.split && nf < BIN_MIN_FORMS) {
+    uint32_t want = (nf + 4 * c->sms - 1) / (4 * c->sms), lanes = 1;
+    while (lanes < want && lanes < 32) lanes *= 2;
+    if (c->thin_lanes) lanes = c->thin_lanes;
+    A.lanes = lanes;
+    blocks = std::min<uint32_t>(c->nslots / 128, std::max<uint32_t>((nf + 4 * lanes - 1) / (4 * lanes), 1));
+  }
   if (nf) { CK(launch_eval(c->stream, A, blocks)); ++c->last_kernels; }
   if (nf && A.fanout && c->batch_has_par) {            // ||| fan-out (a6) + finalize (a8)
     CK(launch_fanout(c->stream, A, c->nslots / 128));

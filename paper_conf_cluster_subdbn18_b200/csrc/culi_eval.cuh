@@ -76,6 +76,7 @@ struct EvalArgs {
   unsigned long long* pcount;
   unsigned long long pcap;
   const uint32_t* wide;        // per form: argument count of a wide top-level form, else 0 (host scan)
+  uint32_t lanes;              // plain kernel: forms per warp (lanes >= this stay idle; 32 = all)
   uint32_t nest;               // nested ||| suspend + help, batch eval kernel only
   struct NestDesc* ndesc;
   uint32_t* nnest;

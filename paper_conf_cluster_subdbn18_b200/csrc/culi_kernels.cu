@@ -245,6 +245,7 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
     C2.vb = A.vst2 + slot;
   }
   bool forms_left = true;
+  if (!SPLIT && !NEST && (threadIdx.x & 31) >= A.lanes) return;   // thin warps for small batches
   uint32_t round = 0;                                   // idle rounds taken (split_claim)
   SplitGroup* G = nullptr;                              // the claimed group whose tasks this lane runs
   uint32_t todo = 0;                                    // its task positions left for this lane
