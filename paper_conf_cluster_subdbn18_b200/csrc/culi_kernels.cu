@@ -54,23 +54,10 @@ __device__ __forceinline__ Ctx make_ctx(const EvalArgs& A, uint32_t slot) {
 // Runs on the thread's secondary stacks (C2).  Element i: f applied to (l1[i] .. lm[i]) at the depth of the
 // ||| call, with the fuel left when the owner suspended.  A failed contiguity check or an element error
 // marks the descriptor bad (the owner's form is then re-evaluated sequentially, exactly).
+
 #if CULI_NEST_TRACE
-// debug: [0] first claim, [1] last element done, [2] owner resumed, [3] owner suspended (min/max globaltimer)
-__device__ unsigned long long culi_nest_trace[8];
-extern "C" int culi_debug_nest_trace(unsigned long long* out) {
-  return cudaMemcpyFromSymbol(out, culi_nest_trace, sizeof(culi_nest_trace)) == cudaSuccess ? 0 : 1;
-}
-extern "C" int culi_debug_nest_trace_reset() {
-  unsigned long long z[8] = {~0ull, 0, 0, ~0ull, 0, 0, 0, 0};
-  return cudaMemcpyToSymbol(culi_nest_trace, z, sizeof(z)) == cudaSuccess ? 0 : 1;
-}
-#define NTRACE_MIN(k) atomicMin(&culi_nest_trace[k], gtime())
-#define NTRACE_MAX(k) atomicMax(&culi_nest_trace[k], gtime())
-#define NTRACE_ADD(k, v) atomicAdd(&culi_nest_trace[k], (unsigned long long)(v))
-#else
-#define NTRACE_MIN(k) do { } while (0)
-#define NTRACE_MAX(k) do { } while (0)
-#define NTRACE_ADD(k, v) do { } while (0)
+extern "C" int culi_debug_nest_trace(unsigned long long* out) { return culi_nest_trace_read(out); }
+extern "C" int culi_debug_nest_trace_reset() { return culi_nest_trace_reset(); }
 #endif
 __device__ __forceinline__ bool nest_run_one(const EvalArgs& A, const Ctx& C2, NestDesc* D) {
   if (*(volatile uint32_t*)&D->ready == 0) return false;
@@ -246,6 +233,7 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
   }
   bool forms_left = true;
   if (!SPLIT && !NEST && (threadIdx.x & 31) >= A.lanes) return;   // thin warps for small batches
+  if (NEST && threadIdx.x == 0) NTRACE_MIN(5);
   uint32_t round = 0;                                   // idle rounds taken (split_claim)
   SplitGroup* G = nullptr;                              // the claimed group whose tasks this lane runs
   uint32_t todo = 0;                                    // its task positions left for this lane
@@ -325,10 +313,11 @@ __global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(cons
   }
   if (NEST) {                                           // no forms left: help until every form is done
     uint32_t ns = 128;                                  // (back off while there is nothing to claim: the
-    while (*(volatile uint32_t*)A.finished < A.nforms) {  //  whole grid polls the same descriptors)
-      if (nest_help_any(A, C2, nullptr)) { ns = 128; continue; }
+    while (*(volatile uint32_t*)A.finished < A.nforms) {  //  whole grid polls the same descriptors; longer
+      if (nest_help_any(A, C2, nullptr)) { ns = 128; continue; }   // before the first one is published)
       __nanosleep(ns);
-      ns = ns * 2 > 2048 ? 2048 : ns * 2;
+      uint32_t cap = *(volatile uint32_t*)A.nnest ? 2048u : 8192u;
+      ns = ns * 2 > cap ? cap : ns * 2;
     }
   }
 }

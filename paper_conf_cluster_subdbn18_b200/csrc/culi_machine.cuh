@@ -125,6 +125,34 @@ __device__ __forceinline__ V unbox(const Ctx& C, uint32_t n) {
 __device__ __forceinline__ uint32_t car_of(const Ctx& C, uint32_t c) { return lo32(nword(C, c)); }
 __device__ __forceinline__ uint32_t cdr_of(const Ctx& C, uint32_t c) { return hi32(nword(C, c)); }
 
+#ifndef CULI_NEST_TRACE
+#define CULI_NEST_TRACE 0
+#endif
+__device__ __forceinline__ unsigned long long gtime_trace() {
+  unsigned long long t;
+  asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+  return t;
+}
+#if CULI_NEST_TRACE
+// debug (-DCULI_NEST_TRACE=1): [0] first claim, [1] last element done, [2] owner resumed, [3] owner suspended,
+// [4] claims, [5] first thread started, [6] owner at DATA_START, [7] owner after the cell count (globaltimer)
+__device__ unsigned long long culi_nest_trace[8];
+__host__ inline int culi_nest_trace_read(unsigned long long* out) {
+  return cudaMemcpyFromSymbol(out, culi_nest_trace, sizeof(culi_nest_trace)) == cudaSuccess ? 0 : 1;
+}
+__host__ inline int culi_nest_trace_reset() {
+  unsigned long long z[8] = {~0ull, 0, 0, ~0ull, 0, ~0ull, 0, 0};
+  return cudaMemcpyToSymbol(culi_nest_trace, z, sizeof(z)) == cudaSuccess ? 0 : 1;
+}
+#define NTRACE_MIN(k) atomicMin(&culi_nest_trace[k], gtime_trace())
+#define NTRACE_MAX(k) atomicMax(&culi_nest_trace[k], gtime_trace())
+#define NTRACE_ADD(k, v) atomicAdd(&culi_nest_trace[k], (unsigned long long)(v))
+#else
+#define NTRACE_MIN(k) do { } while (0)
+#define NTRACE_MAX(k) do { } while (0)
+#define NTRACE_ADD(k, v) do { } while (0)
+#endif
+
 // Length of the cdr chain from c (the count loop of a data list / list).  Reader spines are contiguous
 // (c.14), so the next 16 cells are loaded before their links are checked (branch-free, so all loads are in
 // flight together: one L2 round trip per 16 cells instead of one per cell); a link that leaves the run
@@ -135,16 +163,16 @@ __device__ CULI_COLD uint32_t chain_length(Ctx C, uint32_t c) {
   const uint64_t cap = C.A->H.cap;
   const Node* nodes = C.A->H.tag.p;
   while (c != 0) {
-    if ((uint64_t)c + 16 > cap) { ++n; c = cdr_of(C, c); continue; }
-    // 16 cells per round trip: the cdr halves of 16 nodes, links checked afterwards (all loads in flight)
-    uint32_t q[16];
+    if ((uint64_t)c + 32 > cap) { ++n; c = cdr_of(C, c); continue; }
+    // 32 cells per round trip: the cdr halves of 32 nodes, links checked afterwards (all loads in flight)
+    uint32_t q[32];
 #pragma unroll
-    for (int k = 0; k < 16; ++k) q[k] = reinterpret_cast<const uint32_t*>(nodes + c + k)[1];
-    uint32_t brk = 0, nx = c + 16;
+    for (int k = 0; k < 32; ++k) q[k] = reinterpret_cast<const uint32_t*>(nodes + c + k)[1];
+    uint32_t brk = 0, nx = c + 32;
 #pragma unroll
-    for (int k = 15; k >= 0; --k)
+    for (int k = 31; k >= 0; --k)
       if (q[k] != c + k + 1) { brk |= 1u << k; nx = q[k]; }       // the lowest break wins
-    n += brk ? __ffs(brk) : 16;
+    n += brk ? __ffs(brk) : 32;
     c = nx;
   }
   return n;
@@ -1674,9 +1702,11 @@ DATA_START: {
     bool data = v.t != K_BUILTIN;
     uint32_t n = data ? 1 : 0;
     if (NEST) {                                                 // (batches with wide lists run NEST)
+      NTRACE_MAX(6);
       uint32_t c = cur;
       for (uint32_t k = 0; k < 16 && c != 0; ++k, ++n) c = cdr_of(C, c); // short lists inline;
       if (c != 0) n += chain_length(C, c);                              // long ones 16 cells per load round
+      NTRACE_MAX(7);
     } else {
       for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
     }

@@ -5,7 +5,7 @@ sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 import torch
 from paper_conf_cluster_subdbn18_b200 import build, culi
 from paper_conf_cluster_subdbn18_b200 import workloads as W
-lib = build.build(defines=["CULI_NEST_TRACE=1"], out=os.path.join(os.path.dirname(__file__), "..", "gpurun_out", "libculi_trace.so"))
+lib = build.build(defines=["CULI_NEST_TRACE=1"] + (["CULI_SLEEP_GATE=1"] if os.environ.get("GATE") else []), out=os.path.join(os.path.dirname(__file__), "..", "gpurun_out", "libculi_trace.so"))
 L = culi.load(lib)
 ctx = culi.Context(device=0, stream=torch.cuda.current_stream().cuda_stream)
 ctx.define(W.FIB_DEF)
@@ -20,6 +20,8 @@ for n in (256, 4096, 16384):
             L.culi_debug_nest_trace(T)
             ms, _, _ = ctx.last_timing()
             t = list(T)
-            print(n, form[:10], "eval %.3f ms" % ms[1], "suspend->claim %.1f us" % ((t[0] - t[3]) / 1e3),
+            print(n, form[:10], "eval %.3f ms" % ms[1], "start->DATA_START %.1f us" % ((t[6] - t[5]) / 1e3),
+                  "count %.1f us" % ((t[7] - t[6]) / 1e3), "count->suspend %.1f us" % ((t[3] - t[7]) / 1e3),
+                  "suspend->claim %.1f us" % ((t[0] - t[3]) / 1e3),
                   "claim->lastdone %.1f us" % ((t[1] - t[0]) / 1e3), "lastdone->resume %.1f us" % ((t[2] - t[1]) / 1e3),
                   "claims", t[4])
