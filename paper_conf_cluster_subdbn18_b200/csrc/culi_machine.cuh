@@ -1474,10 +1474,13 @@ APPLY: {                                                        // apply vs[base
   if (h.t == K_CLOSURE) {                                       // PAPER L456-460, c.4 CLOSURE
     if (SPLIT && __builtin_expect(--pollc == 0, 0)) {
       pollc = C.A->split_poll;
-      if (kdirty) *KS(C, sp - 1) = ktop;
-      kdirty = false;
-      try_split(C, sp, steps, fuel, form);
-      if (sp > 0) ktop = *KS(C, sp - 1);                        // the top frame may have become KF_JOIN
+      // (the common answer — no idle warp waits for a ticket — without the call and its register traffic)
+      if (ld_relaxed64(&C.A->sctl->head) > ld_relaxed64(&C.A->sctl->tail)) {
+        if (kdirty) *KS(C, sp - 1) = ktop;
+        kdirty = false;
+        try_split(C, sp, steps, fuel, form);
+        if (sp > 0) ktop = *KS(C, sp - 1);                      // the top frame may have become KF_JOIN
+      }
     }
     uint64_t cwd = nword(C, (uint32_t)h.w);                     // three independent loads
     uint64_t aux = nword(C, (uint32_t)h.w + 1);
