@@ -66,7 +66,7 @@ __device__ __forceinline__ bool nest_run_one(const EvalArgs& A, const Ctx& C2, N
   uint32_t i = fetch_add_grouped(&D->next);           // (one atomic per warp and descriptor)
   if (i >= n) return false;
   NTRACE_MIN(0);
-  NTRACE_ADD(4, 1);
+  if (CULI_NEST_TRACE == 1) NTRACE_ADD(4, 1);
   const DevHeap& H = A.H;
   uint32_t m = D->m, spine = D->spine;
   bool ok = true;

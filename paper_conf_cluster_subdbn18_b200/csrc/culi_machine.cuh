@@ -1708,8 +1708,12 @@ DATA_START: {
       NTRACE_MAX(6);
       uint32_t c = cur;
       for (uint32_t k = 0; k < 16 && c != 0; ++k, ++n) c = cdr_of(C, c); // short lists inline;
-      if (c != 0) n += chain_length(C, c);                              // long ones 16 cells per load round
+      if (c != 0) n += chain_length(C, c);                              // long ones 32 cells per load round
       NTRACE_MAX(7);
+#if CULI_NEST_TRACE > 1
+      if (c != 0) { volatile uint32_t n2 = chain_length(C, c); (void)n2; }   // debug: the same walk, warm
+      NTRACE_MAX(4);
+#endif
     } else {
       for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
     }
