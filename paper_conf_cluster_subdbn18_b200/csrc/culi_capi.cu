@@ -166,7 +166,7 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   c->H.cap = o.heap_nodes;
   c->H.gcap = GCAP;
   // nil and T nodes; every symbol unbound; builtins are resolved by id (reserved names)
-  static const Node n01[2] = {Node{0, K_NIL, {}}, Node{0, K_T, {}}};
+  static const Node n01[2] = {Node{0, K_NIL, {}, 0}, Node{0, K_T, {}, 0}};
   bool ok2 = cudaMemcpyAsync(c->H.tag.p, n01, sizeof(n01), cudaMemcpyHostToDevice, c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->H.gtag, K_UNBOUND, GCAP, c->stream) == cudaSuccess &&
              cudaMemsetAsync(c->flags, 0, 8 * sizeof(int), c->stream) == cudaSuccess &&
@@ -410,6 +410,12 @@ static int upload_image(culi_ctx* c, const Image& img, uint32_t str_base) {
   if (nr) CK(cudaMemcpyAsync(c->roots.p, img.roots.data(), nr * 4, cudaMemcpyHostToDevice, c->stream));
   CK(launch_relocate(c->stream, (const uint8_t*)(c->stage.p + n), c->stage.p, c->H.tag.p, c->mark, n, str_base,
                      c->roots.p, nr, c->sms));
+  if (!img.wide_len.empty()) {                       // wide lists: their element count in O(1) (TAG_LEN)
+    uint32_t np = (uint32_t)(img.wide_len.size() / 2);
+    CK(c->lenpairs.ensure(2 * np));
+    CK(cudaMemcpyAsync(c->lenpairs.p, img.wide_len.data(), 8ull * np, cudaMemcpyHostToDevice, c->stream));
+    CK(launch_lenmark(c->stream, c->H.tag.p, c->mark, c->lenpairs.p, np));
+  }
   return CULI_OK;
 }
 

@@ -166,6 +166,7 @@ struct culi_ctx {
   uint32_t size_first = 1;           // dispatch: closure-free batches biggest forms first (env CULI_SIZE_FIRST)
   uint32_t thin_lanes = 0;           // small plain-kernel batches: forms per warp (0 = auto; env CULI_THIN_LANES)
   DevBuf<uint32_t> wide;
+  DevBuf<uint32_t> lenpairs;         // wide-list length marks of a host image (culi_lenmark_kernel)
   // uploaded batch (culi_upload)
   bool have_batch = false;
   uint64_t batch_nodes = 0;

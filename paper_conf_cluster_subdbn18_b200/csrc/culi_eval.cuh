@@ -106,6 +106,7 @@ constexpr uint8_t E_PENDING = 0xfe;          // internal: record filled in by th
 // a1..an, op in m).  For wide kinds element i evaluates argument i (depth 2); heads[0] = first arg cell.
 enum FanKind : uint32_t { FAN_PAR = 0, FAN_DATA = 1, FAN_LIST = 2, FAN_FOLD = 3 };
 constexpr uint32_t WIDE_MIN = 64;
+static_assert(WIDE_MIN == WIDE_LEN_MIN, "readers mark lists of the size the machine suspends on");
 struct FanDesc {
   uint32_t form, n, m, spine;                // n: result cells; spine: 2n nodes (n cells, then n boxes)
   uint32_t kind, nelem;                      // FanKind; elements to evaluate
@@ -220,6 +221,7 @@ struct ExportArgs {
 cudaError_t launch_relocate(cudaStream_t s, const uint8_t* stag, const uint64_t* sword, Node* nodes, uint64_t base,
                             uint64_t n, uint32_t str_base, uint32_t* roots, uint32_t nroots, int sms);
 cudaError_t launch_eval(cudaStream_t s, const EvalArgs& A, uint32_t blocks);
+cudaError_t launch_lenmark(cudaStream_t s, Node* nodes, uint64_t base, const uint32_t* pairs, uint32_t npairs);
 cudaError_t launch_define(cudaStream_t s, const EvalArgs& A);
 cudaError_t launch_export(cudaStream_t s, const ExportArgs& X, uint32_t blocks);
 cudaError_t launch_reset(cudaStream_t s, unsigned long long* top, unsigned long long top_value,

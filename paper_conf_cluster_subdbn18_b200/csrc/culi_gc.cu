@@ -122,8 +122,9 @@ __global__ void copy_kernel(TagArr tag, WordArr word, const uint32_t* role, cons
   for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < mark; i += (uint64_t)gridDim.x * blockDim.x) {
     uint32_t r = role[i];
     if (i < IMG_FIRST || r == R_DEAD) continue;
-    uint8_t t = tag[i];
-    uint64_t w = word[i];
+    const uint4 q = *reinterpret_cast<const uint4*>(tag.p + i);     // the whole node (incl. a TAG_LEN length)
+    uint8_t t = (uint8_t)q.z;
+    uint64_t w = ((uint64_t)q.y << 32) | q.x;
     if (r == R_AUX2) {
       w = pack2(fwd(pos, lo(w)), fwd(pos, hi(w)));
     } else if (r == R_NODE) {
@@ -136,9 +137,9 @@ __global__ void copy_kernel(TagArr tag, WordArr word, const uint32_t* role, cons
         default: break;                                 // leaves: payload verbatim
       }
     }
-    uint32_t d = pos[i];
-    stag[d] = t;
-    sword[d] = w;
+    uint32_t d = pos[i];                              // (compaction keeps spines contiguous: lengths stay valid)
+    *reinterpret_cast<uint4*>(stag.p + d) = make_uint4((uint32_t)w, (uint32_t)(w >> 32), q.z, q.w);
+    (void)sword;
   }
 }
 

@@ -176,6 +176,10 @@ struct Builder {
     uint8_t valid = special_form_valid(xs) ? TAG_VALID : 0;
     for (uint32_t k = 0; k < n; ++k)
       node((uint8_t)(K_CONS | TAG_PROPER | (k == 0 ? valid : 0)), pack2(xs[k], k + 1 < n ? first + k + 1 : 0));
+    if (n >= WIDE_LEN_MIN + 1) {                       // the device marks the second cell (TAG_LEN)
+      img.wide_len.push_back(first + 1);
+      img.wide_len.push_back(n - 1);
+    }
     return first;
   }
 

@@ -33,6 +33,7 @@ struct Image {
   std::vector<uint32_t> roots;     // local index of each top-level form
   std::string strings;
   uint32_t max_sym = 0;            // largest symbol id referenced + 1
+  std::vector<uint32_t> wide_len;  // pairs (local index of a wide list's second cell, cells from it to the end)
 };
 
 // Returns 0 or CULI_E_PARSE with *err_offset.

@@ -24,6 +24,12 @@ constexpr uint8_t TAG_PROPER = 0x10;
 // names are reserved, c.5) and whose syntax it has already validated per c.5; the device skips the
 // checks for such lists.  Lists built at run time (macro expansions) never carry it.
 constexpr uint8_t TAG_VALID = 0x20;
+// Set by the readers on the second cell of a list with at least WIDE_MIN + 1 cells, whose `len` field
+// (struct Node) then holds the number of cells from it to the end of the list: a wide data list / (list ...)
+// starts its element count there (culi_machine.cuh DATA_START) in O(1) instead of walking the spine.  Any
+// write of a tag byte clears it, so a cell built at run time never carries a stale length.
+constexpr uint8_t TAG_LEN = 0x40;
+constexpr uint32_t WIDE_LEN_MIN = 64;   // == WIDE_MIN (culi_eval.cuh)
 constexpr uint8_t K_AUX = 14;    // second node of a closure/macro: nparams | first param symbol << 32
 constexpr uint8_t KIND_MASK = 0x0f;
 
@@ -61,7 +67,8 @@ CULI_HD uint64_t pack2(uint32_t lo, uint32_t hi) { return (uint64_t)lo | ((uint6
 struct alignas(16) Node {
   uint64_t word;
   uint8_t tag;
-  uint8_t pad[7];
+  uint8_t pad[3];
+  uint32_t len;                // TAG_LEN cells: cells from here to the end of the list
 };
 static_assert(sizeof(Node) == 16, "one 16-byte access per node");
 struct TagArr {

@@ -34,6 +34,20 @@ __global__ void culi_relocate_kernel(const uint8_t* __restrict__ stag, const uin
   }
 }
 
+// Mark the second cell of every wide list of an uploaded image with its remaining length (TAG_LEN): pairs of
+// (image-local cell, cells from it to the end), relocated to base.  One writer per cell.
+__global__ void culi_lenmark_kernel(Node* nodes, uint64_t base, const uint32_t* pairs, uint32_t npairs) {
+  for (uint32_t k = blockIdx.x * blockDim.x + threadIdx.x; k < npairs; k += gridDim.x * blockDim.x) {
+    Node* x = nodes + base + (pairs[2 * k] - IMG_FIRST);
+    x->len = pairs[2 * k + 1];
+    x->tag = (uint8_t)(x->tag | TAG_LEN);
+  }
+}
+cudaError_t launch_lenmark(cudaStream_t s, Node* nodes, uint64_t base, const uint32_t* pairs, uint32_t npairs) {
+  culi_lenmark_kernel<<<(npairs + 255) / 256, 256, 0, s>>>(nodes, base, pairs, npairs);
+  return cudaGetLastError();
+}
+
 __device__ __forceinline__ void write_result(const EvalArgs& A, uint32_t f, const FormOut& o) {
   A.rtag[f] = o.err ? (uint8_t)K_ERROR : (uint8_t)o.t;
   A.rerr[f] = o.err;

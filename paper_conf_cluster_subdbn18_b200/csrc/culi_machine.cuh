@@ -95,7 +95,7 @@ __device__ __forceinline__ void ldnode(const Ctx& C, uint32_t n, uint32_t& t, ui
   }
 #endif
   const uint4 q = *reinterpret_cast<const uint4*>(C.A->H.tag.p + n);   // one 16-byte load per node
-  t = q.z & 0xffu;
+  t = q.z & (0xffu & ~(uint32_t)TAG_LEN);
   w = ((uint64_t)q.y << 32) | q.x;
 }
 __device__ __forceinline__ uint64_t nword(const Ctx& C, uint32_t n) {
@@ -1706,14 +1706,15 @@ DATA_START: {
     uint32_t n = data ? 1 : 0;
     if (NEST) {                                                 // (batches with wide lists run NEST)
       NTRACE_MAX(6);
-      uint32_t c = cur;
-      for (uint32_t k = 0; k < 16 && c != 0; ++k, ++n) c = cdr_of(C, c); // short lists inline;
-      if (c != 0) n += chain_length(C, c);                              // long ones 32 cells per load round
+      const uint4 q0 = cur ? *reinterpret_cast<const uint4*>(H.tag.p + cur) : make_uint4(0, 0, 0, 0);
+      if (q0.z & TAG_LEN) {
+        n += q0.w;                                              // a reader's wide list: its length, O(1)
+      } else {
+        uint32_t c = cur;
+        for (uint32_t k = 0; k < 16 && c != 0; ++k, ++n) c = cdr_of(C, c); // short lists inline;
+        if (c != 0) n += chain_length(C, c);                              // long ones 32 cells per round
+      }
       NTRACE_MAX(7);
-#if CULI_NEST_TRACE > 1
-      if (c != 0) { volatile uint32_t n2 = chain_length(C, c); (void)n2; }   // debug: the same walk, warm
-      NTRACE_MAX(4);
-#endif
     } else {
       for (uint32_t c = cur; c != 0; c = cdr_of(C, c)) ++n;
     }
