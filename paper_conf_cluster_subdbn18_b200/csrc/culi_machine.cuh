@@ -95,7 +95,7 @@ __device__ __forceinline__ void ldnode(const Ctx& C, uint32_t n, uint32_t& t, ui
   }
 #endif
   const uint4 q = *reinterpret_cast<const uint4*>(C.A->H.tag.p + n);   // one 16-byte load per node
-  t = q.z & (0xffu & ~(uint32_t)TAG_LEN);
+  t = q.z & 0xffu;                          // (flag bits PROPER / VALID / LEN: every consumer masks)
   w = ((uint64_t)q.y << 32) | q.x;
 }
 __device__ __forceinline__ uint64_t nword(const Ctx& C, uint32_t n) {
