@@ -293,6 +293,7 @@ __device__ __forceinline__ V lookup(const Ctx& C, uint32_t sym, uint32_t env) {
     uint32_t parent = VS(C, h)->x;
     if (n >= 1 && e.z == sym) return vunpack(e);
     if (n <= 1 && parent == 0) return global_value(C, sym);
+
   }
   return lookup_slow(C, sym, env);
 }
