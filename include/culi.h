@@ -87,7 +87,8 @@ int culi_arena_bytes(const culi_opts* opts, uint64_t* bytes);
 #define CULI_F_NO_STAGING 4u   /* do not stage the global frame / hot code in shared memory (§8(a)4)     */
 #define CULI_F_NO_VOTING  8u   /* batches that neither split nor nest: plain kernel instead of the warp-voting
                                   one (lanes regroup by stack height + continuation at returns) */
-#define CULI_F_NO_NESTED 16u   /* run nested (non-top-level) ||| forms inside one thread (§8(f)1 off)     */
+#define CULI_F_NO_NESTED 16u   /* run nested (non-top-level) ||| forms and wide data lists / (list ...)
+                                  below the top level inside one thread (§8(f)1 off)      */
 #define CULI_F_NO_SPLIT  32u   /* no argument splitting: each form is evaluated by one thread only        */
 #define CULI_F_NO_GC     64u   /* do not compact the persistent heap segment after culi_define (§8(f)3)  */
 #define CULI_F_NO_GRAPH 128u   /* culi_eval_uploaded issues its launches directly (no CUDA-graph replay)  */
