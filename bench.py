@@ -527,7 +527,8 @@ def culi_arm(args):
         "cpu_baseline": cpu,
         "e2e": {"value": e2e_value, "unit": "forms/s", "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
                 "ms_per_step": e2e_ms_step,
-                "path": ("culi_eval_text: pinned host text -> device read -> eval -> host results" if not dist_on
+                "path": ("culi_eval_text: pinned host text -> read (device reader; the host reader for texts of "
+                         "<= 16 KiB) -> eval -> host results" if not dist_on
                          else "per rank: pinned host text -> device read -> eval -> culi_results_export -> NCCL "
                               "all_gather; rank 0: culi_results_import (device merge) -> host results")},
         "e2e_image": {"value": img_value, "unit": "forms/s", "h2d_bytes_per_step": img_h2d,

@@ -92,6 +92,10 @@ int culi_arena_bytes(const culi_opts* opts, uint64_t* bytes);
 #define CULI_F_NO_SPLIT  32u   /* no argument splitting: each form is evaluated by one thread only        */
 #define CULI_F_NO_GC     64u   /* do not compact the persistent heap segment after culi_define (§8(f)3)  */
 #define CULI_F_NO_GRAPH 128u   /* culi_eval_uploaded issues its launches directly (no CUDA-graph replay)  */
+#define CULI_F_DEVICE_READ 256u /* culi_eval_text / culi_upload_text: always read on the device.  Without it
+                                  (and without env CULI_DEVICE_READ=1) host text of at most 16 KiB is read
+                                  by the host reader (same image): below that size the device
+                                  reader's launches and 3 sync points cost more than the parse itself      */
 /* Without flags: batches of <= 4,096 forms with no lambda / defun in them or in any definition run in
  * input order (no dispatch) and without argument splitting; argument splitting runs wherever a closure can
  * exist (binned or not, CULI_F_NO_BINNING included) — DESIGN.md §5.5. */

@@ -123,6 +123,7 @@ int culi_init(const culi_opts* opts, culi_ctx** out) {
   if (const char* e = getenv("CULI_SPLIT_SLEEP")) c->split_sleep = std::max(32, atoi(e));
   if (const char* e = getenv("CULI_STEAL_GATE")) c->steal_gate = atoi(e) != 0;
   if (const char* e = getenv("CULI_SIZE_FIRST")) c->size_first = atoi(e) != 0;
+  if (const char* e = getenv("CULI_DEVICE_READ")) c->force_device_read = atoi(e) != 0;
   if (const char* e = getenv("CULI_THIN_LANES")) c->thin_lanes = std::min(32, std::max(0, atoi(e)));
   if (const char* e = getenv("CULI_WAIT_MS")) c->wait_ns = (unsigned long long)std::max(1, atoi(e)) * 1000000ull;
   bool ok = true;
@@ -650,7 +651,16 @@ static int prepare_batch(culi_ctx* c, const Image& img) {
 }
 
 // Device reader (§8(f)2) -> the same prepared batch.
+// Host text up to this size is read by the host reader in culi_eval_text / culi_upload_text:
+// a read of a few KB costs ~0.2 ms of device-reader launches and sync points, ~0.03-0.17 ms on the host.
+constexpr size_t HOST_READ_MAX = 16384;
 static int prepare_text(culi_ctx* c, const char* text, size_t len, bool on_device, size_t* err_offset) {
+  if (!on_device && len <= HOST_READ_MAX && !(c->opts.flags & CULI_F_DEVICE_READ) && !c->force_device_read) {
+    Image img;                                       // small host text: the host reader is faster here
+    int rc = read_image(*c->syms, text, len, img, err_offset);
+    if (rc) return rc;
+    return prepare_batch(c, img);
+  }
   ReadOut ro;
   int rc = device_read(c, text, len, on_device, &ro, err_offset);
   if (rc) return rc;

@@ -164,6 +164,7 @@ struct culi_ctx {
   uint32_t steal_gate = 1;           // steal only from fully idle warps (env CULI_STEAL_GATE)
   uint32_t split_sleep = 4096;       // idle-warp back-off cap in ns (env CULI_SPLIT_SLEEP)
   uint32_t size_first = 1;           // dispatch: closure-free batches biggest forms first (env CULI_SIZE_FIRST)
+  bool force_device_read = false;    // env CULI_DEVICE_READ=1: culi_*_text never uses the host reader
   uint32_t thin_lanes = 0;           // small plain-kernel batches: forms per warp (0 = auto; env CULI_THIN_LANES)
   DevBuf<uint32_t> wide;
   DevBuf<uint32_t> lenpairs;         // wide-list length marks of a host image (culi_lenmark_kernel)

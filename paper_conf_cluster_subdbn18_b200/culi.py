@@ -25,6 +25,7 @@ CULI_F_NO_NESTED = 16
 CULI_F_NO_SPLIT = 32
 CULI_F_NO_GC = 64
 CULI_F_NO_GRAPH = 128
+CULI_F_DEVICE_READ = 256
 
 SYMBOLS = [
     "culi_default_opts", "culi_init", "culi_shutdown", "culi_read", "culi_image_nforms",

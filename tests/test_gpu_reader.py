@@ -294,3 +294,30 @@ def test_int_literals(culi):
     ctx = culi.Context(**SMALL)
     res = ctx.eval_text("\n".join(cases))
     assert [res.int_value(i) for i in range(len(cases))] == [int(c) for c in cases]
+
+
+def test_small_host_text_uses_host_reader(culi, oracle_mod):
+    """Without CULI_F_DEVICE_READ, culi_eval_text reads host text of <= 16 KiB with the host reader (faster than
+    the device reader's launches at that size): the same results and steps as the device
+    reader and the oracle, wide lists (length marks) included; larger texts still go to the device."""
+    import os as _os
+    forms = "\n".join(["(fib 12)", "(fact 10)", "(sum 30)", "(||| 3 + '(1 2 3) '(4 5 6))", '"str"', "'(a b)",
+                        "(||| 100 fib (%s))" % " ".join(["7"] * 100), "(length (list %s))" % " ".join(["1"] * 90)])
+    old = _os.environ.get("CULI_DEVICE_READ")
+    _os.environ["CULI_DEVICE_READ"] = "0"
+    try:
+        ctx = culi.Context(**SMALL)
+    finally:
+        _os.environ["CULI_DEVICE_READ"] = old if old is not None else "1"
+    ctx.define(DEFS)
+    r_host = ctx.eval_text(forms)
+    ctx.last_stats()
+    assert ctx.last_nested == 2                      # both wide lists suspended (host length marks)
+    ctx_dev = culi.Context(**SMALL, flags=culi.CULI_F_DEVICE_READ)
+    ctx_dev.define(DEFS)
+    r_dev = ctx_dev.eval_text(forms)
+    assert (r_host.printed(), r_host.steps()) == (r_dev.printed(), r_dev.steps())
+    o = oracle_mod.Session()
+    o.define(DEFS)
+    exp = o.eval_batch(forms, nthreads=1).results
+    assert not compare(r_host.printed(), r_host.steps(), exp, forms.splitlines())
