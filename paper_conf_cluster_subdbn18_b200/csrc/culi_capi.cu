@@ -59,7 +59,7 @@ static bool normalize_opts(culi_opts& o, int sms) {
   if (o.heap_nodes > 0x7fffffffull) return false;
   if (o.vstack_entries == 0) o.vstack_entries = 4096;
   if (o.vstack_entries > 65535) return false;
-  if (o.slots == 0) o.slots = (uint32_t)sms * 128 * CULI_BLOCKS_PER_SM;
+  if (o.slots == 0) o.slots = (uint32_t)sms * 128 * std::max(CULI_BLOCKS_PER_SM, CULI_SPLIT_BLOCKS_PER_SM);
   return true;
 }
 
@@ -550,9 +550,13 @@ static int run_batch_device(culi_ctx* c) {
     A.lanes = lanes;
     blocks = std::min<uint32_t>(c->nslots / 128, std::max<uint32_t>((nf + 4 * lanes - 1) / (4 * lanes), 1));
   }
+  // kernels bounded at CULI_BLOCKS_PER_SM resident blocks (voting, plain, fan-out) get one wave at most; they
+  // take their work from counters, so a smaller grid only means fewer, fuller threads
+  const uint32_t one_wave = (uint32_t)c->sms * CULI_BLOCKS_PER_SM;
+  if (!A.nest && !A.split) blocks = std::min(blocks, one_wave);
   if (nf) { CK(launch_eval(c->stream, A, blocks)); ++c->last_kernels; }
   if (nf && A.fanout && c->batch_has_par) {            // ||| fan-out (a6) + finalize (a8)
-    CK(launch_fanout(c->stream, A, c->nslots / 128));
+    CK(launch_fanout(c->stream, A, std::min(c->nslots / 128, one_wave)));
     c->last_kernels += 2;
   }
   CK(record_event(c, 2));
@@ -677,7 +681,9 @@ static int rerun_fallback(culi_ctx* c, uint32_t nfb) {
   A.fanout = 0;
   A.nest = 0;
   A.split = 0;
-  CK(launch_eval(c->stream, A, std::max<uint32_t>(1, std::min<uint32_t>(c->nslots / 128, (nfb + 127) / 128))));
+  CK(launch_eval(c->stream, A, std::max<uint32_t>(1, std::min<uint32_t>(std::min<uint32_t>(c->nslots / 128,
+                                                                                 (uint32_t)c->sms * CULI_BLOCKS_PER_SM),
+                                                                        (nfb + 127) / 128))));
   ExportArgs X{};
   X.tag = c->H.tag;
   X.word = c->H.word;

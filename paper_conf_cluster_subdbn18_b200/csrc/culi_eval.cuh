@@ -23,6 +23,13 @@ constexpr uint32_t STACK_ENV = 0x80000000u;   // env reference into the thread's
 // Resident 128-thread eval blocks per SM (the register budget of __launch_bounds__) and so the default
 // number of stack slots (SM count x 128 x this).  The machine is latency-bound: more warps per scheduler
 // hide more of each warp's dependent-instruction latency.
+// The splitting / nesting kernels (C2, C5, C0) run 9 (56 registers), the others 8 (64 registers):
+// measured per kernel (tools/ab.sh, session 2): split 8 -> 9 blocks C2 62.0 -> 60.5 ms, C5 126.5 -> 123.8 ms;
+// voting (C4) 0.47 -> 0.50 ms and fan-out (C3) 0.165 -> 0.170 ms at 9, so those stay at 8; 10 is worse
+// everywhere.  Stack slots are sized for the larger count.
+#ifndef CULI_SPLIT_BLOCKS_PER_SM
+#define CULI_SPLIT_BLOCKS_PER_SM 9
+#endif
 #ifndef CULI_BLOCKS_PER_SM
 #define CULI_BLOCKS_PER_SM 8
 #endif

@@ -217,7 +217,8 @@ __device__ __noinline__ uint32_t split_claim(const EvalArgs& A, uint32_t& round)
 // a lane that finds no form left is a thief: it evaluates split-off arguments of busy lanes on its own
 // stacks (one eval_form call site serves forms and tasks).
 template <bool FANOUT, bool NEST, bool SPLIT>
-__global__ void __launch_bounds__(128, CULI_BLOCKS_PER_SM) culi_eval_kernel(const __grid_constant__ EvalArgs A) {
+__global__ void __launch_bounds__(128, (NEST || SPLIT) ? CULI_SPLIT_BLOCKS_PER_SM : CULI_BLOCKS_PER_SM)
+culi_eval_kernel(const __grid_constant__ EvalArgs A) {
   uint4* scode = culi_smem;
   uint64_t* sgword = reinterpret_cast<uint64_t*>(culi_smem + A.code_n);
   uint8_t* sgtag = reinterpret_cast<uint8_t*>(sgword + A.gst);
